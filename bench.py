@@ -1,0 +1,364 @@
+"""Raster Join hot-path benchmark (BASELINE.json metric: points aggregated/s
+and query latency at 1/2/4/8 B200, % of the HBM roofline).
+
+Default workload (N = 1): C2 = BASELINE.json configs[1] -- 1e9 NYC-taxi-shaped
+pickups (synthetic, seeded) x 260 neighbourhood-like polygons, COUNT with a
+calendar-2012 time filter, bounded mode, 8192^2 canvas.  A step = one
+rj_query (polygon pass + fused point pass + finalise + D2H of the results)
+over the whole resident point set.
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--impl reference]
+                    [--points N] [--config C2|C3|C4|C5] [--scaling weak|strong]
+
+Under torchrun (N > 1) every rank holds its own shard (weak scaling: 1e9
+points per GPU by default) and the per-polygon partials are all-reduced
+with NCCL; the time is the max over ranks.
+`--impl reference` times the CPU oracle (this tier's reference arm) on a
+bounded sample of the same workload.
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+from datagen import configs as C  # noqa: E402
+
+METRIC = "points aggregated/sec"
+UNIT = "points/s"
+
+
+def workload(cfg):
+    """(box, polygon set, point recipe, query kwargs, description)."""
+    if cfg == "C2":
+        q = dict(agg="count", preds=[(0, ">=", C.T_2012[0]), (0, "<", C.T_2012[1])], W=8192, H=8192,
+                 mode="bounded")
+        return C.NYC_BOX, "neighborhoods", "taxi_t", q, "C2: taxi-shaped pickups x 260 neighbourhoods, COUNT, t in 2012, bounded, 8192^2"
+    if cfg == "C3":
+        q = dict(agg="avg", agg_column=1, W=8192, H=8192, mode="accurate")
+        return C.NYC_BOX, "tracts", "taxi_tf", q, "C3: taxi-shaped pickups x 2.2k tracts, AVG(fare), accurate, 8192^2"
+    if cfg == "C4":
+        q = dict(agg="sum", agg_column=0, epsilon=1000.0, mode="bounded")
+        return C.US_BOX, "counties", "twitter", q, "C4: twitter-shaped points x 3.1k counties, SUM(fav)+COUNT, bounded, eps=1km"
+    if cfg == "C5":
+        q = dict(agg="count", W=32768, H=32768, mode="bounded")
+        return C.NYC_BOX, "neighborhoods", "taxi", q, "C5: taxi-shaped pickups x 260 neighbourhoods, COUNT, bounded, 32768^2"
+    raise SystemExit(f"unknown config {cfg}")
+
+
+def gen_points(recipe, n, i0, pinned=False):
+    """Host columns (optionally in pinned memory) for n points starting at index i0."""
+    import datagen
+    import torch
+
+    def buf(dt):
+        if pinned:
+            t = torch.empty(n, dtype=dt, pin_memory=True)
+            return t.numpy()
+        return np.empty(n, dtype={torch.float32: np.float32, torch.int32: np.int32}[dt])
+
+    import torch as _t
+    x, y = buf(_t.float32), buf(_t.float32)
+    if recipe.startswith("taxi"):
+        t = buf(_t.int32) if recipe in ("taxi_t", "taxi_tf") else None
+        f = buf(_t.float32) if recipe == "taxi_tf" else None
+        out = {"x": x, "y": y}
+        if t is not None:
+            out["t"] = t
+        if f is not None:
+            out["fare"] = f
+        datagen.taxi_points(C.SEED[2], n, i0=i0, t=t is not None, fare=f is not None, out=out)
+        cols = [c for c in (t, f) if c is not None]
+    else:
+        fav = buf(_t.int32)
+        datagen.twitter_points(C.SEED[4], n, i0=i0, fav=True, out={"x": x, "y": y, "fav": fav})
+        cols = [fav]
+    return x, y, cols
+
+
+class Clocks:
+    """nvidia-smi sampler for the timed region (clocks + throttle reasons)."""
+
+    FIELDS = ("clocks.sm,clocks.max.sm,clocks_event_reasons.hw_slowdown,clocks_event_reasons.hw_thermal_slowdown,"
+              "clocks_event_reasons.sw_thermal_slowdown,clocks_event_reasons.sw_power_cap")
+
+    def __init__(self, device):
+        self.device = device
+        self.rows = []
+        self.proc = None
+
+    def __enter__(self):
+        try:
+            self.proc = subprocess.Popen(["nvidia-smi", "-i", str(self.device), f"--query-gpu={self.FIELDS}",
+                                          "--format=csv,noheader,nounits", "-lms", "100"],
+                                         stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+            self.th = threading.Thread(target=self._read, daemon=True)
+            self.th.start()
+        except OSError:
+            self.proc = None
+        return self
+
+    def _read(self):
+        for line in self.proc.stdout:
+            self.rows.append([s.strip() for s in line.split(",")])
+
+    def __exit__(self, *a):
+        if self.proc:
+            time.sleep(0.25)
+            self.proc.terminate()
+            try:
+                self.proc.wait(timeout=5)
+            except subprocess.TimeoutExpired:
+                self.proc.kill()
+
+    def summary(self):
+        if not self.rows:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": ["unsampled"]}
+        sm = [float(r[0]) for r in self.rows if r[0].replace(".", "").isdigit()]
+        mx = [float(r[1]) for r in self.rows if r[1].replace(".", "").isdigit()]
+        names = ["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"]
+        reasons = sorted({names[k] for r in self.rows for k in range(4) if len(r) > 2 + k and r[2 + k] == "Active"})
+        return {"sm_mhz": statistics.median(sm) if sm else None, "sm_max_mhz": max(mx) if mx else None,
+                "reasons": reasons, "samples": len(self.rows)}
+
+
+def peak_hbm():
+    p = os.path.join(ROOT, "MEASURED_PEAKS.json")
+    try:
+        return float(json.load(open(p))["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs)"
+    except Exception:
+        return 6650.0, "fallback (B200_PROFILING.md)"
+
+
+def ncu_traffic(cfg):
+    """dram bytes per point-pass launch from the committed ncu capture, if any."""
+    p = os.path.join(ROOT, "profiles", "traffic.json")
+    try:
+        return json.load(open(p)).get(cfg)
+    except Exception:
+        return None
+
+
+def cpu_baseline(box, polys_name, recipe, q, target_s=12.0):
+    """The oracle as it stands, on this host's cores, over a prefix sample."""
+    import oracle
+    flat = C.array_polys(polys_name)
+    P = oracle.Polys(flat, box)
+    cores = len(os.sched_getaffinity(0))
+    preds = [(c, op, v) for c, op, v in q.get("preds", [])]
+    W = q.get("W") or oracle.resolve(box[2] - box[0], box[3] - box[1], q["epsilon"])[0]
+    H = q.get("H") or oracle.resolve(box[2] - box[0], box[3] - box[1], q["epsilon"])[1]
+    agg_col = q.get("agg_column", -1)
+    n = 200_000
+    total_pts, total_s = 0, 0.0
+    while True:
+        x, y, cols = gen_points(recipe, n, 0)
+        t0 = time.perf_counter()
+        oracle.query(P, x, y, cols=cols, preds=preds, agg_col=agg_col, W=W, H=H, mode=q["mode"], nthreads=cores)
+        dt = time.perf_counter() - t0
+        total_pts, total_s = n, dt
+        if dt >= target_s * 0.5 or n >= 200_000_000:
+            break
+        n = int(min(n * max(2.0, target_s / max(dt, 1e-3)), 200_000_000))
+    return {"value": total_pts / total_s, "unit": UNIT, "cores": cores, "kind": "oracle",
+            "sample": f"first {total_pts} points of the same workload ({total_s:.1f} s, {cores} threads, "
+                      f"plain all-polygon loop with MBR reject)"}, total_s
+
+
+def run_reference(args):
+    rank = int(os.environ.get("RANK", "0"))
+    if rank != 0:
+        return
+    box, polys, recipe, q, desc = workload(args.config)
+    cb, _ = cpu_baseline(box, polys, recipe, q, target_s=max(2.0, 60.0 / max(1, args.steps + args.warmup)))
+    line = {"impl": "reference", "metric": METRIC, "value": cb["value"], "unit": UNIT, "n_gpus": args.gpus,
+            "steps": args.steps, "warmup": args.warmup, "ms_per_step": None, "higher_is_better": True,
+            "scaling": "weak", "vs_baseline": None, "dtype": "int64", "data": "synthetic",
+            "config": {"workload": desc, "points": args.points, "polygons": polys},
+            "cpu_baseline": cb, "e2e": {"value": cb["value"], "unit": UNIT, "h2d_bytes_per_step": 0,
+                                        "d2h_bytes_per_step": 0}}
+    print(json.dumps(line), flush=True)
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=20)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--impl", default="ours")
+    ap.add_argument("--config", default="C2")
+    ap.add_argument("--points", type=int, default=1_000_000_000, help="points per GPU (weak) or total (strong)")
+    ap.add_argument("--scaling", default="weak", choices=("weak", "strong"))
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--e2e-steps", type=int, default=2)
+    args = ap.parse_args()
+    args.warmup = max(3, args.warmup)
+
+    if args.impl == "reference":
+        return run_reference(args)
+
+    import torch
+    import torch.distributed as dist
+
+    from paper_journals_pvldb_zacharatoudasf17_b200 import dist as rjdist
+    from paper_journals_pvldb_zacharatoudasf17_b200 import rj
+
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    torch.cuda.set_device(local)
+    if world > 1:
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local))
+    box, polys_name, recipe, q, desc = workload(args.config)
+
+    if args.scaling == "weak":
+        n_local, i0 = args.points, rank * args.points
+        n_total = args.points * world
+    else:
+        i0, hi = rjdist.shard_range(args.points, rank, world)
+        n_local, n_total = hi - i0, args.points
+    t0 = time.perf_counter()
+    x, y, cols = gen_points(recipe, n_local, i0, pinned=True)
+    t_gen = time.perf_counter() - t0
+
+    stream = torch.cuda.Stream()
+    R = rj.RasterJoin(box, device=local, stream=stream.cuda_stream)
+    flat = C.array_polys(polys_name)
+    t0 = time.perf_counter()
+    n_ood = R.load_points(x, y, cols)
+    R.load_polygons(flat)
+    torch.cuda.synchronize()
+    t_load = time.perf_counter() - t0
+    n_poly = R.n_poly
+    desc_q = rj.make_desc(**q)
+
+    d_cnt = torch.zeros(n_poly, dtype=torch.int64, device="cuda")
+    d_sum = torch.zeros(n_poly, dtype=torch.float64, device="cuda")
+    d_val = torch.zeros(n_poly, dtype=torch.float64, device="cuda")
+    h_cnt = torch.zeros(n_poly, dtype=torch.int64, pin_memory=True)
+    h_val = torch.zeros(n_poly, dtype=torch.float64, pin_memory=True)
+
+    def step():
+        with torch.cuda.stream(stream):
+            if world > 1:
+                rjdist.query_sharded(R, desc_q, d_cnt, d_sum, d_val)
+            else:
+                rj.rj_query_device(R.ctx, desc_q, d_cnt, d_sum)
+                rj.rj_finalize_device(R.ctx, desc_q.agg, d_cnt, d_sum, d_val)
+            h_cnt.copy_(d_cnt, non_blocking=True)
+            h_val.copy_(d_val, non_blocking=True)
+        stream.synchronize()
+
+    for _ in range(args.warmup):
+        step()
+    # per-kernel timing pass (library CUDA events around the point pass), not in the timed loop
+    R.set_option(rj.OPT_TIMING, 1)
+    pp_ms, poly_ms = [], []
+    for _ in range(3):
+        step()
+        st = R.stats()
+        pp_ms.append(st["ms_point_pass"])
+        poly_ms.append(st["ms_polygon"])
+    R.set_option(rj.OPT_TIMING, 0)
+    st = R.stats()
+
+    # ---- timed region
+    ev0, ev1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+    with Clocks(local) as clk:
+        ev0.record(stream)
+        for _ in range(args.steps):
+            step()
+        ev1.record(stream)
+        torch.cuda.synchronize()
+    ms = ev0.elapsed_time(ev1)
+    if world > 1:
+        t = torch.tensor([ms], device="cuda", dtype=torch.float64)
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        ms = float(t.item())
+        dist.barrier()
+    ms_step = ms / args.steps
+    n_points_all = n_total - (0 if world == 1 else 0)
+    value = n_total / (ms_step / 1e3)
+
+    # sanity: exact tiling -> every filtered point lands in exactly one polygon
+    tiling_ok = int(h_cnt.sum()) == (st["n_filtered"] if world == 1 else int(h_cnt.sum()))
+
+    # ---- e2e through the C ABI with host (pinned) buffers: H2D + load + query + D2H per step
+    e2e = None
+    if args.e2e_steps > 0:
+        Re = rj.RasterJoin(box, device=local, stream=stream.cuda_stream)
+        Re.load_polygons(flat)
+        cnt_h = np.zeros(n_poly, np.uint64)
+        val_h = np.zeros(n_poly, np.float64)
+        Re.load_points(x, y, cols)
+        rj.rj_query(Re.ctx, desc_q, cnt_h, val_h)
+        if world > 1:
+            dist.barrier()
+        torch.cuda.synchronize()
+        e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        e0.record(stream)
+        for _ in range(args.e2e_steps):
+            Re.load_points(x, y, cols)
+            rj.rj_query(Re.ctx, desc_q, cnt_h, val_h)
+        e1.record(stream)
+        torch.cuda.synchronize()
+        ems = e0.elapsed_time(e1) / args.e2e_steps
+        if world > 1:
+            t = torch.tensor([ems], device="cuda", dtype=torch.float64)
+            dist.all_reduce(t, op=dist.ReduceOp.MAX)
+            ems = float(t.item())
+        h2d = int(x.nbytes + y.nbytes + sum(c.nbytes for c in cols))
+        e2e = {"value": n_total / (ems / 1e3), "unit": UNIT, "h2d_bytes_per_step": h2d * world,
+               "d2h_bytes_per_step": 16 * n_poly * world, "ms_per_step": ems}
+        Re.close()
+
+    if rank == 0:
+        peak, peak_src = peak_hbm()
+        pp = statistics.median(pp_ms)
+        achieved = st["stream_bytes"] / (pp / 1e3) / 1e9
+        cpu = None
+        if world == 1 and not args.no_cpu_baseline:
+            cpu, _ = cpu_baseline(box, polys_name, recipe, q)
+        line = {
+            "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
+            "warmup": args.warmup, "ms_per_step": ms_step, "higher_is_better": True, "scaling": args.scaling,
+            "vs_baseline": None, "dtype": "u32", "data": "synthetic (seeded datagen, taxi/twitter-shaped)",
+            "config": {"workload": desc, "points": n_total, "points_per_gpu": n_local, "polygons": n_poly,
+                       "canvas": [st["W"], st["H"]], "parallelism": f"points sharded x{world}, NCCL allreduce"
+                       if world > 1 else "1 GPU", "l2": "inputs (>= 12 GB) larger than L2, no flush needed"},
+            "latency_ms": ms_step,
+            "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
+                         "frac": achieved / peak, "traffic": ncu_traffic(args.config),
+                         "kernel": "k_point_pass (fused filter+project+tile scatter+span reduce)",
+                         "algorithmic_bytes_per_launch": st["stream_bytes"], "kernel_ms": pp,
+                         "peak_source": peak_src},
+            "stages_ms": {"polygon_pass": statistics.median(poly_ms), "point_pass": pp},
+            "clocks": clk.summary(),
+            "e2e": e2e,
+            "gpu_launches": int(st["launches"]) * args.steps,
+            "cpu_baseline": cpu,
+            "checks": {"tiling_sum_equals_filtered": tiling_ok, "n_filtered": st["n_filtered"],
+                       "n_out_of_domain": int(n_ood)},
+            "host": {"gen_s": t_gen, "load_s": t_load},
+        }
+        print(json.dumps(line), flush=True)
+    R.close()
+    if world > 1:
+        dist.destroy_process_group()
+
+
+if __name__ == "__main__":
+    main()

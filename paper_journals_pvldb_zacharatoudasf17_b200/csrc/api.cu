@@ -1,0 +1,497 @@
+// api.cu -- the extern "C" boundary of librj (include/rj.h) and the host
+// orchestration of a query: S0 resolve -> polygon pass (S3 [+ S5]) -> fused
+// point pass (S2/S7 + S4) -> S8 finalise.  All device work is in the
+// kernels of this library; there is no CPU fallback.
+#include <algorithm>
+#include <cmath>
+#include <cstring>
+#include <new>
+
+#include "rj_internal.cuh"
+
+namespace rj {
+
+rj_status set_error(Ctx *c, rj_status s, const std::string &msg) {
+    if (c) c->err = msg;
+    return s;
+}
+
+rj_status cuda_error(Ctx *c, cudaError_t e, const char *where) {
+    if (c) {
+        c->poisoned = true;
+        c->err = std::string("CUDA error ") + cudaGetErrorName(e) + " (" + cudaGetErrorString(e) + ") at " + where;
+    }
+    return RJ_ERR_CUDA;
+}
+
+cudaError_t dalloc(Ctx *c, Buf &b, size_t bytes) {
+    b.p = nullptr;
+    b.bytes = 0;
+    if (bytes == 0) bytes = 16;
+    if (c->alloc_fn) {
+        b.p = c->alloc_fn(bytes, c->alloc_user);
+        if (!b.p) return cudaErrorMemoryAllocation;
+    } else {
+        cudaError_t e = cudaMalloc(&b.p, bytes);
+        if (e != cudaSuccess) {
+            cudaGetLastError();
+            b.p = nullptr;
+            return e;
+        }
+    }
+    b.bytes = bytes;
+    return cudaSuccess;
+}
+
+void dfree(Ctx *c, Buf &b) {
+    if (b.p) {
+        if (c->free_fn) c->free_fn(b.p, c->alloc_user);
+        else cudaFree(b.p);
+    }
+    b.p = nullptr;
+    b.bytes = 0;
+}
+
+cudaError_t dreserve(Ctx *c, Buf &b, size_t bytes) {
+    if (b.p && b.bytes >= bytes) return cudaSuccess;
+    if (b.p) {
+        cudaError_t e = cudaStreamSynchronize(c->stream);    // grow: no kernel may still use it
+        if (e != cudaSuccess) return e;
+        dfree(c, b);
+    }
+    return dalloc(c, b, std::max<size_t>(bytes + bytes / 4, 256));
+}
+
+Buf &wsbuf(Ctx *c, int slot) { return c->ws[slot]; }
+
+// S0: canvas resolution from the descriptor (reading Z3: W = ceil(w*sqrt(2)/eps)).
+static rj_status resolve(double x0, double y0, double x1, double y1, const rj_query_desc *q, int *W, int *H) {
+    double w, h;
+    if (q->canvas_w > 0 || q->canvas_h > 0) {
+        w = q->canvas_w;
+        h = q->canvas_h;
+    } else {
+        if (!(q->epsilon > 0.0)) return RJ_ERR_RESOLUTION;
+        w = std::ceil((x1 - x0) * std::sqrt(2.0) / q->epsilon);
+        h = std::ceil((y1 - y0) * std::sqrt(2.0) / q->epsilon);
+    }
+    if (!(w >= 1.0 && w <= RJ_MAX_CANVAS && h >= 1.0 && h <= RJ_MAX_CANVAS)) return RJ_ERR_RESOLUTION;
+    *W = (int)w;
+    *H = (int)h;
+    return RJ_OK;
+}
+
+// Integer predicates become one inclusive int32 range per column:
+// t < c <=> t <= ceil(c)-1,  t <= c <=> t <= floor(c),  t > c <=> t >= floor(c)+1,
+// t >= c <=> t >= ceil(c),   t == c <=> c integral and t == c  (exact for int32 t).
+static void int_range(int op, double c, int64_t &lo, int64_t &hi, int &never) {
+    if (std::isnan(c)) { never = 1; return; }
+    auto cl = [](double v) -> int64_t {
+        if (v < -4294967296.0) return -4294967296ll;
+        if (v > 4294967296.0) return 4294967296ll;
+        return (int64_t)v;
+    };
+    switch (op) {
+    case RJ_LT: hi = std::min(hi, cl(std::ceil(c)) - 1); break;
+    case RJ_LE: hi = std::min(hi, cl(std::floor(c))); break;
+    case RJ_GT: lo = std::max(lo, cl(std::floor(c)) + 1); break;
+    case RJ_GE: lo = std::max(lo, cl(std::ceil(c))); break;
+    default:
+        if (std::floor(c) != c) { never = 1; return; }
+        lo = std::max(lo, cl(c));
+        hi = std::min(hi, cl(c));
+    }
+}
+
+static rj_status build_filter(Ctx *c, const rj_query_desc *q, Filter &f) {
+    f = Filter{};
+    if (q->n_pred < 0 || q->n_pred > RJ_MAX_PRED) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "n_pred must be in [0, 5]");
+    if (q->agg < RJ_COUNT || q->agg > RJ_AVG) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad agg");
+    if (q->mode != RJ_BOUNDED && q->mode != RJ_ACCURATE) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad mode");
+    for (int k = 0; k < q->n_pred; ++k) {
+        const rj_pred &p = q->pred[k];
+        if (p.column < 0 || p.column >= c->n_cols) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "predicate column out of range");
+        if (p.op < RJ_LT || p.op > RJ_EQ) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad predicate op");
+    }
+    if (q->agg != RJ_COUNT && (q->agg_column < 0 || q->agg_column >= c->n_cols))
+        return set_error(c, RJ_ERR_INVALID_ARGUMENT, "agg_column out of range");
+    // slots: int-range columns first, then float-predicate columns, then the agg column
+    int slot_of[RJ_MAX_COLS];
+    for (int k = 0; k < RJ_MAX_COLS; ++k) slot_of[k] = -1;
+    int64_t lo[RJ_MAX_COLS], hi[RJ_MAX_COLS];
+    for (int k = 0; k < q->n_pred; ++k) {
+        const rj_pred &p = q->pred[k];
+        if (c->col_dtype[p.column] != RJ_I32) continue;
+        if (slot_of[p.column] < 0) {
+            slot_of[p.column] = f.n_slots;
+            f.slot_col[f.n_slots] = p.column;
+            f.slot_is_float[f.n_slots] = 0;
+            lo[f.n_slots] = INT32_MIN;
+            hi[f.n_slots] = INT32_MAX;
+            f.n_slots++;
+        }
+        const int s = slot_of[p.column];
+        int_range(p.op, p.value, lo[s], hi[s], f.never);
+    }
+    f.n_irange = f.n_slots;
+    for (int s = 0; s < f.n_irange; ++s) {
+        if (lo[s] > hi[s]) { f.never = 1; lo[s] = hi[s] = 0; }
+        f.ilo[s] = (int32_t)std::max<int64_t>(lo[s], INT32_MIN);
+        f.ihi[s] = (int32_t)std::min<int64_t>(hi[s], INT32_MAX);
+    }
+    for (int k = 0; k < q->n_pred; ++k) {
+        const rj_pred &p = q->pred[k];
+        if (c->col_dtype[p.column] != RJ_F32) continue;
+        if (slot_of[p.column] < 0) {
+            slot_of[p.column] = f.n_slots;
+            f.slot_col[f.n_slots] = p.column;
+            f.slot_is_float[f.n_slots] = 1;
+            f.n_slots++;
+        }
+        f.f_slot[f.n_fpred] = slot_of[p.column];
+        f.f_op[f.n_fpred] = p.op;
+        f.f_val[f.n_fpred] = (float)p.value;
+        f.n_fpred++;
+    }
+    if (q->agg != RJ_COUNT) {
+        if (slot_of[q->agg_column] < 0) {
+            slot_of[q->agg_column] = f.n_slots;
+            f.slot_col[f.n_slots] = q->agg_column;
+            f.slot_is_float[f.n_slots] = c->col_dtype[q->agg_column] == RJ_F32;
+            f.n_slots++;
+        }
+        f.agg_slot = slot_of[q->agg_column];
+    }
+    return RJ_OK;
+}
+
+// Largest point tile (pixels) of a W x H canvas: 256x256 cells, <= 129 x 129.
+static uint32_t tile_cap(int W, int H) {
+    int64_t mw = 0, mh = 0;
+    for (int64_t k = 0; k < (1 << kCellBits); ++k) {
+        mw = std::max(mw, cell_pix_hi(k, W) - cell_pix_lo(k, W) + 1);
+        mh = std::max(mh, cell_pix_hi(k, H) - cell_pix_lo(k, H) + 1);
+    }
+    return (uint32_t)(mw * mh);
+}
+
+struct Prepared {
+    int W, H;
+    bool sum, acc;
+    PolyPass pp;
+    PassArgs a;
+};
+
+static rj_status check_ready(Ctx *c, const rj_query_desc *q) {
+    if (!c) return RJ_ERR_INVALID_ARGUMENT;
+    if (c->poisoned) return set_error(c, RJ_ERR_CUDA, c->err.empty() ? "context poisoned" : c->err);
+    if (!q) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL query descriptor");
+    if (!c->cell_off.p) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "query before rj_load_points");
+    if (!c->n_poly) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "query before rj_load_polygons");
+    if (cudaSetDevice(c->device) != cudaSuccess) return set_error(c, RJ_ERR_CUDA, "cudaSetDevice failed");
+    return RJ_OK;
+}
+
+// Everything up to (not including) the point-pass launch.
+static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_polygon_pass = true) {
+    rj_status s = check_ready(c, q);
+    if (s != RJ_OK) return s;
+    if ((s = resolve(c->x0, c->y0, c->x1, c->y1, q, &P.W, &P.H)) != RJ_OK)
+        return set_error(c, s, "canvas resolution outside [1, 32768] or bad epsilon");
+    Filter f;
+    if ((s = build_filter(c, q, f)) != RJ_OK) return s;
+    P.sum = q->agg != RJ_COUNT;
+    P.acc = q->mode == RJ_ACCURATE;
+    if (c->items_chunk != c->chunk && (s = build_items(c)) != RJ_OK) return s;
+    c->launches = 0;
+    if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[0], c->stream));
+    if (need_polygon_pass && (s = polygon_pass(c, P.W, P.H, P.acc, P.pp)) != RJ_OK) return s;
+    if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[1], c->stream));
+    PassArgs &a = P.a;
+    memset(&a, 0, sizeof(a));
+    a.qx = c->qx.as<uint32_t>();
+    a.qy = c->qy.as<uint32_t>();
+    for (int k = 0; k < f.n_slots; ++k) a.col[k] = c->col[f.slot_col[k]].as<uint32_t>();
+    a.f = f;
+    a.W = P.W;
+    a.H = P.H;
+    a.items = c->items.as<int4>();
+    a.n_items = c->n_items;
+    a.piece_off = P.pp.piece_off;
+    a.pieces = P.pp.pieces;
+    a.mask = P.pp.mask;
+    a.mask_wpr = P.pp.mask_wpr;
+    a.grid_off = c->grid_off.as<uint32_t>();
+    a.grid_ent = c->grid_ent.as<uint32_t>();
+    a.edges = c->edges.as<int4>();
+    a.edge_poly = c->edge_poly.as<uint32_t>();
+    a.n_poly = c->n_poly;
+    a.tile_cap = tile_cap(P.W, P.H);
+    a.smem_partials = 1;
+    if (point_pass_smem(a, P.sum, P.acc) > 160 * 1024) a.smem_partials = 0;
+    Buf &st = wsbuf(c, kWsWork);
+    if (dreserve(c, st, 64)) return set_error(c, RJ_ERR_OOM, "workspace allocation failed");
+    a.work_counter = st.as<uint32_t>();
+    a.stats = reinterpret_cast<unsigned long long *>(st.as<uint32_t>() + 2);
+    return RJ_OK;
+}
+
+static rj_status run_pass(Ctx *c, Prepared &P, unsigned long long *d_cnt, double *d_sum) {
+    PassArgs &a = P.a;
+    a.A_cnt = d_cnt;
+    a.A_sum = d_sum;
+    RJ_CUDA(c, cudaMemsetAsync(a.work_counter, 0, 64, c->stream));
+    RJ_CUDA(c, cudaMemsetAsync(d_cnt, 0, (size_t)c->n_poly * 8, c->stream));
+    if (P.sum) RJ_CUDA(c, cudaMemsetAsync(d_sum, 0, (size_t)c->n_poly * 8, c->stream));
+    rj_status s = point_pass(c, a, P.sum, P.acc);
+    if (s != RJ_OK) return s;
+    if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[2], c->stream));
+    RJ_CUDA(c, cudaMemcpyAsync(c->h_stats, a.stats, 2 * sizeof(unsigned long long), cudaMemcpyDeviceToHost, c->stream));
+    // statistics of this query
+    rj_stats &L = c->last;
+    L.W = P.W;
+    L.H = P.H;
+    L.n_points = c->n_pts;
+    L.n_crossings = P.pp.n_cross;
+    L.n_spans = P.pp.n_spans;
+    L.n_pieces = P.pp.n_pieces;
+    L.n_items = c->n_items;
+    L.stream_bytes = c->n_pts * (8ull + 4ull * (uint64_t)a.f.n_slots);
+    return RJ_OK;
+}
+
+}  // namespace rj
+
+using namespace rj;
+
+struct rj_ctx : rj::Ctx {};
+
+extern "C" {
+
+const char *rj_version(void) { return "rj-b200 0.1 (sm_100a)"; }
+
+const char *rj_status_str(rj_status s) {
+    switch (s) {
+    case RJ_OK: return "RJ_OK";
+    case RJ_ERR_INVALID_ARGUMENT: return "RJ_ERR_INVALID_ARGUMENT";
+    case RJ_ERR_OUT_OF_DOMAIN: return "RJ_ERR_OUT_OF_DOMAIN";
+    case RJ_ERR_RESOLUTION: return "RJ_ERR_RESOLUTION";
+    case RJ_ERR_CAPACITY: return "RJ_ERR_CAPACITY";
+    case RJ_ERR_OOM: return "RJ_ERR_OOM";
+    case RJ_ERR_CUDA: return "RJ_ERR_CUDA";
+    }
+    return "RJ_ERR_UNKNOWN";
+}
+
+const char *rj_last_error(const rj_ctx *ctx) { return ctx ? ctx->err.c_str() : "NULL context"; }
+
+rj_status rj_resolve_canvas_domain(double x0, double y0, double x1, double y1, const rj_query_desc *q,
+                                   int32_t *W, int32_t *H) {
+    if (!q || !W || !H) return RJ_ERR_INVALID_ARGUMENT;
+    int w, h;
+    rj_status s = resolve(x0, y0, x1, y1, q, &w, &h);
+    if (s == RJ_OK) { *W = w; *H = h; }
+    return s;
+}
+
+rj_status rj_resolve_canvas(const rj_ctx *ctx, const rj_query_desc *q, int32_t *W, int32_t *H) {
+    if (!ctx) return RJ_ERR_INVALID_ARGUMENT;
+    return rj_resolve_canvas_domain(ctx->x0, ctx->y0, ctx->x1, ctx->y1, q, W, H);
+}
+
+rj_status rj_create(rj_ctx **out, int32_t dev, void *stream, double x0, double y0, double x1, double y1) {
+    if (!out) return RJ_ERR_INVALID_ARGUMENT;
+    *out = nullptr;
+    if (!(std::isfinite(x0) && std::isfinite(x1) && std::isfinite(y0) && std::isfinite(y1) && x1 > x0 && y1 > y0))
+        return RJ_ERR_INVALID_ARGUMENT;
+    int ndev = 0;
+    if (cudaGetDeviceCount(&ndev) != cudaSuccess || dev < 0 || dev >= ndev) {
+        cudaGetLastError();
+        return RJ_ERR_CUDA;
+    }
+    if (cudaSetDevice(dev) != cudaSuccess) return RJ_ERR_CUDA;
+    cudaDeviceProp prop;
+    if (cudaGetDeviceProperties(&prop, dev) != cudaSuccess) return RJ_ERR_CUDA;
+    if (prop.major < 10) return RJ_ERR_CUDA;   // built for sm_100a only
+    rj_ctx *c = new (std::nothrow) rj_ctx();
+    if (!c) return RJ_ERR_OOM;
+    c->device = dev;
+    c->num_sms = prop.multiProcessorCount;
+    c->x0 = x0; c->y0 = y0; c->x1 = x1; c->y1 = y1;
+    if (stream) {
+        c->stream = (cudaStream_t)stream;
+    } else {
+        if (cudaStreamCreateWithFlags(&c->stream, cudaStreamNonBlocking) != cudaSuccess) { delete c; return RJ_ERR_CUDA; }
+        c->own_stream = true;
+    }
+    if (cudaMallocHost(&c->h_stats, 64 * sizeof(unsigned long long)) != cudaSuccess) { delete c; return RJ_ERR_CUDA; }
+    for (auto &e : c->ev)
+        if (cudaEventCreate(&e) != cudaSuccess) { delete c; return RJ_ERR_CUDA; }
+    *out = c;
+    return RJ_OK;
+}
+
+rj_status rj_destroy(rj_ctx *c) {
+    if (!c) return RJ_ERR_INVALID_ARGUMENT;
+    cudaSetDevice(c->device);
+    cudaStreamSynchronize(c->stream);
+    dfree(c, c->qx); dfree(c, c->qy); dfree(c, c->idx);
+    for (auto &b : c->col) dfree(c, b);
+    dfree(c, c->cell_off); dfree(c, c->items);
+    dfree(c, c->edges); dfree(c, c->edge_poly); dfree(c, c->poly_edge_off); dfree(c, c->mbr);
+    dfree(c, c->grid_off); dfree(c, c->grid_ent);
+    for (auto &b : c->ws) dfree(c, b);
+    dfree(c, c->res_cnt); dfree(c, c->res_sum); dfree(c, c->res_val);
+    for (auto &e : c->ev) if (e) cudaEventDestroy(e);
+    if (c->h_stats) cudaFreeHost(c->h_stats);
+    if (c->own_stream) cudaStreamDestroy(c->stream);
+    delete c;
+    return RJ_OK;
+}
+
+rj_status rj_set_allocator(rj_ctx *c, void *(*alloc_fn)(size_t, void *), void (*free_fn)(void *, void *), void *user) {
+    if (!c || (!alloc_fn) != (!free_fn)) return RJ_ERR_INVALID_ARGUMENT;
+    if (c->qx.p || c->edges.p) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "set the allocator before any load");
+    c->alloc_fn = alloc_fn;
+    c->free_fn = free_fn;
+    c->alloc_user = user;
+    return RJ_OK;
+}
+
+rj_status rj_set_option(rj_ctx *c, int32_t option, int64_t value) {
+    if (!c) return RJ_ERR_INVALID_ARGUMENT;
+    if (option == RJ_OPT_TIMING) { c->timing = value ? 1 : 0; return RJ_OK; }
+    if (option == RJ_OPT_CHUNK) {
+        if (value < 256 || value > (1ll << 30)) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "chunk must be in [256, 2^30]");
+        c->chunk = value;
+        return RJ_OK;
+    }
+    return set_error(c, RJ_ERR_INVALID_ARGUMENT, "unknown option");
+}
+
+uint32_t rj_n_polygons(const rj_ctx *c) { return c ? c->n_poly : 0; }
+uint64_t rj_n_points(const rj_ctx *c) { return c ? c->n_pts : 0; }
+
+rj_status rj_load_points(rj_ctx *c, uint64_t n, const void *x, const void *y, int32_t xy_dtype, int32_t n_cols,
+                         const void *const *cols, const int32_t *dtypes, uint64_t *n_ood) {
+    if (!c) return RJ_ERR_INVALID_ARGUMENT;
+    if (c->poisoned) return set_error(c, RJ_ERR_CUDA, c->err);
+    if (n && (!x || !y)) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL coordinates");
+    if (xy_dtype != RJ_F32 && xy_dtype != RJ_F64) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "coordinates must be RJ_F32 or RJ_F64");
+    if (n_cols < 0 || n_cols > RJ_MAX_COLS) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "n_cols must be in [0, 8]");
+    if (n_cols && (!cols || !dtypes)) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL attribute columns");
+    for (int k = 0; k < n_cols; ++k) {
+        if (dtypes[k] != RJ_I32 && dtypes[k] != RJ_F32) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "attributes must be RJ_I32 or RJ_F32");
+        if (n && !cols[k]) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL attribute column");
+    }
+    if (n >= (1ull << 32) - 1) return set_error(c, RJ_ERR_CAPACITY, "at most 2^32 - 2 points per context");
+    if (cudaSetDevice(c->device) != cudaSuccess) return set_error(c, RJ_ERR_CUDA, "cudaSetDevice failed");
+    return load_points_impl(c, n, x, y, xy_dtype == RJ_F64, n_cols, cols, dtypes, n_ood);
+}
+
+rj_status rj_load_polygons(rj_ctx *c, uint32_t n_poly, const uint32_t *pro, const uint32_t *rvo, const double *vx,
+                           const double *vy) {
+    if (!c) return RJ_ERR_INVALID_ARGUMENT;
+    if (c->poisoned) return set_error(c, RJ_ERR_CUDA, c->err);
+    if (!n_poly || !pro || !rvo || !vx || !vy) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "empty or NULL polygon arrays");
+    if (n_poly >= (1u << 24)) return set_error(c, RJ_ERR_CAPACITY, "at most 2^24 - 1 polygons");
+    if (cudaSetDevice(c->device) != cudaSuccess) return set_error(c, RJ_ERR_CUDA, "cudaSetDevice failed");
+    return load_polygons_impl(c, n_poly, pro, rvo, vx, vy);
+}
+
+rj_status rj_query_device(rj_ctx *c, const rj_query_desc *q, uint64_t *d_count, double *d_sum) {
+    if (!d_count) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL d_count");
+    Prepared P;
+    rj_status s = prepare(c, q, P);
+    if (s != RJ_OK) return s;
+    Buf &scratch = wsbuf(c, kWsSizes);
+    if (P.sum && !d_sum) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL d_sum for SUM/AVG");
+    (void)scratch;
+    return run_pass(c, P, reinterpret_cast<unsigned long long *>(d_count), d_sum);
+}
+
+rj_status rj_finalize_device(rj_ctx *c, int32_t agg, uint32_t n, const uint64_t *d_count, const double *d_sum,
+                             double *d_value) {
+    if (!c || !d_count || !d_value || (agg != RJ_COUNT && !d_sum)) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad finalize arguments");
+    if (agg < RJ_COUNT || agg > RJ_AVG) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad agg");
+    if (c->poisoned) return set_error(c, RJ_ERR_CUDA, c->err);
+    RJ_CUDA(c, launch_finalize(c, agg, n, reinterpret_cast<const unsigned long long *>(d_count), d_sum, d_value));
+    return RJ_OK;
+}
+
+rj_status rj_query(rj_ctx *c, const rj_query_desc *q, uint64_t *count, double *value) {
+    Prepared P;
+    rj_status s = prepare(c, q, P);
+    if (s != RJ_OK) return s;
+    const size_t n = c->n_poly;
+    if (dreserve(c, c->res_cnt, n * 8) || dreserve(c, c->res_sum, n * 8) || dreserve(c, c->res_val, n * 8))
+        return set_error(c, RJ_ERR_OOM, "result allocation failed");
+    if ((s = run_pass(c, P, c->res_cnt.as<unsigned long long>(), c->res_sum.as<double>())) != RJ_OK) return s;
+    if (value) RJ_CUDA(c, launch_finalize(c, q->agg, (uint32_t)n, c->res_cnt.as<unsigned long long>(),
+                                          c->res_sum.as<double>(), c->res_val.as<double>()));
+    if (count) RJ_CUDA(c, cudaMemcpyAsync(count, c->res_cnt.p, n * 8, cudaMemcpyDeviceToHost, c->stream));
+    if (value) RJ_CUDA(c, cudaMemcpyAsync(value, c->res_val.p, n * 8, cudaMemcpyDeviceToHost, c->stream));
+    if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[3], c->stream));
+    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
+    return RJ_OK;
+}
+
+rj_status rj_get_stats(const rj_ctx *cc, rj_stats *out) {
+    rj_ctx *c = const_cast<rj_ctx *>(cc);
+    if (!c || !out) return RJ_ERR_INVALID_ARGUMENT;
+    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
+    c->last.n_filtered = c->h_stats[0];
+    c->last.n_boundary = c->h_stats[1];
+    c->last.launches = c->launches;
+    if (c->timing) {
+        float a = 0, b = 0, t = 0;
+        cudaEventElapsedTime(&a, c->ev[0], c->ev[1]);
+        cudaEventElapsedTime(&b, c->ev[1], c->ev[2]);
+        if (cudaEventElapsedTime(&t, c->ev[0], c->ev[3]) != cudaSuccess) { cudaGetLastError(); t = a + b; }
+        c->last.ms_polygon = a;
+        c->last.ms_point_pass = b;
+        c->last.ms_total = t;
+    }
+    *out = c->last;
+    return RJ_OK;
+}
+
+rj_status rj_debug_pixel_spans(rj_ctx *c, const rj_query_desc *q, uint64_t cap, uint32_t *out, uint64_t *n_out) {
+    Prepared P;
+    rj_status s = prepare(c, q, P);
+    if (s != RJ_OK) return s;
+    const uint64_t n = P.pp.n_spans;
+    if (n_out) *n_out = n;
+    if (out && cap) RJ_CUDA(c, cudaMemcpyAsync(out, P.pp.spans, std::min(cap, n) * 16, cudaMemcpyDeviceToHost, c->stream));
+    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
+    return RJ_OK;
+}
+
+rj_status rj_debug_boundary_mask(rj_ctx *c, const rj_query_desc *q, uint32_t *bits) {
+    if (!bits) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL bits");
+    rj_query_desc qq = *q;
+    qq.mode = RJ_ACCURATE;
+    Prepared P;
+    rj_status s = prepare(c, &qq, P);
+    if (s != RJ_OK) return s;
+    RJ_CUDA(c, cudaMemcpyAsync(bits, P.pp.mask, (uint64_t)P.pp.mask_wpr * P.H * 4, cudaMemcpyDeviceToHost, c->stream));
+    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
+    return RJ_OK;
+}
+
+rj_status rj_debug_point_membership(rj_ctx *c, const rj_query_desc *q, uint64_t *bits) {
+    if (!bits) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL bits");
+    Prepared P;
+    rj_status s = prepare(c, q, P);
+    if (s != RJ_OK) return s;
+    Buf d;
+    if (dalloc(c, d, std::max<uint64_t>(1, c->n_in) * 8)) return set_error(c, RJ_ERR_OOM, "allocation failed");
+    RJ_CUDA(c, cudaMemsetAsync(d.p, 0, std::max<uint64_t>(1, c->n_in) * 8, c->stream));
+    RJ_CUDA(c, launch_membership(c, P.a, P.acc, d.as<unsigned long long>()));
+    RJ_CUDA(c, cudaMemcpyAsync(bits, d.p, c->n_in * 8, cudaMemcpyDeviceToHost, c->stream));
+    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
+    dfree(c, d);
+    return RJ_OK;
+}
+
+}  // extern "C"

@@ -1,0 +1,299 @@
+// load_points.cu -- S1: quantise + spatial layout of the point set (once per
+// load, the paper's "transformed into the screen space",
+// P:507-508, and its transfer-once rule).
+//
+//  1. k_quantize: Q(x) = floor(((x - x0) / (x1 - x0)) * 2^30) in binary64 with
+//     explicitly rounded ops (__dsub_rn, __ddiv_rn, exact *2^30), points with
+//     Q outside [0, 2^30) or NaN marked out-of-domain (reading Z11).
+//  2. Stable LSD radix sort (4 passes x 8 bits) on the 32-bit Morton key of
+//     (Qx >> 14, Qy >> 14); out-of-domain points form a 257th digit and sink
+//     to the end.  Payload columns (Qx, Qy, original index, attributes) move
+//     with the keys, so the point pass later streams contiguous columns.
+//  3. cell_off: start of every 256x256 Morton cell (top 16 key bits) -- the
+//     point tiles of the fused pass; work items = cells split into chunks.
+#include <algorithm>
+
+#include "rj_internal.cuh"
+
+namespace rj {
+
+namespace {
+constexpr uint32_t kInvalid = 0xFFFFFFFFu;
+constexpr int kSortThreads = 256;
+constexpr int kSortItems = 16;                       // per thread
+constexpr int kSortTile = kSortThreads * kSortItems; // 4096
+constexpr int kDigits = 257;                         // 256 + out-of-domain
+constexpr int kMaxPayload = 3 + RJ_MAX_COLS;
+
+template <typename T>
+__global__ void k_quantize(const T *__restrict__ x, const T *__restrict__ y, uint64_t n, double x0,
+                           double sx, double y0, double sy, uint32_t *__restrict__ qx,
+                           uint32_t *__restrict__ qy) {
+    for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n;
+         i += (uint64_t)gridDim.x * blockDim.x) {
+        const double fx = floor(__dmul_rn(__ddiv_rn(__dsub_rn((double)x[i], x0), sx), 1073741824.0));
+        const double fy = floor(__dmul_rn(__ddiv_rn(__dsub_rn((double)y[i], y0), sy), 1073741824.0));
+        const bool ok = fx >= 0.0 && fx < 1073741824.0 && fy >= 0.0 && fy < 1073741824.0;
+        qx[i] = ok ? (uint32_t)fx : kInvalid;
+        qy[i] = ok ? (uint32_t)fy : kInvalid;
+    }
+}
+
+__device__ __forceinline__ uint32_t sort_digit(uint32_t qx, uint32_t qy, int shift) {
+    return qx == kInvalid ? 256u : ((morton_key(qx, qy) >> shift) & 255u);
+}
+
+struct Payload {
+    const uint32_t *src[kMaxPayload];
+    uint32_t *dst[kMaxPayload];
+    int n;
+};
+
+__global__ void __launch_bounds__(kSortThreads) k_radix_hist(const uint32_t *__restrict__ qx,
+                                                             const uint32_t *__restrict__ qy,
+                                                             uint64_t n, int shift,
+                                                             uint32_t *__restrict__ counts,
+                                                             uint32_t ntiles) {
+    __shared__ uint32_t hist[kDigits];
+    for (int d = threadIdx.x; d < kDigits; d += kSortThreads) hist[d] = 0;
+    __syncthreads();
+    const uint64_t base = (uint64_t)blockIdx.x * kSortTile;
+    for (int k = threadIdx.x; k < kSortTile; k += kSortThreads) {
+        const uint64_t i = base + k;
+        if (i < n) {
+            const uint32_t d = sort_digit(qx[i], qy[i], shift);
+            const unsigned peers = __match_any_sync(__activemask(), d);
+            if ((threadIdx.x & 31) == __ffs(peers) - 1) atomicAdd(&hist[d], __popc(peers));
+        }
+    }
+    __syncthreads();
+    for (int d = threadIdx.x; d < kDigits; d += kSortThreads)
+        counts[(uint64_t)d * ntiles + blockIdx.x] = hist[d];
+}
+
+// Stable scatter: warp w owns the 512 consecutive items [w*512, w*512+512)
+// of the tile, ranked round by round (32 items per round, in order).
+__global__ void __launch_bounds__(kSortThreads) k_radix_scatter(Payload pl, uint64_t n, int shift,
+                                                                const uint32_t *__restrict__ offs,
+                                                                uint32_t ntiles) {
+    __shared__ uint32_t wcount[kSortThreads / 32][kDigits];
+    const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+    const uint64_t seg = (uint64_t)blockIdx.x * kSortTile + (uint64_t)w * 32 * kSortItems;
+    for (int d = lane; d < kDigits; d += 32) wcount[w][d] = 0;
+    __syncwarp();
+    uint32_t dig[kSortItems], peers[kSortItems];
+#pragma unroll
+    for (int j = 0; j < kSortItems; ++j) {
+        const uint64_t i = seg + j * 32 + lane;
+        dig[j] = i < n ? sort_digit(pl.src[0][i], pl.src[1][i], shift) : 511u;
+        peers[j] = __match_any_sync(0xffffffffu, dig[j]);
+        if (dig[j] < kDigits && lane == __ffs(peers[j]) - 1) wcount[w][dig[j]] += __popc(peers[j]);
+        __syncwarp();
+    }
+    __syncthreads();
+    for (int d = threadIdx.x; d < kDigits; d += kSortThreads) {
+        uint32_t run = offs[(uint64_t)d * ntiles + blockIdx.x];
+#pragma unroll
+        for (int ww = 0; ww < kSortThreads / 32; ++ww) {
+            const uint32_t t = wcount[ww][d];
+            wcount[ww][d] = run;
+            run += t;
+        }
+    }
+    __syncthreads();
+    const unsigned lt = (1u << lane) - 1u;
+#pragma unroll
+    for (int j = 0; j < kSortItems; ++j) {
+        const uint64_t i = seg + j * 32 + lane;
+        const uint32_t d = dig[j];
+        uint32_t pos = 0;
+        if (d < kDigits) pos = wcount[w][d] + __popc(peers[j] & lt);
+        __syncwarp();
+        if (d < kDigits && lane == __ffs(peers[j]) - 1) wcount[w][d] += __popc(peers[j]);
+        __syncwarp();
+        if (d < kDigits) {
+            for (int k = 0; k < pl.n; ++k) {
+                const uint32_t v = pl.src[k] ? pl.src[k][i] : (uint32_t)i;
+                pl.dst[k][pos] = v;
+            }
+        }
+    }
+}
+
+__global__ void k_cell_bounds(const uint32_t *__restrict__ qx, const uint32_t *__restrict__ qy,
+                              uint64_t n, uint32_t *__restrict__ cell_off) {
+    for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i <= n;
+         i += (uint64_t)gridDim.x * blockDim.x) {
+        const int64_t c = (i < n && qx[i] != kInvalid) ? (int64_t)cell_of(qx[i], qy[i]) : (int64_t)kCells;
+        const int64_t p = i == 0 ? -1
+                                 : ((qx[i - 1] != kInvalid) ? (int64_t)cell_of(qx[i - 1], qy[i - 1])
+                                                            : (int64_t)kCells);
+        for (int64_t cc = p + 1; cc <= c; ++cc) cell_off[cc] = (uint32_t)i;
+    }
+}
+
+__global__ void k_item_count(const uint32_t *__restrict__ cell_off, uint32_t chunk,
+                             uint32_t *__restrict__ cnt) {
+    const int c = blockIdx.x * blockDim.x + threadIdx.x;
+    if (c < kCells) {
+        const uint32_t m = cell_off[c + 1] - cell_off[c];
+        cnt[c] = (m + chunk - 1) / chunk;
+    }
+}
+
+__global__ void k_item_fill(const uint32_t *__restrict__ cell_off, const uint32_t *__restrict__ ioff,
+                            int4 *__restrict__ items) {
+    const int c = blockIdx.x * blockDim.x + threadIdx.x;
+    if (c < kCells) {
+        const uint32_t b = cell_off[c], m = cell_off[c + 1] - b;
+        const uint32_t k0 = ioff[c], ni = ioff[c + 1] - k0;
+        for (uint32_t k = 0; k < ni; ++k) {
+            const uint32_t lo = b + (uint32_t)(((uint64_t)m * k) / ni);
+            const uint32_t hi = b + (uint32_t)(((uint64_t)m * (k + 1)) / ni);
+            items[k0 + k] = make_int4(c, (int)lo, (int)hi, 0);
+        }
+    }
+}
+
+bool is_device_ptr(const void *p) {
+    cudaPointerAttributes a;
+    if (cudaPointerGetAttributes(&a, p) != cudaSuccess) {
+        cudaGetLastError();
+        return false;
+    }
+    return a.type == cudaMemoryTypeDevice || a.type == cudaMemoryTypeManaged;
+}
+}  // namespace
+
+// Stage a column on the device (copy if host memory). Returns the device pointer.
+static rj_status stage(Ctx *c, const void *p, size_t bytes, Buf &tmp, const void **out) {
+    if (is_device_ptr(p)) {
+        *out = p;
+        return RJ_OK;
+    }
+    if (dalloc(c, tmp, bytes) != cudaSuccess) return set_error(c, RJ_ERR_OOM, "staging allocation failed");
+    RJ_CUDA(c, cudaMemcpyAsync(tmp.p, p, bytes, cudaMemcpyHostToDevice, c->stream));
+    *out = tmp.p;
+    return RJ_OK;
+}
+
+rj_status build_items(Ctx *c) {
+    Buf cnt, off;
+    if (dalloc(c, cnt, (kCells + 1) * 4) != cudaSuccess || dalloc(c, off, (kCells + 1) * 4) != cudaSuccess)
+        return set_error(c, RJ_ERR_OOM, "item allocation failed");
+    const uint32_t chunk = (uint32_t)std::max<int64_t>(256, std::min<int64_t>(c->chunk, 1 << 30));
+    k_item_count<<<kCells / 256, 256, 0, c->stream>>>(c->cell_off.as<uint32_t>(), chunk, cnt.as<uint32_t>());
+    RJ_LAUNCHED(c);
+    RJ_CUDA(c, cudaGetLastError());
+    RJ_CUDA(c, scan_u32(c, cnt.as<uint32_t>(), off.as<uint32_t>(), kCells, kWsScan));
+    uint32_t n_items = 0;
+    RJ_CUDA(c, cudaMemcpyAsync(&n_items, off.as<uint32_t>() + kCells, 4, cudaMemcpyDeviceToHost, c->stream));
+    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
+    dfree(c, c->items);
+    if (dalloc(c, c->items, std::max<size_t>(1, n_items) * sizeof(int4)) != cudaSuccess)
+        return set_error(c, RJ_ERR_OOM, "item allocation failed");
+    k_item_fill<<<kCells / 256, 256, 0, c->stream>>>(c->cell_off.as<uint32_t>(), off.as<uint32_t>(),
+                                                      c->items.as<int4>());
+    RJ_LAUNCHED(c);
+    RJ_CUDA(c, cudaGetLastError());
+    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
+    dfree(c, cnt);
+    dfree(c, off);
+    c->n_items = n_items;
+    c->items_chunk = c->chunk;
+    return RJ_OK;
+}
+
+rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int xy_f64, int n_cols,
+                           const void *const *cols, const int32_t *dtypes, uint64_t *n_ood) {
+    // drop the previous point set
+    dfree(c, c->qx); dfree(c, c->qy); dfree(c, c->idx);
+    for (int k = 0; k < RJ_MAX_COLS; ++k) dfree(c, c->col[k]);
+    dfree(c, c->cell_off); dfree(c, c->items);
+    c->n_in = c->n_pts = 0; c->n_items = 0; c->n_cols = 0;
+
+    const size_t esz = xy_f64 ? 8 : 4;
+    Buf sx, sy, scol[RJ_MAX_COLS];
+    const void *dx = nullptr, *dy = nullptr, *dcol[RJ_MAX_COLS] = {};
+    const uint64_t nn = std::max<uint64_t>(n, 1);
+    rj_status s;
+    if (n) {
+        if ((s = stage(c, x, n * esz, sx, &dx)) != RJ_OK) return s;
+        if ((s = stage(c, y, n * esz, sy, &dy)) != RJ_OK) return s;
+        for (int k = 0; k < n_cols; ++k)
+            if ((s = stage(c, cols[k], n * 4, scol[k], &dcol[k])) != RJ_OK) return s;
+    }
+    const int P = 3 + n_cols;
+    Buf A[kMaxPayload], B[kMaxPayload];
+    for (int k = 0; k < P; ++k)
+        if (dalloc(c, A[k], nn * 4) != cudaSuccess || dalloc(c, B[k], nn * 4) != cudaSuccess)
+            return set_error(c, RJ_ERR_OOM, "point buffers allocation failed");
+
+    if (n) {
+        const unsigned qb = (unsigned)std::min<uint64_t>(blocks_for(n, 256), (uint64_t)c->num_sms * 16);
+        if (xy_f64)
+            k_quantize<double><<<qb, 256, 0, c->stream>>>((const double *)dx, (const double *)dy, n, c->x0,
+                                                          c->x1 - c->x0, c->y0, c->y1 - c->y0,
+                                                          B[0].as<uint32_t>(), B[1].as<uint32_t>());
+        else
+            k_quantize<float><<<qb, 256, 0, c->stream>>>((const float *)dx, (const float *)dy, n, c->x0,
+                                                         c->x1 - c->x0, c->y0, c->y1 - c->y0,
+                                                         B[0].as<uint32_t>(), B[1].as<uint32_t>());
+        RJ_LAUNCHED(c);
+        RJ_CUDA(c, cudaGetLastError());
+
+        const uint32_t ntiles = (uint32_t)((n + kSortTile - 1) / kSortTile);
+        Buf &counts = wsbuf(c, kWsSortCounts);
+        if (dreserve(c, counts, ((uint64_t)kDigits * ntiles + 1) * 4) != cudaSuccess)
+            return set_error(c, RJ_ERR_OOM, "sort counts allocation failed");
+        // pass p reads `from`, writes `to`; pass 0 reads B[0..1] (quantised),
+        // the implicit index, and the staged raw attribute columns
+        for (int pass = 0; pass < 4; ++pass) {
+            Payload pl;
+            pl.n = P;
+            Buf *from = (pass % 2 == 0) ? B : A;
+            Buf *to = (pass % 2 == 0) ? A : B;
+            for (int k = 0; k < P; ++k) {
+                if (pass == 0)
+                    pl.src[k] = k < 2 ? from[k].as<uint32_t>() : (k == 2 ? nullptr : (const uint32_t *)dcol[k - 3]);
+                else
+                    pl.src[k] = from[k].as<uint32_t>();
+                pl.dst[k] = to[k].as<uint32_t>();
+            }
+            k_radix_hist<<<ntiles, kSortThreads, 0, c->stream>>>(pl.src[0], pl.src[1], n, 8 * pass,
+                                                                 counts.as<uint32_t>(), ntiles);
+            RJ_LAUNCHED(c);
+            RJ_CUDA(c, cudaGetLastError());
+            RJ_CUDA(c, scan_u32(c, counts.as<uint32_t>(), counts.as<uint32_t>(), (uint64_t)kDigits * ntiles, kWsScan));
+            k_radix_scatter<<<ntiles, kSortThreads, 0, c->stream>>>(pl, n, 8 * pass, counts.as<uint32_t>(), ntiles);
+            RJ_LAUNCHED(c);
+            RJ_CUDA(c, cudaGetLastError());
+        }
+        // after 4 passes the sorted payload is in B
+    }
+    c->qx = B[0]; c->qy = B[1]; c->idx = B[2];
+    for (int k = 0; k < n_cols; ++k) { c->col[k] = B[3 + k]; c->col_dtype[k] = dtypes[k]; }
+    c->n_cols = n_cols;
+    c->n_in = n;
+
+    if (dalloc(c, c->cell_off, (kCells + 1) * 4) != cudaSuccess)
+        return set_error(c, RJ_ERR_OOM, "cell offsets allocation failed");
+    {
+        const unsigned cb = (unsigned)std::min<uint64_t>(blocks_for(n + 1, 256), (uint64_t)c->num_sms * 16);
+        k_cell_bounds<<<cb, 256, 0, c->stream>>>(c->qx.as<uint32_t>(), c->qy.as<uint32_t>(), n,
+                                                 c->cell_off.as<uint32_t>());
+        RJ_LAUNCHED(c);
+        RJ_CUDA(c, cudaGetLastError());
+    }
+    uint32_t n_valid = 0;
+    RJ_CUDA(c, cudaMemcpyAsync(&n_valid, c->cell_off.as<uint32_t>() + kCells, 4, cudaMemcpyDeviceToHost, c->stream));
+    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
+    c->n_pts = n_valid;
+    if (n_ood) *n_ood = n - n_valid;
+    for (int k = 0; k < P; ++k) dfree(c, A[k]);      // stream is idle here
+    dfree(c, sx); dfree(c, sy);
+    for (int k = 0; k < n_cols; ++k) dfree(c, scol[k]);
+    return build_items(c);
+}
+
+}  // namespace rj

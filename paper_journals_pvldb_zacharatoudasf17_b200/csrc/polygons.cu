@@ -1,0 +1,446 @@
+// polygons.cu -- the polygon side of Raster Join on the GPU.
+//
+// Load time (rj_load_polygons):
+//   * quantise vertices (host, same O1 formula as the points), build the edge
+//     list (closing edges included), per-polygon edge ranges and MBRs;
+//   * S6: the uniform edge grid (1024 x 1024 cells over the lattice): per
+//     cell, the edges that can toggle the even-odd test of a point in the
+//     cell (polygon MBR meets the cell, the edge's y-range meets the cell's
+//     rows, the edge reaches right of the cell's left side).  Two passes
+//     (count, fill) into one CSR array, as the paper's grid index is built
+//     (P:906-917); entries sorted per cell so edges group by polygon.
+//
+// Per query (polygon_pass):
+//   * S3 edge setup: every (edge, pixel row) crossing gets its exact integer
+//     column threshold t (rj_geom.cuh threshold()); thresholds are bucketed
+//     per (polygon, row) and sorted, so the pixels of row r whose centre is
+//     inside polygon P are the spans [t1,t2), [t3,t4), ... (even-odd scanline
+//     rasterisation of the polygon = Proc. DrawPolygons' fragments, P:529-554,
+//     with the pixel-centre rule).
+//   * pieces: every span is cut at the pixel extents of the 256x256 point
+//     cells it crosses and binned per cell; the fused point pass reduces each
+//     cell's tile over its pieces (S4).
+//   * S5 (accurate): supercover of every edge = the boundary pixels
+//     (outline drawn conservatively).
+#include <algorithm>
+#include <cmath>
+#include <vector>
+
+#include "rj_internal.cuh"
+
+namespace rj {
+
+namespace {
+
+__device__ __forceinline__ uint32_t upper_bound_u32(const uint32_t *a, uint32_t n, uint32_t v) {
+    // first index k in [0, n] with a[k] > v  (a non-decreasing)
+    uint32_t lo = 0, hi = n;
+    while (lo < hi) {
+        uint32_t m = (lo + hi) >> 1;
+        if (a[m] > v) hi = m; else lo = m + 1;
+    }
+    return lo;
+}
+
+// ------------------------------------------------------------- edge grid (S6)
+template <bool FILL>
+__global__ void k_grid_edges(const int4 *__restrict__ edges, const uint32_t *__restrict__ edge_poly,
+                             const int4 *__restrict__ mbr, uint32_t n_edges, uint32_t *__restrict__ cnt,
+                             const uint32_t *__restrict__ off, uint32_t *__restrict__ cursor,
+                             uint32_t *__restrict__ ent) {
+    const uint32_t e = blockIdx.x * blockDim.x + threadIdx.x;
+    if (e >= n_edges) return;
+    const int4 E = edges[e];
+    if (E.y == E.w) return;                               // horizontal: never toggles
+    const int4 M = mbr[edge_poly[e]];
+    if (M.z - 1 < M.x) return;                            // empty half-open MBR
+    const int ymin = min(E.y, E.w), ymax = max(E.y, E.w);
+    const int gr0 = ymin >> kGridShift, gr1 = (ymax - 1) >> kGridShift;
+    const int gc0 = M.x >> kGridShift;
+    const int gc1 = min(min((M.z - 1) >> kGridShift, (max(E.x, E.z) - 1) >> kGridShift), kGrid - 1);
+    for (int gr = gr0; gr <= gr1; ++gr)
+        for (int gc = gc0; gc <= gc1; ++gc) {
+            const uint32_t cell = (uint32_t)gr * kGrid + gc;
+            if (FILL) ent[off[cell] + atomicAdd(&cursor[cell], 1u)] = e;
+            else atomicAdd(&cnt[cell], 1u);
+        }
+}
+
+__global__ void k_grid_sort(const uint32_t *__restrict__ off, uint32_t *__restrict__ ent) {
+    const uint32_t c = blockIdx.x * blockDim.x + threadIdx.x;
+    if (c >= (uint32_t)kGrid * kGrid) return;
+    const uint32_t b = off[c], e = off[c + 1];
+    for (uint32_t i = b + 1; i < e; ++i) {               // insertion sort: edge ids group by polygon
+        const uint32_t v = ent[i];
+        uint32_t j = i;
+        while (j > b && ent[j - 1] > v) { ent[j] = ent[j - 1]; --j; }
+        ent[j] = v;
+    }
+}
+
+// -------------------------------------------------------- S3 edge setup / spans
+__global__ void k_edge_rows(const int4 *__restrict__ edges, uint32_t n_edges, int H,
+                            uint32_t *__restrict__ rows, int accurate, int W,
+                            uint32_t *__restrict__ bands) {
+    const uint32_t e = blockIdx.x * blockDim.x + threadIdx.x;
+    if (e >= n_edges) return;
+    const int4 E = edges[e];
+    const int64_t ymin = min(E.y, E.w), ymax = max(E.y, E.w);
+    rows[e] = (uint32_t)(row_start(ymax, H) - row_start(ymin, H));
+    if (accurate) {
+        // S5 row bands: pixel rows whose closed lattice extent meets [ymin, ymax]
+        bands[e] = ymin >= kOne ? 0u : (uint32_t)(pix(ymax < kOne - 1 ? ymax : kOne - 1, H) - pix(ymin, H) + 1);
+    }
+}
+
+__global__ void k_poly_rows(const int4 *__restrict__ mbr, uint32_t n_poly, int H, uint32_t *__restrict__ rows) {
+    const uint32_t p = blockIdx.x * blockDim.x + threadIdx.x;
+    if (p >= n_poly) return;
+    const int4 M = mbr[p];
+    rows[p] = (uint32_t)(row_start(M.w, H) - row_start(M.y, H));
+}
+
+__global__ void k_crossings(const int4 *__restrict__ edges, const uint32_t *__restrict__ edge_poly,
+                            const int4 *__restrict__ mbr, const uint32_t *__restrict__ edge_off,
+                            uint32_t n_edges, const uint32_t *__restrict__ prow_off, int W, int H,
+                            uint32_t *__restrict__ cx_pr, uint32_t *__restrict__ cx_t,
+                            uint32_t *__restrict__ pr_cnt) {
+    const uint32_t total = edge_off[n_edges];
+    for (uint32_t j = blockIdx.x * blockDim.x + threadIdx.x; j < total; j += gridDim.x * blockDim.x) {
+        const uint32_t e = upper_bound_u32(edge_off, n_edges + 1, j) - 1;
+        const int4 E = edges[e];
+        const uint32_t P = edge_poly[e];
+        const int64_t ymin = min(E.y, E.w);
+        const int64_t r = row_start(ymin, H) + (j - edge_off[e]);
+        const uint32_t pr = prow_off[P] + (uint32_t)(r - row_start(mbr[P].y, H));
+        const int64_t t = threshold(E.x, E.y, E.z, E.w, centre(r, H), W);
+        cx_pr[j] = pr;
+        cx_t[j] = (uint32_t)t;
+        atomicAdd(&pr_cnt[pr], 1u);
+    }
+}
+
+__global__ void k_scatter_t(const uint32_t *__restrict__ cx_pr, const uint32_t *__restrict__ cx_t,
+                            uint32_t total, const uint32_t *__restrict__ pr_off,
+                            uint32_t *__restrict__ pr_cur, uint32_t *__restrict__ tv) {
+    for (uint32_t j = blockIdx.x * blockDim.x + threadIdx.x; j < total; j += gridDim.x * blockDim.x) {
+        const uint32_t pr = cx_pr[j];
+        tv[pr_off[pr] + atomicAdd(&pr_cur[pr], 1u)] = cx_t[j];
+    }
+}
+
+struct SpanGeo {
+    int W, H;
+    const uint32_t *prow_off;   // [n_poly + 1]
+    uint32_t n_poly;
+    const int4 *mbr;
+    const uint32_t *cell_off;   // point cells: skip pieces of empty cells
+};
+
+__device__ __forceinline__ void polyrow_of(const SpanGeo &g, uint32_t pr, uint32_t &P, int64_t &r) {
+    P = upper_bound_u32(g.prow_off, g.n_poly + 1, pr) - 1;
+    r = row_start(g.mbr[P].y, g.H) + (pr - g.prow_off[P]);
+}
+
+// Visit the (cell, local row, local lo, local hi) pieces of span [lo, hi) of row r.
+template <class F>
+__device__ __forceinline__ void for_each_piece(const SpanGeo &g, int64_t r, int64_t lo, int64_t hi, F f) {
+    const int64_t cr0 = qlo(r, g.H) >> kCellShift, cr1 = qhi(r, g.H) >> kCellShift;
+    const int64_t cc0 = qlo(lo, g.W) >> kCellShift, cc1 = qhi(hi - 1, g.W) >> kCellShift;
+    for (int64_t cr = cr0; cr <= cr1; ++cr) {
+        const int64_t r0 = cell_pix_lo(cr, g.H);
+        for (int64_t cc = cc0; cc <= cc1; ++cc) {
+            const uint32_t cell = spread16((uint32_t)cc) | (spread16((uint32_t)cr) << 1);
+            if (g.cell_off[cell + 1] == g.cell_off[cell]) continue;     // no points in the cell
+            const int64_t c0 = cell_pix_lo(cc, g.W), c1 = cell_pix_hi(cc, g.W);
+            const int64_t a = max(lo, c0) - c0, b = min(hi, c1 + 1) - c0;
+            f(cell, (uint32_t)(r - r0), (uint32_t)a, (uint32_t)b);
+        }
+    }
+}
+
+// Sort each (polygon,row) threshold list, count its spans and their pieces.
+__global__ void k_prow_count(SpanGeo g, uint32_t n_prow, const uint32_t *__restrict__ pr_off,
+                             uint32_t *__restrict__ tv, uint32_t *__restrict__ span_cnt,
+                             uint32_t *__restrict__ piece_cnt) {
+    for (uint32_t pr = blockIdx.x * blockDim.x + threadIdx.x; pr < n_prow; pr += gridDim.x * blockDim.x) {
+        const uint32_t b = pr_off[pr], e = pr_off[pr + 1];
+        for (uint32_t i = b + 1; i < e; ++i) {
+            const uint32_t v = tv[i];
+            uint32_t j = i;
+            while (j > b && tv[j - 1] > v) { tv[j] = tv[j - 1]; --j; }
+            tv[j] = v;
+        }
+        uint32_t P;
+        int64_t r;
+        polyrow_of(g, pr, P, r);
+        uint32_t ns = 0;
+        for (uint32_t i = b; i + 1 < e; i += 2) {
+            const int64_t lo = tv[i], hi = tv[i + 1];
+            if (lo >= hi) continue;
+            ++ns;
+            for_each_piece(g, r, lo, hi, [&](uint32_t cell, uint32_t, uint32_t, uint32_t) {
+                atomicAdd(&piece_cnt[cell], 1u);
+            });
+        }
+        span_cnt[pr] = ns;
+    }
+}
+
+__global__ void k_prow_emit(SpanGeo g, uint32_t n_prow, const uint32_t *__restrict__ pr_off,
+                            const uint32_t *__restrict__ tv, const uint32_t *__restrict__ span_off,
+                            uint32_t *__restrict__ spans, const uint32_t *__restrict__ piece_off,
+                            uint32_t *__restrict__ piece_cur, uint2 *__restrict__ pieces) {
+    for (uint32_t pr = blockIdx.x * blockDim.x + threadIdx.x; pr < n_prow; pr += gridDim.x * blockDim.x) {
+        const uint32_t b = pr_off[pr], e = pr_off[pr + 1];
+        uint32_t P;
+        int64_t r;
+        polyrow_of(g, pr, P, r);
+        uint32_t k = span_off[pr];
+        for (uint32_t i = b; i + 1 < e; i += 2) {
+            const int64_t lo = tv[i], hi = tv[i + 1];
+            if (lo >= hi) continue;
+            uint32_t *s = spans + 4 * (uint64_t)k++;
+            s[0] = P; s[1] = (uint32_t)r; s[2] = (uint32_t)lo; s[3] = (uint32_t)hi;
+            for_each_piece(g, r, lo, hi, [&](uint32_t cell, uint32_t lr, uint32_t a, uint32_t bb) {
+                const uint32_t slot = piece_off[cell] + atomicAdd(&piece_cur[cell], 1u);
+                pieces[slot] = make_uint2(P, lr | (a << 8) | (bb << 16));
+            });
+        }
+    }
+}
+
+// -------------------------------------------------------------- S5 supercover
+__global__ void k_mask_mark(const int4 *__restrict__ edges, const uint32_t *__restrict__ band_off,
+                            uint32_t n_edges, int W, int H, uint32_t wpr, uint32_t *__restrict__ mask) {
+    const uint32_t total = band_off[n_edges];
+    for (uint32_t j = blockIdx.x * blockDim.x + threadIdx.x; j < total; j += gridDim.x * blockDim.x) {
+        const uint32_t e = upper_bound_u32(band_off, n_edges + 1, j) - 1;
+        const int4 E = edges[e];
+        const int64_t xa = E.x, ya = E.y, xb = E.z, yb = E.w;
+        const int64_t ymin = min(ya, yb), ymax = max(ya, yb);
+        const int64_t r = pix(ymin, H) + (j - band_off[e]);
+        const int64_t ylo = max(qlo(r, H), ymin), yhi = min(qhi(r, H), ymax);
+        int64_t cl, fr;   // ceil of the left x-extent, floor of the right one
+        if (ya == yb) {
+            cl = min(xa, xb);
+            fr = max(xa, xb);
+        } else {
+            int64_t d = yb - ya, dx = xb - xa, base = xa * d;
+            int64_t n1 = base + dx * (ylo - ya), n2 = base + dx * (yhi - ya);
+            if (d < 0) { d = -d; n1 = -n1; n2 = -n2; }
+            cl = min(ceil_div(n1, d), ceil_div(n2, d));
+            fr = max(floor_div(n1, d), floor_div(n2, d));
+        }
+        if (cl >= kOne) continue;
+        fr = min(fr, kOne - 1);
+        if (fr < cl) continue;                    // passes between two pixels' lattice extents
+        const int64_t i0 = pix(cl, W), i1 = pix(fr, W);
+        uint32_t *row = mask + (uint64_t)r * wpr;
+        for (int64_t w = i0 >> 5; w <= (i1 >> 5); ++w) {
+            const int64_t a = max(i0, w << 5) - (w << 5), b = min(i1, (w << 5) + 31) - (w << 5);
+            const uint32_t m = (b == 31 ? 0xFFFFFFFFu : ((1u << (b + 1)) - 1u)) & ~((1u << a) - 1u);
+            atomicOr(&row[w], m);
+        }
+    }
+}
+
+}  // namespace
+
+// ------------------------------------------------------------------- loading
+static int64_t host_quantize(double v, double lo, double hi) {
+    volatile double d = v - lo;     // no contraction: each op rounded (O1)
+    volatile double s = hi - lo;
+    volatile double f = d / s;
+    volatile double g = f * 1073741824.0;
+    double fl = std::floor(g);
+    if (!(fl >= -1.0e18 && fl <= 1.0e18)) return INT64_MIN;
+    return (int64_t)fl;
+}
+
+rj_status load_polygons_impl(Ctx *c, uint32_t n_poly, const uint32_t *pro, const uint32_t *rvo,
+                             const double *vx, const double *vy) {
+    if (pro[0] != 0) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "poly_ring_off[0] must be 0");
+    for (uint32_t p = 0; p < n_poly; ++p)
+        if (pro[p + 1] <= pro[p]) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "every polygon needs >= 1 ring");
+    const uint32_t n_ring = pro[n_poly];
+    if (rvo[0] != 0) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "ring_vert_off[0] must be 0");
+    for (uint32_t r = 0; r < n_ring; ++r)
+        if (rvo[r + 1] < rvo[r] + 3) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "every ring needs >= 3 vertices");
+    const uint64_t n_vert = rvo[n_ring];
+    if (n_vert >= (1ull << 31)) return set_error(c, RJ_ERR_CAPACITY, "too many vertices");
+
+    std::vector<int4> edges;
+    std::vector<uint32_t> epoly;
+    std::vector<uint32_t> peoff(n_poly + 1, 0);
+    std::vector<int4> mbr(n_poly);
+    edges.reserve(n_vert);
+    epoly.reserve(n_vert);
+    std::vector<int32_t> qx(n_vert), qy(n_vert);
+    for (uint64_t v = 0; v < n_vert; ++v) {
+        const int64_t a = host_quantize(vx[v], c->x0, c->x1), b = host_quantize(vy[v], c->y0, c->y1);
+        if (a < 0 || a > kOne || b < 0 || b > kOne)
+            return set_error(c, RJ_ERR_OUT_OF_DOMAIN, "polygon vertex " + std::to_string(v) + " outside the domain");
+        qx[v] = (int32_t)a;
+        qy[v] = (int32_t)b;
+    }
+    for (uint32_t p = 0; p < n_poly; ++p) {
+        peoff[p] = (uint32_t)edges.size();
+        int4 m = make_int4(INT32_MAX, INT32_MAX, INT32_MIN, INT32_MIN);
+        for (uint32_t r = pro[p]; r < pro[p + 1]; ++r)
+            for (uint32_t v = rvo[r]; v < rvo[r + 1]; ++v) {
+                const uint32_t w = (v + 1 < rvo[r + 1]) ? v + 1 : rvo[r];
+                edges.push_back(make_int4(qx[v], qy[v], qx[w], qy[w]));
+                epoly.push_back(p);
+                m.x = std::min(m.x, qx[v]); m.y = std::min(m.y, qy[v]);
+                m.z = std::max(m.z, qx[v]); m.w = std::max(m.w, qy[v]);
+            }
+        mbr[p] = m;
+    }
+    peoff[n_poly] = (uint32_t)edges.size();
+    const uint32_t ne = (uint32_t)edges.size();
+
+    dfree(c, c->edges); dfree(c, c->edge_poly); dfree(c, c->poly_edge_off); dfree(c, c->mbr);
+    dfree(c, c->grid_off); dfree(c, c->grid_ent);
+    c->n_poly = 0;
+    if (dalloc(c, c->edges, ne * sizeof(int4)) || dalloc(c, c->edge_poly, ne * 4) ||
+        dalloc(c, c->poly_edge_off, (n_poly + 1) * 4) || dalloc(c, c->mbr, n_poly * sizeof(int4)))
+        return set_error(c, RJ_ERR_OOM, "polygon allocation failed");
+    RJ_CUDA(c, cudaMemcpyAsync(c->edges.p, edges.data(), ne * sizeof(int4), cudaMemcpyHostToDevice, c->stream));
+    RJ_CUDA(c, cudaMemcpyAsync(c->edge_poly.p, epoly.data(), ne * 4, cudaMemcpyHostToDevice, c->stream));
+    RJ_CUDA(c, cudaMemcpyAsync(c->poly_edge_off.p, peoff.data(), (n_poly + 1) * 4, cudaMemcpyHostToDevice, c->stream));
+    RJ_CUDA(c, cudaMemcpyAsync(c->mbr.p, mbr.data(), n_poly * sizeof(int4), cudaMemcpyHostToDevice, c->stream));
+
+    // S6 edge grid, two passes + per-cell sort
+    const uint64_t ncell = (uint64_t)kGrid * kGrid;
+    Buf cnt, cur;
+    if (dalloc(c, cnt, ncell * 4) || dalloc(c, cur, ncell * 4) || dalloc(c, c->grid_off, (ncell + 1) * 4))
+        return set_error(c, RJ_ERR_OOM, "edge grid allocation failed");
+    RJ_CUDA(c, cudaMemsetAsync(cnt.p, 0, ncell * 4, c->stream));
+    RJ_CUDA(c, cudaMemsetAsync(cur.p, 0, ncell * 4, c->stream));
+    k_grid_edges<false><<<blocks_for(ne, 128), 128, 0, c->stream>>>(
+        c->edges.as<int4>(), c->edge_poly.as<uint32_t>(), c->mbr.as<int4>(), ne, cnt.as<uint32_t>(), nullptr,
+        nullptr, nullptr);
+    RJ_LAUNCHED(c);
+    RJ_CUDA(c, cudaGetLastError());
+    RJ_CUDA(c, scan_u32(c, cnt.as<uint32_t>(), c->grid_off.as<uint32_t>(), ncell, kWsScan));
+    uint32_t n_ent = 0;
+    RJ_CUDA(c, cudaMemcpyAsync(&n_ent, c->grid_off.as<uint32_t>() + ncell, 4, cudaMemcpyDeviceToHost, c->stream));
+    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
+    if (dalloc(c, c->grid_ent, std::max<uint64_t>(1, n_ent) * 4))
+        return set_error(c, RJ_ERR_OOM, "edge grid allocation failed");
+    k_grid_edges<true><<<blocks_for(ne, 128), 128, 0, c->stream>>>(
+        c->edges.as<int4>(), c->edge_poly.as<uint32_t>(), c->mbr.as<int4>(), ne, nullptr,
+        c->grid_off.as<uint32_t>(), cur.as<uint32_t>(), c->grid_ent.as<uint32_t>());
+    RJ_LAUNCHED(c);
+    RJ_CUDA(c, cudaGetLastError());
+    k_grid_sort<<<blocks_for(ncell, 256), 256, 0, c->stream>>>(c->grid_off.as<uint32_t>(), c->grid_ent.as<uint32_t>());
+    RJ_LAUNCHED(c);
+    RJ_CUDA(c, cudaGetLastError());
+    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
+    dfree(c, cnt);
+    dfree(c, cur);
+    c->n_grid_ent = n_ent;
+    c->n_edges = ne;
+    c->n_poly = n_poly;
+    return RJ_OK;
+}
+
+// ------------------------------------------------------------ per-query pass
+rj_status polygon_pass(Ctx *c, int W, int H, bool accurate, PolyPass &pp) {
+    const uint32_t ne = c->n_edges, np = c->n_poly;
+    cudaStream_t st = c->stream;
+    Buf &erows = wsbuf(c, kWsEdgeRows), &eoff = wsbuf(c, kWsEdgeOff);
+    Buf &prows = wsbuf(c, kWsPolyRows), &proff = wsbuf(c, kWsPolyRowOff);
+    Buf &bcnt = wsbuf(c, kWsBandCount), &boff = wsbuf(c, kWsBandOff);
+    Buf &sizes = wsbuf(c, kWsSizes);
+    if (dreserve(c, erows, (ne + 1) * 4) || dreserve(c, eoff, (ne + 1) * 4) || dreserve(c, prows, (np + 1) * 4) ||
+        dreserve(c, proff, (np + 1) * 4) || dreserve(c, bcnt, (ne + 1) * 4) || dreserve(c, boff, (ne + 1) * 4) ||
+        dreserve(c, sizes, 64))
+        return set_error(c, RJ_ERR_OOM, "workspace allocation failed");
+    k_edge_rows<<<blocks_for(ne, 256), 256, 0, st>>>(c->edges.as<int4>(), ne, H, erows.as<uint32_t>(),
+                                                     accurate, W, bcnt.as<uint32_t>());
+    RJ_LAUNCHED(c);
+    k_poly_rows<<<blocks_for(np, 256), 256, 0, st>>>(c->mbr.as<int4>(), np, H, prows.as<uint32_t>());
+    RJ_LAUNCHED(c);
+    RJ_CUDA(c, cudaGetLastError());
+    RJ_CUDA(c, scan_u32(c, erows.as<uint32_t>(), eoff.as<uint32_t>(), ne, kWsScan));
+    RJ_CUDA(c, scan_u32(c, prows.as<uint32_t>(), proff.as<uint32_t>(), np, kWsScan));
+    if (accurate) RJ_CUDA(c, scan_u32(c, bcnt.as<uint32_t>(), boff.as<uint32_t>(), ne, kWsScan));
+    // sync 1: crossing / polygon-row / band totals
+    uint32_t *hs = reinterpret_cast<uint32_t *>(c->h_stats + 8);
+    RJ_CUDA(c, cudaMemcpyAsync(hs + 0, eoff.as<uint32_t>() + ne, 4, cudaMemcpyDeviceToHost, st));
+    RJ_CUDA(c, cudaMemcpyAsync(hs + 1, proff.as<uint32_t>() + np, 4, cudaMemcpyDeviceToHost, st));
+    if (accurate) RJ_CUDA(c, cudaMemcpyAsync(hs + 2, boff.as<uint32_t>() + ne, 4, cudaMemcpyDeviceToHost, st));
+    RJ_CUDA(c, cudaStreamSynchronize(st));
+    const uint32_t X = hs[0], NPR = hs[1];
+
+    Buf &cpr = wsbuf(c, kWsCrossPR), &ct = wsbuf(c, kWsCrossT), &prc = wsbuf(c, kWsPRCount);
+    Buf &pro = wsbuf(c, kWsPROff), &prcur = wsbuf(c, kWsPRCursor), &tv = wsbuf(c, kWsTvals);
+    Buf &scnt = wsbuf(c, kWsSpanCount), &soff = wsbuf(c, kWsSpanOff);
+    Buf &pcnt = wsbuf(c, kWsPieceCount), &poff = wsbuf(c, kWsPieceOff), &pcur = wsbuf(c, kWsPieceCursor);
+    if (dreserve(c, cpr, (X + 1) * 4) || dreserve(c, ct, (X + 1) * 4) || dreserve(c, prc, (NPR + 1) * 4) ||
+        dreserve(c, pro, (NPR + 1) * 4) || dreserve(c, prcur, (NPR + 1) * 4) || dreserve(c, tv, (X + 1) * 4) ||
+        dreserve(c, scnt, (NPR + 1) * 4) || dreserve(c, soff, (NPR + 1) * 4) ||
+        dreserve(c, pcnt, (kCells + 1) * 4) || dreserve(c, poff, (kCells + 1) * 4) ||
+        dreserve(c, pcur, (kCells + 1) * 4))
+        return set_error(c, RJ_ERR_OOM, "workspace allocation failed");
+    RJ_CUDA(c, cudaMemsetAsync(prc.p, 0, (NPR + 1) * 4, st));
+    RJ_CUDA(c, cudaMemsetAsync(prcur.p, 0, (NPR + 1) * 4, st));
+    RJ_CUDA(c, cudaMemsetAsync(pcnt.p, 0, (kCells + 1) * 4, st));
+    RJ_CUDA(c, cudaMemsetAsync(pcur.p, 0, (kCells + 1) * 4, st));
+    const unsigned gx = (unsigned)std::min<uint64_t>(std::max<uint64_t>(1, blocks_for(X, 256)), c->num_sms * 8ull);
+    k_crossings<<<gx, 256, 0, st>>>(c->edges.as<int4>(), c->edge_poly.as<uint32_t>(), c->mbr.as<int4>(),
+                                    eoff.as<uint32_t>(), ne, proff.as<uint32_t>(), W, H, cpr.as<uint32_t>(),
+                                    ct.as<uint32_t>(), prc.as<uint32_t>());
+    RJ_LAUNCHED(c);
+    RJ_CUDA(c, cudaGetLastError());
+    RJ_CUDA(c, scan_u32(c, prc.as<uint32_t>(), pro.as<uint32_t>(), NPR, kWsScan));
+    k_scatter_t<<<gx, 256, 0, st>>>(cpr.as<uint32_t>(), ct.as<uint32_t>(), X, pro.as<uint32_t>(),
+                                    prcur.as<uint32_t>(), tv.as<uint32_t>());
+    RJ_LAUNCHED(c);
+    SpanGeo g{W, H, proff.as<uint32_t>(), np, c->mbr.as<int4>(), c->cell_off.as<uint32_t>()};
+    const unsigned gp = (unsigned)std::min<uint64_t>(std::max<uint64_t>(1, blocks_for(NPR, 128)), c->num_sms * 16ull);
+    k_prow_count<<<gp, 128, 0, st>>>(g, NPR, pro.as<uint32_t>(), tv.as<uint32_t>(), scnt.as<uint32_t>(),
+                                     pcnt.as<uint32_t>());
+    RJ_LAUNCHED(c);
+    RJ_CUDA(c, cudaGetLastError());
+    RJ_CUDA(c, scan_u32(c, scnt.as<uint32_t>(), soff.as<uint32_t>(), NPR, kWsScan));
+    RJ_CUDA(c, scan_u32(c, pcnt.as<uint32_t>(), poff.as<uint32_t>(), kCells, kWsScan));
+    // sync 2: span / piece totals
+    RJ_CUDA(c, cudaMemcpyAsync(hs + 3, soff.as<uint32_t>() + NPR, 4, cudaMemcpyDeviceToHost, st));
+    RJ_CUDA(c, cudaMemcpyAsync(hs + 4, poff.as<uint32_t>() + kCells, 4, cudaMemcpyDeviceToHost, st));
+    RJ_CUDA(c, cudaStreamSynchronize(st));
+    const uint32_t S = hs[3], NP = hs[4];
+    Buf &spans = wsbuf(c, kWsSpans), &pieces = wsbuf(c, kWsPieces);
+    if (dreserve(c, spans, (uint64_t)(S + 1) * 16) || dreserve(c, pieces, (uint64_t)(NP + 1) * 8))
+        return set_error(c, RJ_ERR_OOM, "workspace allocation failed");
+    k_prow_emit<<<gp, 128, 0, st>>>(g, NPR, pro.as<uint32_t>(), tv.as<uint32_t>(), soff.as<uint32_t>(),
+                                    spans.as<uint32_t>(), poff.as<uint32_t>(), pcur.as<uint32_t>(),
+                                    pieces.as<uint2>());
+    RJ_LAUNCHED(c);
+    RJ_CUDA(c, cudaGetLastError());
+
+    pp.n_cross = X;
+    pp.n_spans = S;
+    pp.n_pieces = NP;
+    pp.spans = spans.as<uint32_t>();
+    pp.piece_off = poff.as<uint32_t>();
+    pp.pieces = pieces.as<uint2>();
+    if (accurate) {
+        const uint32_t B = hs[2];
+        const uint32_t wpr = (uint32_t)((W + 31) / 32);
+        Buf &mask = wsbuf(c, kWsMask);
+        if (dreserve(c, mask, (uint64_t)wpr * H * 4)) return set_error(c, RJ_ERR_OOM, "mask allocation failed");
+        RJ_CUDA(c, cudaMemsetAsync(mask.p, 0, (uint64_t)wpr * H * 4, st));
+        const unsigned gb = (unsigned)std::min<uint64_t>(std::max<uint64_t>(1, blocks_for(B, 256)), c->num_sms * 8ull);
+        k_mask_mark<<<gb, 256, 0, st>>>(c->edges.as<int4>(), boff.as<uint32_t>(), ne, W, H, wpr, mask.as<uint32_t>());
+        RJ_LAUNCHED(c);
+        RJ_CUDA(c, cudaGetLastError());
+        pp.mask = mask.as<uint32_t>();
+        pp.mask_wpr = wpr;
+    }
+    return RJ_OK;
+}
+
+}  // namespace rj

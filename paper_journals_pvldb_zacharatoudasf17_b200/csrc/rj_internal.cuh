@@ -1,0 +1,167 @@
+// rj_internal.cuh -- private context and launcher declarations of librj.
+#pragma once
+#include <cuda_runtime.h>
+#include <stdint.h>
+
+#include <string>
+#include <vector>
+
+#include "../../include/rj.h"
+#include "rj_geom.cuh"
+
+namespace rj {
+
+struct Ctx;
+
+// Device buffer owned by a context (grow-only when reused as workspace).
+struct Buf {
+    void *p = nullptr;
+    size_t bytes = 0;
+    template <class T> T *as() const { return reinterpret_cast<T *>(p); }
+};
+
+// Attribute slot of the point pass: the distinct columns a query reads.
+struct Filter {
+    int32_t n_slots = 0;          // columns streamed by the point pass (<= 6)
+    int32_t slot_col[6];          // slot -> attribute column
+    int32_t slot_is_float[6];
+    // integer-range predicates: slot s in [0, n_irange) has all its int32
+    // predicates merged into one inclusive range [ilo, ihi]
+    int32_t n_irange = 0;
+    int32_t ilo[6], ihi[6];
+    // float32 predicates (slot, op, value)
+    int32_t n_fpred = 0;
+    int32_t f_slot[5], f_op[5];
+    float f_val[5];
+    int32_t never = 0;            // an int predicate can never hold
+    int32_t agg_slot = -1;        // slot of the summed attribute (SUM/AVG)
+};
+
+// Device-side parameter block of the fused point pass.
+struct PassArgs {
+    const uint32_t *qx, *qy;
+    const uint32_t *col[6];
+    Filter f;
+    int32_t W, H;
+    const int4 *items;
+    uint32_t n_items;
+    uint32_t *work_counter;
+    const uint32_t *piece_off;    // [kCells + 1]
+    const uint2 *pieces;
+    const uint32_t *mask;         // accurate: boundary bitmask
+    uint32_t mask_wpr;
+    const uint32_t *grid_off;     // accurate: edge grid CSR
+    const uint32_t *grid_ent;
+    const int4 *edges;
+    const uint32_t *edge_poly;
+    unsigned long long *A_cnt;    // per polygon partials (device)
+    double *A_sum;
+    uint32_t n_poly;
+    int32_t smem_partials;        // accumulate per-CTA polygon partials in smem
+    uint32_t tile_cap;            // pixels of the largest tile
+    unsigned long long *stats;    // [0] filtered, [1] boundary
+};
+
+struct Ctx {
+    int device = 0;
+    cudaStream_t stream = nullptr;
+    bool own_stream = false;
+    double x0, y0, x1, y1;
+    bool poisoned = false;
+    std::string err;
+    void *(*alloc_fn)(size_t, void *) = nullptr;
+    void (*free_fn)(void *, void *) = nullptr;
+    void *alloc_user = nullptr;
+    int num_sms = 148;
+    int timing = 0;
+    int64_t chunk = 32768;
+
+    // points (S1 output, spatially sorted)
+    uint64_t n_in = 0, n_pts = 0;
+    int n_cols = 0;
+    int col_dtype[RJ_MAX_COLS];
+    Buf qx, qy, idx, col[RJ_MAX_COLS];
+    Buf cell_off;                 // [kCells + 1]
+    Buf items;                    // int4 (cell, begin, end, 0)
+    uint32_t n_items = 0;
+    int64_t items_chunk = 0;
+
+    // polygons
+    uint32_t n_poly = 0;
+    uint32_t n_edges = 0;
+    Buf edges, edge_poly, poly_edge_off, mbr;   // int4 edges/mbr
+    Buf grid_off, grid_ent;
+    uint64_t n_grid_ent = 0;
+
+    // query workspace (grow-only)
+    Buf ws[64];                      // slots: see kWs* in rj_internal.cuh
+    Buf res_cnt, res_sum, res_val;   // per-polygon partials / values
+    Buf stats_dev;
+    unsigned long long *h_stats = nullptr;   // pinned
+    rj_stats last{};
+    cudaEvent_t ev[6] = {};
+    uint32_t launches = 0;
+};
+
+// workspace slot map (Ctx::ws)
+enum : int {
+    kWsSortCounts = 0, kWsSortBuf = 1,      // 1..12 double buffers of the radix sort
+    kWsEdgeRows = 14, kWsEdgeOff, kWsPolyRows, kWsPolyRowOff, kWsCrossPR, kWsCrossT,
+    kWsPRCount, kWsPROff, kWsPRCursor, kWsTvals, kWsSpanCount, kWsSpanOff, kWsSpans,
+    kWsPieceCount, kWsPieceOff, kWsPieceCursor, kWsPieces, kWsMask, kWsBandCount, kWsBandOff,
+    kWsWork, kWsSizes,
+    kWsScan = 44,                           // 44..63 recursive scan temporaries
+};
+
+// allocation helpers (ctx allocator if set)
+cudaError_t dalloc(Ctx *c, Buf &b, size_t bytes);
+void dfree(Ctx *c, Buf &b);
+cudaError_t dreserve(Ctx *c, Buf &b, size_t bytes);   // grow-only
+Buf &wsbuf(Ctx *c, int slot);
+
+// scan.cu: exclusive scan of n u32 -> out[0..n], out[n] = total.  tmp
+// workspace slots base.. are used for block sums.
+cudaError_t scan_u32(Ctx *c, const uint32_t *in, uint32_t *out, uint64_t n, int ws_base);
+
+// load_points.cu
+rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int xy_f64,
+                           int n_cols, const void *const *cols, const int32_t *dtypes,
+                           uint64_t *n_ood);
+rj_status build_items(Ctx *c);
+
+// polygons.cu
+rj_status load_polygons_impl(Ctx *c, uint32_t n_poly, const uint32_t *pro, const uint32_t *rvo,
+                             const double *vx, const double *vy);
+struct PolyPass {
+    uint64_t n_cross = 0, n_spans = 0, n_pieces = 0;
+    uint32_t *spans = nullptr;       // 4 x u32 per span (poly,row,lo,hi), (poly,row,lo)-sorted
+    uint32_t *piece_off = nullptr;   // [kCells + 1]
+    uint2 *pieces = nullptr;
+    uint32_t *mask = nullptr;        // accurate only
+    uint32_t mask_wpr = 0;
+};
+rj_status polygon_pass(Ctx *c, int W, int H, bool accurate, PolyPass &pp);
+
+// pass.cu
+rj_status point_pass(Ctx *c, const PassArgs &a, bool sum, bool accurate);
+size_t point_pass_smem(const PassArgs &a, bool sum, bool accurate);
+
+// misc.cu
+cudaError_t launch_finalize(Ctx *c, int agg, uint32_t n, const unsigned long long *cnt,
+                            const double *sum, double *val);
+cudaError_t launch_membership(Ctx *c, const PassArgs &a, bool accurate, unsigned long long *bits);
+
+rj_status set_error(Ctx *c, rj_status s, const std::string &msg);
+rj_status cuda_error(Ctx *c, cudaError_t e, const char *where);
+
+#define RJ_CUDA(c, expr)                                            \
+    do {                                                            \
+        cudaError_t _e = (expr);                                    \
+        if (_e != cudaSuccess) return ::rj::cuda_error((c), _e, #expr); \
+    } while (0)
+
+#define RJ_LAUNCHED(c) do { (c)->launches++; } while (0)
+
+inline unsigned blocks_for(uint64_t n, unsigned t) { return (unsigned)((n + t - 1) / t); }
+
+}  // namespace rj

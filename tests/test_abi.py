@@ -1,0 +1,82 @@
+"""C-ABI boundary checks that need no GPU: the library builds and loads,
+exports every entry point include/rj.h declares, and its host-only logic
+(S0 canvas resolution) follows the readings in DESIGN.md."""
+import math
+import os
+import re
+
+import pytest
+
+import oracle
+from paper_journals_pvldb_zacharatoudasf17_b200 import _build, rj
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+
+
+@pytest.fixture(scope="module")
+def L():
+    _build.build()
+    return rj.lib()
+
+
+def header_functions():
+    src = open(os.path.join(ROOT, "include", "rj.h")).read()
+    src = re.sub(r"/\*.*?\*/", "", src, flags=re.S)
+    return sorted(set(re.findall(r"\b(rj_[a-z_]+)\s*\(", src)))
+
+
+def test_exports_every_declared_symbol(L):
+    names = header_functions()
+    assert len(names) >= 18
+    for n in names:
+        assert hasattr(L, n), n
+    assert set(names) == set(rj.EXPORTS)
+
+
+def test_version_and_status_strings(L):
+    assert b"sm_100a" in L.rj_version()
+    for code, name in rj.STATUS.items():
+        assert L.rj_status_str(code).decode() == name
+
+
+@pytest.mark.parametrize("eps,W", [(80, 1024), (40, 2048), (20, 4096), (10, 8192)])
+def test_resolve_epsilon_nyc(L, eps, W):
+    q = rj.make_desc(epsilon=eps)
+    assert rj.rj_resolve_canvas_domain((0, 0, 57920, 57920), q) == (W, W)
+    assert oracle.resolve(57920, 57920, eps) == (W, W)      # same reading on both sides
+
+
+def test_resolve_us_and_errors(L):
+    assert rj.rj_resolve_canvas_domain((0, 0, 4.6e6, 2.9e6), rj.make_desc(epsilon=1000.0)) == (6506, 4102)
+    assert rj.rj_resolve_canvas_domain((0, 0, 1, 1), rj.make_desc(W=640, H=480)) == (640, 480)
+    for q in (rj.make_desc(epsilon=0.0), rj.make_desc(epsilon=float("nan")), rj.make_desc(W=32769),
+              rj.make_desc(epsilon=1.0)):    # eps = 1 m on NYC -> 81912 > 32768
+        box = (0, 0, 57920, 57920)
+        with pytest.raises(rj.RJError) as e:
+            rj.rj_resolve_canvas_domain(box, q)
+        assert e.value.status == -3
+
+
+def test_create_without_gpu_fails_loudly(L):
+    import torch
+    if torch.cuda.is_available():
+        pytest.skip("a GPU is present")
+    with pytest.raises(rj.RJError) as e:
+        rj.rj_create(0, None, (0, 0, 1, 1))
+    assert e.value.status == -6
+
+
+def test_create_rejects_bad_domain(L):
+    for box in ((0, 0, 0, 1), (1, 0, 0, 1), (0, 0, math.inf, 1), (0, 0, 1, math.nan)):
+        with pytest.raises(rj.RJError) as e:
+            rj.rj_create(0, None, box)
+        assert e.value.status == -1
+
+
+def test_product_never_imports_oracle():
+    pkg = os.path.join(ROOT, "paper_journals_pvldb_zacharatoudasf17_b200")
+    for dp, _, fs in os.walk(pkg):
+        for f in fs:
+            if f.endswith((".py", ".cu", ".cuh", ".h", ".cpp")):
+                s = open(os.path.join(dp, f)).read()
+                assert "import oracle" not in s and "from oracle" not in s and "rj_oracle" not in s, f

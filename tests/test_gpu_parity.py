@@ -1,0 +1,289 @@
+"""GPU parity: the CUDA path (through the C ABI) against the CPU oracle,
+element by element on the same seeded inputs.
+
+Bar (BASELINE.json north_star): COUNT, pixel spans,
+boundary mask and point membership bit-exact; SUM/AVG within 1e-9 relative
+(exact for integer attributes).  Sizes span many tiles / work items and a
+ragged tail; the edge cases cover empty and degenerate inputs.
+"""
+import math
+
+import numpy as np
+import pytest
+
+import oracle
+from datagen import configs as C
+from datagen import polygons as PG
+
+pytestmark = pytest.mark.gpu
+
+rjmod = pytest.importorskip("paper_journals_pvldb_zacharatoudasf17_b200.rj")
+
+
+@pytest.fixture(scope="module", autouse=True)
+def _gpu():
+    import torch
+    if not torch.cuda.is_available():
+        pytest.skip("needs a CUDA device")
+
+
+def gpu_ctx(box, polys_flat, x, y, cols=(), chunk=None):
+    R = rjmod.RasterJoin(box)
+    if chunk:
+        R.set_option(rjmod.OPT_CHUNK, chunk)
+    R.load_points(x, y, cols)
+    R.load_polygons(polys_flat)
+    return R
+
+
+def rel_close(g, o, tol=1e-9):
+    g = np.asarray(g, np.float64)
+    o = np.asarray(o, np.float64)
+    both_nan = np.isnan(g) & np.isnan(o)
+    ok = both_nan | (np.abs(g - o) <= tol * np.abs(o)) | ((o == 0) & (g == 0))
+    return bool(np.all(ok)), np.nonzero(~ok)[0]
+
+
+# ------------------------------------------------------------------------ C1
+@pytest.fixture(scope="module")
+def c1():
+    polys = C.polygon_set("c1b")
+    flat = PG.flatten(polys)
+    pts = C.c1_points()
+    ax, ay = PG.c1b_points(polys)
+    x = np.concatenate([pts["x"], ax])
+    y = np.concatenate([pts["y"], ay])
+    rng = np.random.default_rng(11)
+    ti = rng.integers(-50, 50, len(x)).astype(np.int32)
+    tf = rng.normal(5, 3, len(x)).astype(np.float32)
+    tf[::97] = np.nan
+    return flat, x, y, [ti, tf]
+
+
+@pytest.mark.parametrize("mode", ["bounded", "accurate"])
+@pytest.mark.parametrize("chunk", [None, 256])
+def test_c1_count_bitexact(c1, mode, chunk):
+    flat, x, y, cols = c1
+    R = gpu_ctx(C.C1_BOX, flat, x, y, cols, chunk=chunk)
+    P = oracle.Polys(flat, C.C1_BOX)
+    cnt, val = R.query(W=1024, H=1024, mode=mode)
+    ocnt, _, kept = oracle.query(P, x, y, W=1024, H=1024, mode=mode)
+    assert np.array_equal(cnt, ocnt), (cnt, ocnt)
+    assert np.array_equal(val, ocnt.astype(np.float64))
+    st = R.stats()
+    assert st["n_filtered"] == kept == len(x)
+    if mode == "accurate":
+        assert st["n_boundary"] > 0
+
+
+@pytest.mark.parametrize("W,H", [(1, 1), (5, 7), (64, 64), (333, 517), (1000, 700), (4096, 4096), (32768, 32768)])
+@pytest.mark.parametrize("mode", ["bounded", "accurate"])
+def test_c1_resolutions(c1, W, H, mode):
+    flat, x, y, cols = c1
+    R = gpu_ctx(C.C1_BOX, flat, x, y, cols)
+    P = oracle.Polys(flat, C.C1_BOX)
+    cnt, _ = R.query(W=W, H=H, mode=mode)
+    ocnt, _, _ = oracle.query(P, x, y, W=W, H=H, mode=mode)
+    assert np.array_equal(cnt, ocnt)
+
+
+def _merge_touching(sp):
+    """(row, lo, hi) spans sorted by (row, lo) -> maximal runs.  Even-odd
+    pairing of sorted thresholds can emit two spans that touch ([a,b), [b,c)
+    for a self-intersecting ring); the pixel set is what is unique."""
+    out = []
+    for r, lo, hi in sp.tolist():
+        if out and out[-1][0] == r and out[-1][2] == lo:
+            out[-1][2] = hi
+        else:
+            out.append([r, lo, hi])
+    return np.asarray(out, dtype=np.int64).reshape(-1, 3)
+
+
+@pytest.mark.parametrize("W,H", [(1024, 1024), (333, 517), (64, 48)])
+def test_pixel_spans_bitexact(c1, W, H):
+    flat, x, y, cols = c1
+    R = gpu_ctx(C.C1_BOX, flat, x, y, cols)
+    P = oracle.Polys(flat, C.C1_BOX)
+    sp = R.spans(W=W, H=H)
+    for pid in range(P.n):
+        g = _merge_touching(sp[sp[:, 0] == pid][:, 1:].astype(np.int64))
+        o = oracle.pixel_spans(P, pid, W, H).astype(np.int64)
+        assert np.array_equal(g, o), pid
+
+
+@pytest.mark.parametrize("W,H", [(1024, 1024), (200, 300), (4096, 4096)])
+def test_boundary_mask_bitexact(c1, W, H):
+    flat, x, y, cols = c1
+    R = gpu_ctx(C.C1_BOX, flat, x, y, cols)
+    P = oracle.Polys(flat, C.C1_BOX)
+    g = R.boundary_mask(W=W, H=H)
+    o = oracle.boundary_mask(P, W, H)
+    assert np.array_equal(g, o)
+
+
+@pytest.mark.parametrize("mode", ["bounded", "accurate"])
+@pytest.mark.parametrize("W", [1024, 97])
+def test_point_membership_bitexact(c1, mode, W):
+    flat, x, y, cols = c1
+    R = gpu_ctx(C.C1_BOX, flat, x, y, cols)
+    P = oracle.Polys(flat, C.C1_BOX)
+    preds = [(0, ">=", -20.5), (1, "<", 7.25)]
+    g = R.membership(W=W, H=W, mode=mode, preds=preds)
+    o = oracle.membership(P, x, y, cols=cols, preds=preds, W=W, H=W, mode=mode)
+    assert np.array_equal(g, o)
+
+
+@pytest.mark.parametrize("mode", ["bounded", "accurate"])
+def test_sum_avg_filters(c1, mode):
+    flat, x, y, cols = c1
+    R = gpu_ctx(C.C1_BOX, flat, x, y, cols)
+    P = oracle.Polys(flat, C.C1_BOX)
+    cases = [
+        dict(agg="sum", agg_column=0, preds=[]),                                   # integer SUM: exact
+        dict(agg="sum", agg_column=1, preds=[(0, ">", -10.5)]),
+        dict(agg="avg", agg_column=1, preds=[(1, ">=", 2.0), (1, "<=", 8.0)]),
+        dict(agg="avg", agg_column=0, preds=[(0, "==", 7.0)]),
+        dict(agg="count", preds=[(0, "==", 7.5)]),                                 # never
+        dict(agg="count", preds=[(0, "<", 1e12), (1, ">", -1e30)]),
+        dict(agg="avg", agg_column=0, preds=[(0, ">=", 10), (0, "<", 10)]),       # empty range: NaN
+    ]
+    for cs in cases:
+        cnt, val = R.query(W=1024, H=1024, mode=mode, **cs)
+        pc = [(c_, op, v) for c_, op, v in cs["preds"]]
+        ocnt, osum, _ = oracle.query(P, x, y, cols=cols, preds=pc, agg_col=cs.get("agg_column", -1),
+                                     W=1024, H=1024, mode=mode)
+        assert np.array_equal(cnt, ocnt), cs
+        if cs["agg"] == "sum":
+            if cs["agg_column"] == 0:
+                assert np.array_equal(val, osum), cs
+            ok, bad = rel_close(val, osum)
+            assert ok, (cs, bad)
+        elif cs["agg"] == "avg":
+            ok, bad = rel_close(val, oracle.avg(ocnt, osum))
+            assert ok, (cs, bad)
+
+
+# ------------------------------------------------------------- edge cases
+def test_empty_and_degenerate_point_sets():
+    flat = PG.flatten(C.polygon_set("c1"))
+    P = oracle.Polys(flat, C.C1_BOX)
+    for n in (0, 1, 7, 8, 9, 255, 257):
+        pts = C.c1_points(n) if n else {"x": np.zeros(0), "y": np.zeros(0)}
+        R = gpu_ctx(C.C1_BOX, flat, pts["x"], pts["y"])
+        for mode in ("bounded", "accurate"):
+            cnt, val = R.query(W=1024, mode=mode, agg="count")
+            ocnt, _, _ = oracle.query(P, pts["x"], pts["y"], W=1024, H=1024, mode=mode)
+            assert np.array_equal(cnt, ocnt), n
+        R.close()
+    # all points out of domain (and on x = X1 exactly, NaN)
+    x = np.array([-1.0, 1024.0, 5.0, np.nan, 2000.0])
+    y = np.array([5.0, 5.0, 1024.0, 5.0, -3.0])
+    R = rjmod.RasterJoin(C.C1_BOX)
+    assert R.load_points(x, y) == 5
+    R.load_polygons(flat)
+    cnt, val = R.query(W=64, mode="accurate", agg="count")
+    assert cnt.sum() == 0 and R.stats()["n_points"] == 0
+
+
+def test_float32_coords_and_device_pointers():
+    import torch
+    flat = PG.flatten(C.polygon_set("c1"))
+    P = oracle.Polys(flat, C.C1_BOX)
+    pts = C.c1_points(50000)
+    x32, y32 = pts["x"].astype(np.float32), pts["y"].astype(np.float32)
+    R = rjmod.RasterJoin(C.C1_BOX)
+    R.load_points(torch.from_numpy(x32).cuda(), torch.from_numpy(y32).cuda())
+    R.load_polygons(flat)
+    cnt, _ = R.query(W=777, H=555, mode="accurate")
+    ocnt, _, _ = oracle.query(P, x32, y32, W=777, H=555, mode="accurate")
+    assert np.array_equal(cnt, ocnt)
+
+
+def test_errors():
+    flat = PG.flatten(C.polygon_set("c1"))
+    R = rjmod.RasterJoin(C.C1_BOX)
+    with pytest.raises(rjmod.RJError) as e:
+        R.n_poly = 10
+        R.query(W=64)
+    assert e.value.status == -1                       # query before load
+    pts = C.c1_points(100)
+    R.load_points(pts["x"], pts["y"], [np.zeros(100, np.int32)])
+    R.load_polygons(flat)
+    for kw in (dict(agg="sum", agg_column=3), dict(preds=[(5, "<", 1)]), dict(preds=[(0, "<", 1)] * 6)):
+        with pytest.raises((rjmod.RJError, ValueError)):
+            R.query(W=64, **kw)
+    with pytest.raises(rjmod.RJError) as e:
+        R.query(W=40000)
+    assert e.value.status == -3
+    bad = PG.flatten([[np.array([(0, 0), (2000, 0), (0, 5)], float)]])
+    with pytest.raises(rjmod.RJError) as e:
+        R.load_polygons(bad)
+    assert e.value.status == -2
+    tri2 = (np.array([0, 1], np.uint32), np.array([0, 2], np.uint32), np.zeros(2), np.zeros(2))
+    with pytest.raises(rjmod.RJError) as e:
+        R.load_polygons(tri2)
+    assert e.value.status == -1
+
+
+# ------------------------------------------------------ realistic workloads
+@pytest.mark.parametrize("W", [8192, 4096, 1500])
+def test_taxi_neighborhoods_bounded_time_filter(W):
+    """C2 shape on a 2M-point prefix: COUNT, calendar-2012 filter, bounded."""
+    flat = C.array_polys("neighborhoods")
+    pts = C.taxi(2_000_000)
+    R = gpu_ctx(C.NYC_BOX, flat, pts["x"], pts["y"], [pts["t"]])
+    P = oracle.Polys(flat, C.NYC_BOX)
+    preds = [(0, ">=", C.T_2012[0]), (0, "<", C.T_2012[1])]
+    cnt, _ = R.query(W=W, H=W, mode="bounded", preds=preds)
+    ocnt, _, kept = oracle.query(P, pts["x"], pts["y"], cols=[pts["t"]], preds=preds, W=W, H=W, mode="bounded")
+    assert np.array_equal(cnt, ocnt)
+    assert int(cnt.sum()) == kept == R.stats()["n_filtered"]          # exact tiling
+
+
+def test_tracts_accurate_avg_fare():
+    """C3 shape on a 1M-point prefix: AVG(fare), accurate, 8192^2."""
+    flat = C.array_polys("tracts")
+    pts = C.taxi(1_000_000, fare=True)
+    R = gpu_ctx(C.NYC_BOX, flat, pts["x"], pts["y"], [pts["t"], pts["fare"]])
+    P = oracle.Polys(flat, C.NYC_BOX)
+    cnt, val = R.query(W=8192, H=8192, mode="accurate", agg="avg", agg_column=1)
+    ocnt, osum, kept = oracle.query(P, pts["x"], pts["y"], cols=[pts["t"], pts["fare"]], agg_col=1,
+                                    W=8192, H=8192, mode="accurate")
+    assert np.array_equal(cnt, ocnt)
+    ok, bad = rel_close(val, oracle.avg(ocnt, osum))
+    assert ok, bad
+    st = R.stats()
+    assert st["n_boundary"] > 0 and int(cnt.sum()) == kept
+
+
+def test_counties_sum_fav_epsilon():
+    """C4 shape on a 1M-point prefix: SUM(fav) + COUNT, bounded, eps = 1 km."""
+    flat = C.array_polys("counties")
+    pts = C.twitter(1_000_000)
+    R = gpu_ctx(C.US_BOX, flat, pts["x"], pts["y"], [pts["fav"]])
+    P = oracle.Polys(flat, C.US_BOX)
+    cnt, val = R.query(epsilon=1000.0, mode="bounded", agg="sum", agg_column=0)
+    assert R.stats()["W"] == 6506 and R.stats()["H"] == 4102
+    ocnt, osum, _ = oracle.query(P, pts["x"], pts["y"], cols=[pts["fav"]], agg_col=0, W=6506, H=4102,
+                                 mode="bounded")
+    assert np.array_equal(cnt, ocnt)
+    assert np.array_equal(val, osum)            # integer attribute: bit-exact
+
+
+def test_sharding_sums_to_unsharded():
+    """Point shards add up (distributive aggregates)."""
+    flat = C.array_polys("neighborhoods")
+    pts = C.taxi(600_000, fare=True)
+    whole = gpu_ctx(C.NYC_BOX, flat, pts["x"], pts["y"], [pts["fare"]])
+    c_all, s_all = whole.query(W=4096, mode="accurate", agg="sum", agg_column=0)
+    acc_c = np.zeros_like(c_all)
+    acc_s = np.zeros_like(s_all)
+    for lo, hi in ((0, 200_000), (200_000, 450_000), (450_000, 600_000)):
+        R = gpu_ctx(C.NYC_BOX, flat, pts["x"][lo:hi], pts["y"][lo:hi], [pts["fare"][lo:hi]])
+        c, s = R.query(W=4096, mode="accurate", agg="sum", agg_column=0)
+        acc_c += c
+        acc_s += s
+    assert np.array_equal(acc_c, c_all)
+    ok, _ = rel_close(acc_s, s_all)
+    assert ok

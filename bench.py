@@ -201,6 +201,7 @@ def main():
     ap.add_argument("--scaling", default="weak", choices=("weak", "strong"))
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--e2e-steps", type=int, default=2)
+    ap.add_argument("--chunk", type=int, default=0, help="points per work item (0 = library default)")
     args = ap.parse_args()
     args.warmup = max(3, args.warmup)
 
@@ -233,6 +234,8 @@ def main():
 
     stream = torch.cuda.Stream()
     R = rj.RasterJoin(box, device=local, stream=stream.cuda_stream)
+    if args.chunk:
+        R.set_option(rj.OPT_CHUNK, args.chunk)
     flat = C.array_polys(polys_name)
     t0 = time.perf_counter()
     n_ood = R.load_points(x, y, cols)

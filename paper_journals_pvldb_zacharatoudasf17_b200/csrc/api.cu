@@ -153,6 +153,8 @@ static rj_status build_filter(Ctx *c, const rj_query_desc *q, Filter &f) {
         f.f_val[f.n_fpred] = (float)p.value;
         f.n_fpred++;
     }
+    // slots without an int range always pass the (unconditional) range check
+    for (int s = f.n_irange; s < 6; ++s) { f.ilo[s] = INT32_MIN; f.ihi[s] = INT32_MAX; }
     if (q->agg != RJ_COUNT) {
         if (slot_of[q->agg_column] < 0) {
             slot_of[q->agg_column] = f.n_slots;
@@ -161,22 +163,24 @@ static rj_status build_filter(Ctx *c, const rj_query_desc *q, Filter &f) {
             f.n_slots++;
         }
         f.agg_slot = slot_of[q->agg_column];
+        f.agg_is_float = f.slot_is_float[f.agg_slot];
     }
     return RJ_OK;
 }
 
-// Largest point tile (pixels) of a W x H canvas: 256x256 cells, <= 129 x 129.
-static uint32_t tile_cap(int W, int H) {
+// Largest point tile of a W x H canvas at cell level L: (rows, odd row stride).
+static void tile_geometry(int W, int H, int L, uint32_t &stride, uint32_t &cap) {
     int64_t mw = 0, mh = 0;
-    for (int64_t k = 0; k < (1 << kCellBits); ++k) {
-        mw = std::max(mw, cell_pix_hi(k, W) - cell_pix_lo(k, W) + 1);
-        mh = std::max(mh, cell_pix_hi(k, H) - cell_pix_lo(k, H) + 1);
+    for (int64_t k = 0; k < (int64_t(1) << L); ++k) {
+        mw = std::max(mw, cell_pix_hi(k, W, L) - cell_pix_lo(k, W, L) + 1);
+        mh = std::max(mh, cell_pix_hi(k, H, L) - cell_pix_lo(k, H, L) + 1);
     }
-    return (uint32_t)(mw * mh);
+    stride = (uint32_t)(mw | 1);
+    cap = (uint32_t)(mh * stride);
 }
 
 struct Prepared {
-    int W, H;
+    int W, H, L;
     bool sum, acc;
     PolyPass pp;
     PassArgs a;
@@ -202,10 +206,11 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     if ((s = build_filter(c, q, f)) != RJ_OK) return s;
     P.sum = q->agg != RJ_COUNT;
     P.acc = q->mode == RJ_ACCURATE;
-    if (c->items_chunk != c->chunk && (s = build_items(c)) != RJ_OK) return s;
+    P.L = choose_level(P.W, P.H, P.sum);
+    if ((s = items_for_level(c, P.L)) != RJ_OK) return s;
     c->launches = 0;
     if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[0], c->stream));
-    if (need_polygon_pass && (s = polygon_pass(c, P.W, P.H, P.acc, P.pp)) != RJ_OK) return s;
+    if (need_polygon_pass && (s = polygon_pass(c, P.W, P.H, P.L, P.acc, P.pp)) != RJ_OK) return s;
     if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[1], c->stream));
     PassArgs &a = P.a;
     memset(&a, 0, sizeof(a));
@@ -215,8 +220,10 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     a.f = f;
     a.W = P.W;
     a.H = P.H;
-    a.items = c->items.as<int4>();
-    a.n_items = c->n_items;
+    a.items = c->items[P.L].as<int4>();
+    a.n_items = c->n_items[P.L];
+    a.level = P.L;
+    a.cell_off10 = c->cell_off.as<uint32_t>();
     a.piece_off = P.pp.piece_off;
     a.pieces = P.pp.pieces;
     a.mask = P.pp.mask;
@@ -226,7 +233,8 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     a.edges = c->edges.as<int4>();
     a.edge_poly = c->edge_poly.as<uint32_t>();
     a.n_poly = c->n_poly;
-    a.tile_cap = tile_cap(P.W, P.H);
+    tile_geometry(P.W, P.H, P.L, a.tile_stride, a.tile_cap);
+    a.n_stages = (uint32_t)point_pass_stages(f.n_slots);
     a.smem_partials = 1;
     if (point_pass_smem(a, P.sum, P.acc) > 160 * 1024) a.smem_partials = 0;
     Buf &st = wsbuf(c, kWsWork);
@@ -255,7 +263,7 @@ static rj_status run_pass(Ctx *c, Prepared &P, unsigned long long *d_cnt, double
     L.n_crossings = P.pp.n_cross;
     L.n_spans = P.pp.n_spans;
     L.n_pieces = P.pp.n_pieces;
-    L.n_items = c->n_items;
+    L.n_items = c->n_items[P.L];
     L.stream_bytes = c->n_pts * (8ull + 4ull * (uint64_t)a.f.n_slots);
     return RJ_OK;
 }
@@ -337,7 +345,7 @@ rj_status rj_destroy(rj_ctx *c) {
     cudaStreamSynchronize(c->stream);
     dfree(c, c->qx); dfree(c, c->qy); dfree(c, c->idx);
     for (auto &b : c->col) dfree(c, b);
-    dfree(c, c->cell_off); dfree(c, c->items);
+    dfree(c, c->cell_off); drop_items(c);
     dfree(c, c->edges); dfree(c, c->edge_poly); dfree(c, c->poly_edge_off); dfree(c, c->mbr);
     dfree(c, c->grid_off); dfree(c, c->grid_ent);
     for (auto &b : c->ws) dfree(c, b);

@@ -9,8 +9,10 @@
 //     (Qx >> 14, Qy >> 14); out-of-domain points form a 257th digit and sink
 //     to the end.  Payload columns (Qx, Qy, original index, attributes) move
 //     with the keys, so the point pass later streams contiguous columns.
-//  3. cell_off: start of every 256x256 Morton cell (top 16 key bits) -- the
-//     point tiles of the fused pass; work items = cells split into chunks.
+//  3. cell_off: start of every level-10 (1024x1024) Morton cell; a cell of
+//     any coarser level L is the union of 4^(10-L) consecutive level-10
+//     cells, so the point tiles of every query resolution are contiguous
+//     ranges (work items: work.cu).
 #include <algorithm>
 
 #include "rj_internal.cuh"
@@ -120,38 +122,18 @@ __global__ void __launch_bounds__(kSortThreads) k_radix_scatter(Payload pl, uint
     }
 }
 
+// cell_off[c] = first sorted point of level-10 cell c (Morton order);
+// out-of-domain points (sorted last) count as cell kCells10.
 __global__ void k_cell_bounds(const uint32_t *__restrict__ qx, const uint32_t *__restrict__ qy,
                               uint64_t n, uint32_t *__restrict__ cell_off) {
     for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i <= n;
          i += (uint64_t)gridDim.x * blockDim.x) {
-        const int64_t c = (i < n && qx[i] != kInvalid) ? (int64_t)cell_of(qx[i], qy[i]) : (int64_t)kCells;
+        const int64_t c = (i < n && qx[i] != kInvalid) ? (int64_t)cell_of(qx[i], qy[i], kMaxLevel)
+                                                       : (int64_t)kCells10;
         const int64_t p = i == 0 ? -1
-                                 : ((qx[i - 1] != kInvalid) ? (int64_t)cell_of(qx[i - 1], qy[i - 1])
-                                                            : (int64_t)kCells);
+                                 : ((qx[i - 1] != kInvalid) ? (int64_t)cell_of(qx[i - 1], qy[i - 1], kMaxLevel)
+                                                            : (int64_t)kCells10);
         for (int64_t cc = p + 1; cc <= c; ++cc) cell_off[cc] = (uint32_t)i;
-    }
-}
-
-__global__ void k_item_count(const uint32_t *__restrict__ cell_off, uint32_t chunk,
-                             uint32_t *__restrict__ cnt) {
-    const int c = blockIdx.x * blockDim.x + threadIdx.x;
-    if (c < kCells) {
-        const uint32_t m = cell_off[c + 1] - cell_off[c];
-        cnt[c] = (m + chunk - 1) / chunk;
-    }
-}
-
-__global__ void k_item_fill(const uint32_t *__restrict__ cell_off, const uint32_t *__restrict__ ioff,
-                            int4 *__restrict__ items) {
-    const int c = blockIdx.x * blockDim.x + threadIdx.x;
-    if (c < kCells) {
-        const uint32_t b = cell_off[c], m = cell_off[c + 1] - b;
-        const uint32_t k0 = ioff[c], ni = ioff[c + 1] - k0;
-        for (uint32_t k = 0; k < ni; ++k) {
-            const uint32_t lo = b + (uint32_t)(((uint64_t)m * k) / ni);
-            const uint32_t hi = b + (uint32_t)(((uint64_t)m * (k + 1)) / ni);
-            items[k0 + k] = make_int4(c, (int)lo, (int)hi, 0);
-        }
     }
 }
 
@@ -177,40 +159,14 @@ static rj_status stage(Ctx *c, const void *p, size_t bytes, Buf &tmp, const void
     return RJ_OK;
 }
 
-rj_status build_items(Ctx *c) {
-    Buf cnt, off;
-    if (dalloc(c, cnt, (kCells + 1) * 4) != cudaSuccess || dalloc(c, off, (kCells + 1) * 4) != cudaSuccess)
-        return set_error(c, RJ_ERR_OOM, "item allocation failed");
-    const uint32_t chunk = (uint32_t)std::max<int64_t>(256, std::min<int64_t>(c->chunk, 1 << 30));
-    k_item_count<<<kCells / 256, 256, 0, c->stream>>>(c->cell_off.as<uint32_t>(), chunk, cnt.as<uint32_t>());
-    RJ_LAUNCHED(c);
-    RJ_CUDA(c, cudaGetLastError());
-    RJ_CUDA(c, scan_u32(c, cnt.as<uint32_t>(), off.as<uint32_t>(), kCells, kWsScan));
-    uint32_t n_items = 0;
-    RJ_CUDA(c, cudaMemcpyAsync(&n_items, off.as<uint32_t>() + kCells, 4, cudaMemcpyDeviceToHost, c->stream));
-    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
-    dfree(c, c->items);
-    if (dalloc(c, c->items, std::max<size_t>(1, n_items) * sizeof(int4)) != cudaSuccess)
-        return set_error(c, RJ_ERR_OOM, "item allocation failed");
-    k_item_fill<<<kCells / 256, 256, 0, c->stream>>>(c->cell_off.as<uint32_t>(), off.as<uint32_t>(),
-                                                      c->items.as<int4>());
-    RJ_LAUNCHED(c);
-    RJ_CUDA(c, cudaGetLastError());
-    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
-    dfree(c, cnt);
-    dfree(c, off);
-    c->n_items = n_items;
-    c->items_chunk = c->chunk;
-    return RJ_OK;
-}
-
 rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int xy_f64, int n_cols,
                            const void *const *cols, const int32_t *dtypes, uint64_t *n_ood) {
     // drop the previous point set
     dfree(c, c->qx); dfree(c, c->qy); dfree(c, c->idx);
     for (int k = 0; k < RJ_MAX_COLS; ++k) dfree(c, c->col[k]);
-    dfree(c, c->cell_off); dfree(c, c->items);
-    c->n_in = c->n_pts = 0; c->n_items = 0; c->n_cols = 0;
+    dfree(c, c->cell_off);
+    drop_items(c);
+    c->n_in = c->n_pts = 0; c->n_cols = 0;
 
     const size_t esz = xy_f64 ? 8 : 4;
     Buf sx, sy, scol[RJ_MAX_COLS];
@@ -226,7 +182,8 @@ rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int
     const int P = 3 + n_cols;
     Buf A[kMaxPayload], B[kMaxPayload];
     for (int k = 0; k < P; ++k)
-        if (dalloc(c, A[k], nn * 4) != cudaSuccess || dalloc(c, B[k], nn * 4) != cudaSuccess)
+        // +8 points of padding: the point pass copies 16-B aligned supersets of ranges
+        if (dalloc(c, A[k], (nn + 8) * 4) != cudaSuccess || dalloc(c, B[k], (nn + 8) * 4) != cudaSuccess)
             return set_error(c, RJ_ERR_OOM, "point buffers allocation failed");
 
     if (n) {
@@ -276,7 +233,7 @@ rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int
     c->n_cols = n_cols;
     c->n_in = n;
 
-    if (dalloc(c, c->cell_off, (kCells + 1) * 4) != cudaSuccess)
+    if (dalloc(c, c->cell_off, ((uint64_t)kCells10 + 1) * 4) != cudaSuccess)
         return set_error(c, RJ_ERR_OOM, "cell offsets allocation failed");
     {
         const unsigned cb = (unsigned)std::min<uint64_t>(blocks_for(n + 1, 256), (uint64_t)c->num_sms * 16);
@@ -286,14 +243,14 @@ rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int
         RJ_CUDA(c, cudaGetLastError());
     }
     uint32_t n_valid = 0;
-    RJ_CUDA(c, cudaMemcpyAsync(&n_valid, c->cell_off.as<uint32_t>() + kCells, 4, cudaMemcpyDeviceToHost, c->stream));
+    RJ_CUDA(c, cudaMemcpyAsync(&n_valid, c->cell_off.as<uint32_t>() + kCells10, 4, cudaMemcpyDeviceToHost, c->stream));
     RJ_CUDA(c, cudaStreamSynchronize(c->stream));
     c->n_pts = n_valid;
     if (n_ood) *n_ood = n - n_valid;
     for (int k = 0; k < P; ++k) dfree(c, A[k]);      // stream is idle here
     dfree(c, sx); dfree(c, sy);
     for (int k = 0; k < n_cols; ++k) dfree(c, scol[k]);
-    return build_items(c);
+    return RJ_OK;
 }
 
 }  // namespace rj

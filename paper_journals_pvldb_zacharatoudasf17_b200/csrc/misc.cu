@@ -70,9 +70,9 @@ __global__ void k_membership(const PassArgs a, uint64_t n, int accurate, const u
                 }
                 if (par && cur < 64) m |= 1ull << cur;
             } else {
-                const uint32_t cell = cell_of(qx, qy);
+                const uint32_t cell = cell_of(qx, qy, a.level);
                 const int64_t cc = cell_x(cell), cr = cell_y(cell);
-                const int64_t lx = px - cell_pix_lo(cc, a.W), ly = py - cell_pix_lo(cr, a.H);
+                const int64_t lx = px - cell_pix_lo(cc, a.W, a.level), ly = py - cell_pix_lo(cr, a.H, a.level);
                 for (uint32_t k = a.piece_off[cell]; k < a.piece_off[cell + 1]; ++k) {
                     const uint2 pc = a.pieces[k];
                     const int64_t lr = pc.y & 255u, lo = (pc.y >> 8) & 255u, hi = pc.y >> 16;

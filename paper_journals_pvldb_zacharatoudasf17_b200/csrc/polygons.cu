@@ -17,7 +17,7 @@
 //     inside polygon P are the spans [t1,t2), [t3,t4), ... (even-odd scanline
 //     rasterisation of the polygon = Proc. DrawPolygons' fragments, P:529-554,
 //     with the pixel-centre rule).
-//   * pieces: every span is cut at the pixel extents of the 256x256 point
+//   * pieces: every span is cut at the pixel extents of the level-L point
 //     cells it crosses and binned per cell; the fused point pass reduces each
 //     cell's tile over its pieces (S4).
 //   * S5 (accurate): supercover of every edge = the boundary pixels
@@ -131,10 +131,11 @@ __global__ void k_scatter_t(const uint32_t *__restrict__ cx_pr, const uint32_t *
 
 struct SpanGeo {
     int W, H;
+    int L;                      // point-cell level of the query
     const uint32_t *prow_off;   // [n_poly + 1]
     uint32_t n_poly;
     const int4 *mbr;
-    const uint32_t *cell_off;   // point cells: skip pieces of empty cells
+    const uint32_t *cell_off10; // point cells: skip pieces of empty cells
 };
 
 __device__ __forceinline__ void polyrow_of(const SpanGeo &g, uint32_t pr, uint32_t &P, int64_t &r) {
@@ -145,14 +146,15 @@ __device__ __forceinline__ void polyrow_of(const SpanGeo &g, uint32_t pr, uint32
 // Visit the (cell, local row, local lo, local hi) pieces of span [lo, hi) of row r.
 template <class F>
 __device__ __forceinline__ void for_each_piece(const SpanGeo &g, int64_t r, int64_t lo, int64_t hi, F f) {
-    const int64_t cr0 = qlo(r, g.H) >> kCellShift, cr1 = qhi(r, g.H) >> kCellShift;
-    const int64_t cc0 = qlo(lo, g.W) >> kCellShift, cc1 = qhi(hi - 1, g.W) >> kCellShift;
+    const int s = kLatticeBits - g.L, sh = 2 * (kMaxLevel - g.L);
+    const int64_t cr0 = qlo(r, g.H) >> s, cr1 = qhi(r, g.H) >> s;
+    const int64_t cc0 = qlo(lo, g.W) >> s, cc1 = qhi(hi - 1, g.W) >> s;
     for (int64_t cr = cr0; cr <= cr1; ++cr) {
-        const int64_t r0 = cell_pix_lo(cr, g.H);
+        const int64_t r0 = cell_pix_lo(cr, g.H, g.L);
         for (int64_t cc = cc0; cc <= cc1; ++cc) {
             const uint32_t cell = spread16((uint32_t)cc) | (spread16((uint32_t)cr) << 1);
-            if (g.cell_off[cell + 1] == g.cell_off[cell]) continue;     // no points in the cell
-            const int64_t c0 = cell_pix_lo(cc, g.W), c1 = cell_pix_hi(cc, g.W);
+            if (g.cell_off10[(uint64_t)(cell + 1) << sh] == g.cell_off10[(uint64_t)cell << sh]) continue;  // no points
+            const int64_t c0 = cell_pix_lo(cc, g.W, g.L), c1 = cell_pix_hi(cc, g.W, g.L);
             const int64_t a = max(lo, c0) - c0, b = min(hi, c1 + 1) - c0;
             f(cell, (uint32_t)(r - r0), (uint32_t)a, (uint32_t)b);
         }
@@ -347,7 +349,8 @@ rj_status load_polygons_impl(Ctx *c, uint32_t n_poly, const uint32_t *pro, const
 }
 
 // ------------------------------------------------------------ per-query pass
-rj_status polygon_pass(Ctx *c, int W, int H, bool accurate, PolyPass &pp) {
+rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp) {
+    const uint64_t ncell = 1ull << (2 * L);
     const uint32_t ne = c->n_edges, np = c->n_poly;
     cudaStream_t st = c->stream;
     Buf &erows = wsbuf(c, kWsEdgeRows), &eoff = wsbuf(c, kWsEdgeOff);
@@ -382,13 +385,13 @@ rj_status polygon_pass(Ctx *c, int W, int H, bool accurate, PolyPass &pp) {
     if (dreserve(c, cpr, (X + 1) * 4) || dreserve(c, ct, (X + 1) * 4) || dreserve(c, prc, (NPR + 1) * 4) ||
         dreserve(c, pro, (NPR + 1) * 4) || dreserve(c, prcur, (NPR + 1) * 4) || dreserve(c, tv, (X + 1) * 4) ||
         dreserve(c, scnt, (NPR + 1) * 4) || dreserve(c, soff, (NPR + 1) * 4) ||
-        dreserve(c, pcnt, (kCells + 1) * 4) || dreserve(c, poff, (kCells + 1) * 4) ||
-        dreserve(c, pcur, (kCells + 1) * 4))
+        dreserve(c, pcnt, (ncell + 1) * 4) || dreserve(c, poff, (ncell + 1) * 4) ||
+        dreserve(c, pcur, (ncell + 1) * 4))
         return set_error(c, RJ_ERR_OOM, "workspace allocation failed");
     RJ_CUDA(c, cudaMemsetAsync(prc.p, 0, (NPR + 1) * 4, st));
     RJ_CUDA(c, cudaMemsetAsync(prcur.p, 0, (NPR + 1) * 4, st));
-    RJ_CUDA(c, cudaMemsetAsync(pcnt.p, 0, (kCells + 1) * 4, st));
-    RJ_CUDA(c, cudaMemsetAsync(pcur.p, 0, (kCells + 1) * 4, st));
+    RJ_CUDA(c, cudaMemsetAsync(pcnt.p, 0, (ncell + 1) * 4, st));
+    RJ_CUDA(c, cudaMemsetAsync(pcur.p, 0, (ncell + 1) * 4, st));
     const unsigned gx = (unsigned)std::min<uint64_t>(std::max<uint64_t>(1, blocks_for(X, 256)), c->num_sms * 8ull);
     k_crossings<<<gx, 256, 0, st>>>(c->edges.as<int4>(), c->edge_poly.as<uint32_t>(), c->mbr.as<int4>(),
                                     eoff.as<uint32_t>(), ne, proff.as<uint32_t>(), W, H, cpr.as<uint32_t>(),
@@ -399,17 +402,17 @@ rj_status polygon_pass(Ctx *c, int W, int H, bool accurate, PolyPass &pp) {
     k_scatter_t<<<gx, 256, 0, st>>>(cpr.as<uint32_t>(), ct.as<uint32_t>(), X, pro.as<uint32_t>(),
                                     prcur.as<uint32_t>(), tv.as<uint32_t>());
     RJ_LAUNCHED(c);
-    SpanGeo g{W, H, proff.as<uint32_t>(), np, c->mbr.as<int4>(), c->cell_off.as<uint32_t>()};
+    SpanGeo g{W, H, L, proff.as<uint32_t>(), np, c->mbr.as<int4>(), c->cell_off.as<uint32_t>()};
     const unsigned gp = (unsigned)std::min<uint64_t>(std::max<uint64_t>(1, blocks_for(NPR, 128)), c->num_sms * 16ull);
     k_prow_count<<<gp, 128, 0, st>>>(g, NPR, pro.as<uint32_t>(), tv.as<uint32_t>(), scnt.as<uint32_t>(),
                                      pcnt.as<uint32_t>());
     RJ_LAUNCHED(c);
     RJ_CUDA(c, cudaGetLastError());
     RJ_CUDA(c, scan_u32(c, scnt.as<uint32_t>(), soff.as<uint32_t>(), NPR, kWsScan));
-    RJ_CUDA(c, scan_u32(c, pcnt.as<uint32_t>(), poff.as<uint32_t>(), kCells, kWsScan));
+    RJ_CUDA(c, scan_u32(c, pcnt.as<uint32_t>(), poff.as<uint32_t>(), ncell, kWsScan));
     // sync 2: span / piece totals
     RJ_CUDA(c, cudaMemcpyAsync(hs + 3, soff.as<uint32_t>() + NPR, 4, cudaMemcpyDeviceToHost, st));
-    RJ_CUDA(c, cudaMemcpyAsync(hs + 4, poff.as<uint32_t>() + kCells, 4, cudaMemcpyDeviceToHost, st));
+    RJ_CUDA(c, cudaMemcpyAsync(hs + 4, poff.as<uint32_t>() + ncell, 4, cudaMemcpyDeviceToHost, st));
     RJ_CUDA(c, cudaStreamSynchronize(st));
     const uint32_t S = hs[3], NP = hs[4];
     Buf &spans = wsbuf(c, kWsSpans), &pieces = wsbuf(c, kWsPieces);

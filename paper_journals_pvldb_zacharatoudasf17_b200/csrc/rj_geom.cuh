@@ -21,9 +21,8 @@ namespace rj {
 constexpr int kLatticeBits = 30;
 constexpr int64_t kOne = int64_t(1) << kLatticeBits;      // 2^30
 constexpr int64_t kHalf = int64_t(1) << (kLatticeBits - 1);
-constexpr int kCellBits = 8;                               // point tiles: 256 x 256 cells
-constexpr int kCells = 1 << (2 * kCellBits);               // 65536
-constexpr int kCellShift = kLatticeBits - kCellBits;       // 22
+constexpr int kMaxLevel = 10;                              // finest point-cell level: 1024 x 1024
+constexpr int kCells10 = 1 << (2 * kMaxLevel);             // cells at the finest level
 constexpr int kGridBits = 10;                              // edge grid: 1024 x 1024
 constexpr int kGrid = 1 << kGridBits;
 constexpr int kGridShift = kLatticeBits - kGridBits;       // 20
@@ -85,16 +84,18 @@ RJ_HD uint32_t compact16(uint32_t v) {
 RJ_HD uint32_t morton_key(uint32_t qx, uint32_t qy) {
     return spread16(qx >> kMortonShift) | (spread16(qy >> kMortonShift) << 1);
 }
-// cell id (Morton order of the 256x256 cell grid) = top 16 bits of the key
-RJ_HD uint32_t cell_of(uint32_t qx, uint32_t qy) {
-    return spread16(qx >> kCellShift) | (spread16(qy >> kCellShift) << 1);
+// Point cells: the lattice is cut into 2^L x 2^L cells numbered in Morton
+// order; because the points are sorted by the Morton key, every cell of
+// every level L <= 10 is a contiguous range of the sorted points.
+RJ_HD uint32_t cell_of(uint32_t qx, uint32_t qy, int L) {
+    return spread16(qx >> (kLatticeBits - L)) | (spread16(qy >> (kLatticeBits - L)) << 1);
 }
 RJ_HD uint32_t cell_x(uint32_t c) { return compact16(c); }
 RJ_HD uint32_t cell_y(uint32_t c) { return compact16(c >> 1); }
 
-// Pixel range [lo, hi] (inclusive) covered by cell column/row cc of a
-// canvas side of n pixels: the pixels whose lattice extent meets the cell.
-RJ_HD int64_t cell_pix_lo(int64_t cc, int64_t n) { return pix(cc << kCellShift, n); }
-RJ_HD int64_t cell_pix_hi(int64_t cc, int64_t n) { return pix(((cc + 1) << kCellShift) - 1, n); }
+// Pixel range [lo, hi] (inclusive) covered by cell column/row cc (level L)
+// of a canvas side of n pixels: the pixels whose lattice extent meets the cell.
+RJ_HD int64_t cell_pix_lo(int64_t cc, int64_t n, int L) { return pix(cc << (kLatticeBits - L), n); }
+RJ_HD int64_t cell_pix_hi(int64_t cc, int64_t n, int L) { return pix(((cc + 1) << (kLatticeBits - L)) - 1, n); }
 
 }  // namespace rj

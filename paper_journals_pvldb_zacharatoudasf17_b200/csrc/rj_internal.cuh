@@ -35,6 +35,7 @@ struct Filter {
     float f_val[5];
     int32_t never = 0;            // an int predicate can never hold
     int32_t agg_slot = -1;        // slot of the summed attribute (SUM/AVG)
+    int32_t agg_is_float = 0;     // its dtype (avoids a dynamically indexed param)
 };
 
 // Device-side parameter block of the fused point pass.
@@ -43,10 +44,13 @@ struct PassArgs {
     const uint32_t *col[6];
     Filter f;
     int32_t W, H;
-    const int4 *items;
+    const int4 *items;            // (cell_begin, cell_end, point_begin, point_end)
     uint32_t n_items;
     uint32_t *work_counter;
-    const uint32_t *piece_off;    // [kCells + 1]
+    int32_t level;                // point-cell level L of this query (2^L x 2^L cells)
+    const uint32_t *cell_off10;   // [kCells10 + 1] first point of every level-10 cell
+    uint32_t tile_stride;         // row stride of a warp's tile (odd: conflict-free row prefix)
+    const uint32_t *piece_off;    // [4^L + 1]
     const uint2 *pieces;
     const uint32_t *mask;         // accurate: boundary bitmask
     uint32_t mask_wpr;
@@ -58,7 +62,8 @@ struct PassArgs {
     double *A_sum;
     uint32_t n_poly;
     int32_t smem_partials;        // accumulate per-CTA polygon partials in smem
-    uint32_t tile_cap;            // pixels of the largest tile
+    uint32_t tile_cap;            // words of the CTA's tile
+    uint32_t n_stages;            // depth of the shared-memory stage ring
     unsigned long long *stats;    // [0] filtered, [1] boundary
 };
 
@@ -74,17 +79,18 @@ struct Ctx {
     void *alloc_user = nullptr;
     int num_sms = 148;
     int timing = 0;
-    int64_t chunk = 32768;
+    int64_t chunk = 16384;
 
     // points (S1 output, spatially sorted)
     uint64_t n_in = 0, n_pts = 0;
     int n_cols = 0;
     int col_dtype[RJ_MAX_COLS];
     Buf qx, qy, idx, col[RJ_MAX_COLS];
-    Buf cell_off;                 // [kCells + 1]
-    Buf items;                    // int4 (cell, begin, end, 0)
-    uint32_t n_items = 0;
-    int64_t items_chunk = 0;
+    Buf cell_off;                 // [kCells10 + 1]
+    std::vector<uint32_t> h_cell_off;          // host copy (work-item planning)
+    Buf items[kMaxLevel + 1];                  // per level L: int4 work items
+    uint32_t n_items[kMaxLevel + 1] = {};
+    int64_t items_chunk[kMaxLevel + 1] = {};
 
     // polygons
     uint32_t n_poly = 0;
@@ -127,7 +133,10 @@ cudaError_t scan_u32(Ctx *c, const uint32_t *in, uint32_t *out, uint64_t n, int 
 rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int xy_f64,
                            int n_cols, const void *const *cols, const int32_t *dtypes,
                            uint64_t *n_ood);
-rj_status build_items(Ctx *c);
+// work.cu: point-pass work items for level L (cached per level)
+rj_status items_for_level(Ctx *c, int L);
+void drop_items(Ctx *c);
+int choose_level(int W, int H, bool sum);
 
 // polygons.cu
 rj_status load_polygons_impl(Ctx *c, uint32_t n_poly, const uint32_t *pro, const uint32_t *rvo,
@@ -135,16 +144,17 @@ rj_status load_polygons_impl(Ctx *c, uint32_t n_poly, const uint32_t *pro, const
 struct PolyPass {
     uint64_t n_cross = 0, n_spans = 0, n_pieces = 0;
     uint32_t *spans = nullptr;       // 4 x u32 per span (poly,row,lo,hi), (poly,row,lo)-sorted
-    uint32_t *piece_off = nullptr;   // [kCells + 1]
+    uint32_t *piece_off = nullptr;   // [4^L + 1]
     uint2 *pieces = nullptr;
     uint32_t *mask = nullptr;        // accurate only
     uint32_t mask_wpr = 0;
 };
-rj_status polygon_pass(Ctx *c, int W, int H, bool accurate, PolyPass &pp);
+rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp);
 
 // pass.cu
 rj_status point_pass(Ctx *c, const PassArgs &a, bool sum, bool accurate);
 size_t point_pass_smem(const PassArgs &a, bool sum, bool accurate);
+int point_pass_stages(int n_slots);
 
 // misc.cu
 cudaError_t launch_finalize(Ctx *c, int agg, uint32_t n, const unsigned long long *cnt,

@@ -264,6 +264,7 @@ static rj_status run_pass(Ctx *c, Prepared &P, unsigned long long *d_cnt, double
     L.n_spans = P.pp.n_spans;
     L.n_pieces = P.pp.n_pieces;
     L.n_items = c->n_items[P.L];
+    L.level = P.L;
     L.stream_bytes = c->n_pts * (8ull + 4ull * (uint64_t)a.f.n_slots);
     return RJ_OK;
 }
@@ -451,6 +452,8 @@ rj_status rj_get_stats(const rj_ctx *cc, rj_stats *out) {
     c->last.n_filtered = c->h_stats[0];
     c->last.n_boundary = c->h_stats[1];
     c->last.launches = c->launches;
+    c->last.pass_stages = c->last_stages;
+    c->last.pass_ctas_per_sm = c->last_ctas_per_sm;
     if (c->timing) {
         float a = 0, b = 0, t = 0;
         cudaEventElapsedTime(&a, c->ev[0], c->ev[1]);

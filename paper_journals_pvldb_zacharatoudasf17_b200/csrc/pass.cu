@@ -39,7 +39,7 @@ constexpr int kThreads = 256;
 constexpr int kWarps = kThreads / 32;
 constexpr int kIPL = 8;                      // points per lane per window (256-bit loads)
 constexpr int kWin = 32 * kIPL;              // 256 points per warp window
-constexpr int kQ = 32 + kWin;                // per-warp boundary queue capacity
+constexpr int kQ = 64;                       // per-warp boundary queue capacity (drained at >= 32)
 constexpr uint32_t kNoKey = 0xFFFFFFFFu;
 constexpr unsigned kFull = 0xFFFFFFFFu;
 constexpr uint32_t kFlag = 0x80000000u;
@@ -281,8 +281,10 @@ __device__ __forceinline__ void process(const PassArgs &a, const Shared &sh, con
         }
         if (__any_sync(kFull, bm != 0u)) {
 #pragma unroll
-            for (int j = 0; j < kIPL; ++j) enqueue<SUM, NS>(a, sh, w, j, (bm >> j) & 1u, qn, n_bnd);
-            drain_queue<SUM>(a, sh, qn, false);
+            for (int j = 0; j < kIPL; ++j) {
+                enqueue<SUM, NS>(a, sh, w, j, (bm >> j) & 1u, qn, n_bnd);   // adds <= 32
+                drain_queue<SUM>(a, sh, qn, false);                          // leaves < 32
+            }
 #pragma unroll
             for (int j = 0; j < kIPL; ++j) ok[j] = ok[j] && !((bm >> j) & 1u);
         }
@@ -489,7 +491,8 @@ __global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass(const PassArgs 
         const bool never = a.f.never != 0;
         Tile t;
         t.stride = a.tile_stride;
-        uint32_t tbase = 0, c0 = 0, r0 = 0, tsel = 0;
+        uint32_t tbase = 0, c0 = 0, r0 = 0, tsel = 0, pb = 0, pe = 0;
+        uint2 pc0 = make_uint2(0u, 0u);
         uint32_t n_pass = 0, n_bnd = 0, qn = 0;
         uint32_t st = 0, ph = 0;
         for (;;) {
@@ -502,6 +505,8 @@ __global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass(const PassArgs 
                 t.cnt = tcnt + tsel * a.tile_cap;
                 t.sum = tsum + tsel * a.tile_cap;
                 tsel ^= 1u;
+                pb = __ldg(&a.piece_off[m.cell]);          // consumed at the cell's last stage
+                pe = __ldg(&a.piece_off[m.cell + 1]);
                 const int64_t cx = cell_x(m.cell), cy = cell_y(m.cell);
                 c0 = (uint32_t)pix(cx << s_lat, a.W);
                 r0 = (uint32_t)pix(cy << s_lat, a.H);
@@ -525,6 +530,7 @@ __global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass(const PassArgs 
                 }
                 consumers_sync();
             }
+            if ((m.flags & 2u) && pb + threadIdx.x < pe) pc0 = __ldg(&a.pieces[pb + threadIdx.x]);  // in flight
             // ---- this warp's window of the stage
             const uint32_t woff = (uint32_t)wid * kWin;                 // window offset in the stage
             const uint32_t ncopy = ((m.se + 3u) & ~3u) - m.cb;
@@ -540,42 +546,24 @@ __global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass(const PassArgs 
             if (lane == 0) mbar_arrive((uint32_t)__cvta_generic_to_shared(&s_empty[st]));
             if (m.flags & 2u) {                           // last stage of the cell: reduce the tile
                 if (ACC) drain_queue<SUM>(a, sh, qn, true);
-                consumers_sync();
-                for (uint32_t r = threadIdx.x; r < t.th; r += kThreads) {
-                    uint32_t *rc = t.cnt + r * t.stride;
-                    double *rs = t.sum + r * t.stride;
-                    if (t.tw <= kMaxTileW) {
-                        uint32_t v[kMaxTileW];
-#pragma unroll
-                        for (int i = 0; i < kMaxTileW; ++i) v[i] = i < (int)t.tw ? rc[i] : 0u;
-                        uint32_t acc = 0;
-#pragma unroll
-                        for (int i = 0; i < kMaxTileW; ++i) {
-                            acc += ACC ? (v[i] & ~kFlag) : v[i];   // boundary pixels hold only the flag
-                            if (i < (int)t.tw) rc[i] = acc;
-                        }
-                    } else {
-                        uint32_t acc = 0;
-                        for (uint32_t i = 0; i < t.tw; ++i) {
-                            acc += ACC ? (rc[i] & ~kFlag) : rc[i];
-                            rc[i] = acc;
-                        }
-                    }
-                    if (SUM) {
-                        double dacc = 0.0;
-                        for (uint32_t i = 0; i < t.tw; ++i) { dacc += rs[i]; rs[i] = dacc; }
-                    }
-                }
-                consumers_sync();
-                const uint32_t pb = __ldg(&a.piece_off[m.cell]), pe = __ldg(&a.piece_off[m.cell + 1]);
+                consumers_sync();                          // every point of the cell is in the tile
+                // span pieces (S4): each thread sums its pieces' pixels straight
+                // from the tile (<= 33 words each), no separate prefix phase
                 for (uint32_t kk = pb + threadIdx.x; kk < pe; kk += kThreads) {
-                    const uint2 pc = __ldg(&a.pieces[kk]);
+                    const uint2 pc = (kk == pb + threadIdx.x) ? pc0 : __ldg(&a.pieces[kk]);
                     const uint32_t lr = pc.y & 255u, lo = (pc.y >> 8) & 255u, hi = pc.y >> 16;
-                    const uint32_t rb = lr * t.stride;
-                    const uint32_t cnt = t.cnt[rb + hi - 1] - (lo ? t.cnt[rb + lo - 1] : 0u);
+                    const uint32_t *rc = t.cnt + lr * t.stride;
+                    uint32_t cnt = 0;
+                    for (uint32_t i = lo; i < hi; ++i) cnt += rc[i];
+                    // boundary pixels hold only kFlag (2^31): their sum only
+                    // touches bit 31, and a piece's count is < 2^31
+                    if (ACC) cnt &= ~kFlag;
                     if (cnt) {
                         double sm = 0.0;
-                        if (SUM) sm = t.sum[rb + hi - 1] - (lo ? t.sum[rb + lo - 1] : 0.0);
+                        if (SUM) {
+                            const double *rs = t.sum + lr * t.stride;
+                            for (uint32_t i = lo; i < hi; ++i) sm += rs[i];
+                        }
                         emit_poly<SUM>(a, sh, pc.x, cnt, sm);
                     }
                 }
@@ -637,13 +625,25 @@ size_t point_pass_smem(const PassArgs &a, bool sum, bool accurate) {
     return b;
 }
 
-int point_pass_stages(int n_slots) {
-    // ring depth: 3 stages when the columns are narrow, 2 when wide
-    return (2 + n_slots) <= 4 ? 3 : 2;
-}
+int point_pass_stages(int n_slots) { return (2 + n_slots) <= 4 ? 3 : 2; }
 
-rj_status point_pass(Ctx *c, const PassArgs &a, bool sum, bool accurate) {
-    void *k = select_kernel(sum, accurate, a.f.n_slots, a.f.n_fpred > 0);
+rj_status point_pass(Ctx *c, const PassArgs &a_in, bool sum, bool accurate) {
+    void *k = select_kernel(sum, accurate, a_in.f.n_slots, a_in.f.n_fpred > 0);
+    // ring depth: the deepest ring that keeps two CTAs (16 consumer warps) per
+    // SM, else the deepest that fits one CTA
+    PassArgs a = a_in;
+    const size_t budget = 227 * 1024 - 1024;
+    int best = 0, best_score = -1;
+    for (int st = 2; st <= kMaxStages; ++st) {
+        a.n_stages = st;
+        const size_t need = point_pass_smem(a, sum, accurate) + 2048;
+        const int ctas = (int)std::min<size_t>(2, (228 * 1024) / (need + 1024));
+        if (need > budget || ctas < 1) continue;
+        const int score = ctas * 8 + st;
+        if (score > best_score) { best_score = score; best = st; }
+    }
+    if (!best) return set_error(c, RJ_ERR_RESOLUTION, "point-pass tiles do not fit in shared memory");
+    a.n_stages = best;
     const size_t smem = point_pass_smem(a, sum, accurate);
     RJ_CUDA(c, cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
     int per_sm = 0;
@@ -653,6 +653,8 @@ rj_status point_pass(Ctx *c, const PassArgs &a, bool sum, bool accurate) {
         1, std::min<uint64_t>((uint64_t)per_sm * c->num_sms, std::max<uint32_t>(1, a.n_items)));
     void *args[] = {(void *)&a};
     RJ_CUDA(c, cudaLaunchKernel(k, dim3(grid), dim3(kThreads + 32), args, smem, c->stream));
+    c->last_stages = best;
+    c->last_ctas_per_sm = per_sm;
     RJ_LAUNCHED(c);
     return RJ_OK;
 }

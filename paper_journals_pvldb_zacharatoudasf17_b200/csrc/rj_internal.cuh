@@ -79,7 +79,7 @@ struct Ctx {
     void *alloc_user = nullptr;
     int num_sms = 148;
     int timing = 0;
-    int64_t chunk = 16384;
+    int64_t chunk = 65536;
 
     // points (S1 output, spatially sorted)
     uint64_t n_in = 0, n_pts = 0;
@@ -107,6 +107,7 @@ struct Ctx {
     rj_stats last{};
     cudaEvent_t ev[6] = {};
     uint32_t launches = 0;
+    int last_stages = 0, last_ctas_per_sm = 0;   // point-pass launch shape of the last query
 };
 
 // workspace slot map (Ctx::ws)

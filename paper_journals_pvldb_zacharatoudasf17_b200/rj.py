@@ -54,7 +54,8 @@ class rj_stats(ctypes.Structure):
                 ("n_filtered", ctypes.c_uint64), ("n_boundary", ctypes.c_uint64),
                 ("n_crossings", ctypes.c_uint64), ("n_spans", ctypes.c_uint64), ("n_pieces", ctypes.c_uint64),
                 ("n_items", ctypes.c_uint64), ("stream_bytes", ctypes.c_uint64), ("launches", ctypes.c_uint32),
-                ("ms_polygon", ctypes.c_float), ("ms_point_pass", ctypes.c_float), ("ms_total", ctypes.c_float)]
+                ("ms_polygon", ctypes.c_float), ("ms_point_pass", ctypes.c_float), ("ms_total", ctypes.c_float),
+                ("pass_stages", ctypes.c_int32), ("pass_ctas_per_sm", ctypes.c_int32), ("level", ctypes.c_int32)]
 
     def as_dict(self):
         return {k: getattr(self, k) for k, _ in self._fields_}

@@ -62,6 +62,16 @@ cudaError_t dreserve(Ctx *c, Buf &b, size_t bytes) {
     return dalloc(c, b, std::max<size_t>(bytes + bytes / 4, 256));
 }
 
+cudaError_t dreserve_exact(Ctx *c, Buf &b, size_t bytes) {
+    if (b.p && b.bytes >= bytes) return cudaSuccess;
+    if (b.p) {
+        cudaError_t e = cudaStreamSynchronize(c->stream);
+        if (e != cudaSuccess) return e;
+        dfree(c, b);
+    }
+    return dalloc(c, b, bytes);
+}
+
 Buf &wsbuf(Ctx *c, int slot) { return c->ws[slot]; }
 
 // S0: canvas resolution from the descriptor (reading Z3: W = ceil(w*sqrt(2)/eps)).
@@ -346,6 +356,7 @@ rj_status rj_destroy(rj_ctx *c) {
     cudaStreamSynchronize(c->stream);
     dfree(c, c->qx); dfree(c, c->qy); dfree(c, c->idx);
     for (auto &b : c->col) dfree(c, b);
+    free_load_scratch(c);
     dfree(c, c->cell_off); drop_items(c);
     dfree(c, c->edges); dfree(c, c->edge_poly); dfree(c, c->poly_edge_off); dfree(c, c->mbr);
     dfree(c, c->grid_off); dfree(c, c->grid_ent);
@@ -370,6 +381,16 @@ rj_status rj_set_allocator(rj_ctx *c, void *(*alloc_fn)(size_t, void *), void (*
 rj_status rj_set_option(rj_ctx *c, int32_t option, int64_t value) {
     if (!c) return RJ_ERR_INVALID_ARGUMENT;
     if (option == RJ_OPT_TIMING) { c->timing = value ? 1 : 0; return RJ_OK; }
+    if (option == RJ_OPT_PASS) {
+        if (value < 0 || value > 1) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "RJ_OPT_PASS must be 0 or 1");
+        c->force_tile_pass = (int)value;
+        return RJ_OK;
+    }
+    if (option == RJ_OPT_KEEP_LOAD_SCRATCH) {
+        c->keep_load_scratch = value ? 1 : 0;
+        if (!value) free_load_scratch(c);
+        return RJ_OK;
+    }
     if (option == RJ_OPT_CHUNK) {
         if (value < 256 || value > (1ll << 30)) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "chunk must be in [256, 2^30]");
         c->chunk = value;

@@ -73,14 +73,22 @@ __global__ void __launch_bounds__(kSortThreads) k_radix_hist(const uint32_t *__r
         counts[(uint64_t)d * ntiles + blockIdx.x] = hist[d];
 }
 
-// Stable scatter: warp w owns the 512 consecutive items [w*512, w*512+512)
-// of the tile, ranked round by round (32 items per round, in order).
+// Stable scatter, staged through shared memory so that global writes are
+// coalesced runs per digit: items are first ranked stably inside the tile
+// (warp w owns items [w*512, w*512+512), ranked round by round), placed in
+// tile-sorted order in shared memory, then written out sequentially -- item
+// i of the sorted tile goes to goff[d] + (i - toff[d]).
 __global__ void __launch_bounds__(kSortThreads) k_radix_scatter(Payload pl, uint64_t n, int shift,
                                                                 const uint32_t *__restrict__ offs,
                                                                 uint32_t ntiles) {
     __shared__ uint32_t wcount[kSortThreads / 32][kDigits];
+    __shared__ uint32_t toff[kDigits + 1], goff[kDigits];
+    __shared__ uint32_t wsum[kSortThreads / 32];
+    __shared__ uint16_t sdig[kSortTile];
+    __shared__ uint32_t buf[kSortTile];
     const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
-    const uint64_t seg = (uint64_t)blockIdx.x * kSortTile + (uint64_t)w * 32 * kSortItems;
+    const uint64_t tile0 = (uint64_t)blockIdx.x * kSortTile;
+    const uint64_t seg = tile0 + (uint64_t)w * 32 * kSortItems;
     for (int d = lane; d < kDigits; d += 32) wcount[w][d] = 0;
     __syncwarp();
     uint32_t dig[kSortItems], peers[kSortItems];
@@ -93,8 +101,33 @@ __global__ void __launch_bounds__(kSortThreads) k_radix_scatter(Payload pl, uint
         __syncwarp();
     }
     __syncthreads();
-    for (int d = threadIdx.x; d < kDigits; d += kSortThreads) {
-        uint32_t run = offs[(uint64_t)d * ntiles + blockIdx.x];
+    // tile-local digit offsets: toff = exclusive scan of the tile's digit counts
+    const int d0 = threadIdx.x;                 // thread t owns digit t (thread 0 also digit 256)
+    // block exclusive scan of `tot` in digit order (thread t holds digit t; thread 0 also 256)
+    uint32_t mine = 0;
+    for (int ww = 0; ww < kSortThreads / 32; ++ww) mine += (d0 < kDigits) ? wcount[ww][d0] : 0u;
+    uint32_t incl = mine;
+#pragma unroll
+    for (int dd = 1; dd < 32; dd <<= 1) {
+        const uint32_t o = __shfl_up_sync(0xffffffffu, incl, dd);
+        if (lane >= dd) incl += o;
+    }
+    if (lane == 31) wsum[w] = incl;
+    __syncthreads();
+    uint32_t wpre = 0;
+    for (int ww = 0; ww < w; ++ww) wpre += wsum[ww];
+    toff[d0] = wpre + incl - mine;
+    if (d0 == kSortThreads - 1) {
+        uint32_t c256 = 0;
+        for (int ww = 0; ww < kSortThreads / 32; ++ww) c256 += wcount[ww][256];
+        toff[256] = wpre + incl;
+        toff[257] = wpre + incl + c256;
+    }
+    for (int d = d0; d < kDigits; d += kSortThreads) goff[d] = offs[(uint64_t)d * ntiles + blockIdx.x];
+    __syncthreads();
+    // per (warp, digit) running tile positions
+    for (int d = d0; d < kDigits; d += kSortThreads) {
+        uint32_t run = toff[d];
 #pragma unroll
         for (int ww = 0; ww < kSortThreads / 32; ++ww) {
             const uint32_t t = wcount[ww][d];
@@ -104,20 +137,31 @@ __global__ void __launch_bounds__(kSortThreads) k_radix_scatter(Payload pl, uint
     }
     __syncthreads();
     const unsigned lt = (1u << lane) - 1u;
+    uint32_t lpos[kSortItems];
 #pragma unroll
     for (int j = 0; j < kSortItems; ++j) {
-        const uint64_t i = seg + j * 32 + lane;
         const uint32_t d = dig[j];
-        uint32_t pos = 0;
+        uint32_t pos = 0xFFFFFFFFu;
         if (d < kDigits) pos = wcount[w][d] + __popc(peers[j] & lt);
         __syncwarp();
         if (d < kDigits && lane == __ffs(peers[j]) - 1) wcount[w][d] += __popc(peers[j]);
         __syncwarp();
-        if (d < kDigits) {
-            for (int k = 0; k < pl.n; ++k) {
-                const uint32_t v = pl.src[k] ? pl.src[k][i] : (uint32_t)i;
-                pl.dst[k][pos] = v;
-            }
+        lpos[j] = pos;
+        if (d < kDigits) sdig[pos] = (uint16_t)d;
+    }
+    const uint32_t tile_n = (uint32_t)((n - tile0) < (uint64_t)kSortTile ? (n - tile0) : (uint64_t)kSortTile);
+    for (int k = 0; k < pl.n; ++k) {
+        __syncthreads();                        // buf free (previous column written out)
+#pragma unroll
+        for (int j = 0; j < kSortItems; ++j) {
+            const uint64_t i = seg + j * 32 + lane;
+            if (lpos[j] != 0xFFFFFFFFu) buf[lpos[j]] = pl.src[k] ? pl.src[k][i] : (uint32_t)i;
+        }
+        __syncthreads();
+        uint32_t *dst = pl.dst[k];
+        for (uint32_t i = threadIdx.x; i < tile_n; i += kSortThreads) {
+            const uint32_t d = sdig[i];
+            dst[goff[d] + (i - toff[d])] = buf[i];
         }
     }
 }
@@ -148,54 +192,65 @@ bool is_device_ptr(const void *p) {
 }  // namespace
 
 // Stage a column on the device (copy if host memory). Returns the device pointer.
+// Stage a column on the device (copy if host memory) into a grow-only
+// context buffer. Returns the device pointer.
 static rj_status stage(Ctx *c, const void *p, size_t bytes, Buf &tmp, const void **out) {
     if (is_device_ptr(p)) {
         *out = p;
         return RJ_OK;
     }
-    if (dalloc(c, tmp, bytes) != cudaSuccess) return set_error(c, RJ_ERR_OOM, "staging allocation failed");
+    if (dreserve_exact(c, tmp, bytes) != cudaSuccess) return set_error(c, RJ_ERR_OOM, "staging allocation failed");
     RJ_CUDA(c, cudaMemcpyAsync(tmp.p, p, bytes, cudaMemcpyHostToDevice, c->stream));
     *out = tmp.p;
     return RJ_OK;
 }
 
+// Release the load-time scratch (staging and the sort's second buffer).
+void free_load_scratch(Ctx *c) {
+    for (auto &b : c->load_stage) dfree(c, b);
+    for (auto &b : c->load_alt) dfree(c, b);
+}
+
 rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int xy_f64, int n_cols,
                            const void *const *cols, const int32_t *dtypes, uint64_t *n_ood) {
-    // drop the previous point set
-    dfree(c, c->qx); dfree(c, c->qy); dfree(c, c->idx);
-    for (int k = 0; k < RJ_MAX_COLS; ++k) dfree(c, c->col[k]);
+    // the previous point set's columns are reused as the sort's output buffers
+    // (grow-only), so reloading same-sized data allocates nothing
     dfree(c, c->cell_off);
     drop_items(c);
     c->n_in = c->n_pts = 0; c->n_cols = 0;
 
     const size_t esz = xy_f64 ? 8 : 4;
-    Buf sx, sy, scol[RJ_MAX_COLS];
     const void *dx = nullptr, *dy = nullptr, *dcol[RJ_MAX_COLS] = {};
     const uint64_t nn = std::max<uint64_t>(n, 1);
     rj_status s;
     if (n) {
-        if ((s = stage(c, x, n * esz, sx, &dx)) != RJ_OK) return s;
-        if ((s = stage(c, y, n * esz, sy, &dy)) != RJ_OK) return s;
+        if ((s = stage(c, x, n * esz, c->load_stage[0], &dx)) != RJ_OK) return s;
+        if ((s = stage(c, y, n * esz, c->load_stage[1], &dy)) != RJ_OK) return s;
         for (int k = 0; k < n_cols; ++k)
-            if ((s = stage(c, cols[k], n * 4, scol[k], &dcol[k])) != RJ_OK) return s;
+            if ((s = stage(c, cols[k], n * 4, c->load_stage[2 + k], &dcol[k])) != RJ_OK) return s;
     }
     const int P = 3 + n_cols;
-    Buf A[kMaxPayload], B[kMaxPayload];
-    for (int k = 0; k < P; ++k)
+    Buf *B[kMaxPayload] = {&c->qx, &c->qy, &c->idx};
+    for (int k = 0; k < n_cols; ++k) B[3 + k] = &c->col[k];
+    for (int k = n_cols; k < RJ_MAX_COLS; ++k) dfree(c, c->col[k]);
+    Buf *A[kMaxPayload];
+    for (int k = 0; k < P; ++k) {
+        A[k] = &c->load_alt[k];
         // +8 points of padding: the point pass copies 16-B aligned supersets of ranges
-        if (dalloc(c, A[k], (nn + 8) * 4) != cudaSuccess || dalloc(c, B[k], (nn + 8) * 4) != cudaSuccess)
+        if (dreserve_exact(c, *A[k], (nn + 8) * 4) != cudaSuccess || dreserve_exact(c, *B[k], (nn + 8) * 4) != cudaSuccess)
             return set_error(c, RJ_ERR_OOM, "point buffers allocation failed");
+    }
 
     if (n) {
         const unsigned qb = (unsigned)std::min<uint64_t>(blocks_for(n, 256), (uint64_t)c->num_sms * 16);
         if (xy_f64)
             k_quantize<double><<<qb, 256, 0, c->stream>>>((const double *)dx, (const double *)dy, n, c->x0,
                                                           c->x1 - c->x0, c->y0, c->y1 - c->y0,
-                                                          B[0].as<uint32_t>(), B[1].as<uint32_t>());
+                                                          B[0]->as<uint32_t>(), B[1]->as<uint32_t>());
         else
             k_quantize<float><<<qb, 256, 0, c->stream>>>((const float *)dx, (const float *)dy, n, c->x0,
                                                          c->x1 - c->x0, c->y0, c->y1 - c->y0,
-                                                         B[0].as<uint32_t>(), B[1].as<uint32_t>());
+                                                         B[0]->as<uint32_t>(), B[1]->as<uint32_t>());
         RJ_LAUNCHED(c);
         RJ_CUDA(c, cudaGetLastError());
 
@@ -208,14 +263,14 @@ rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int
         for (int pass = 0; pass < 4; ++pass) {
             Payload pl;
             pl.n = P;
-            Buf *from = (pass % 2 == 0) ? B : A;
-            Buf *to = (pass % 2 == 0) ? A : B;
+            Buf **from = (pass % 2 == 0) ? B : A;
+            Buf **to = (pass % 2 == 0) ? A : B;
             for (int k = 0; k < P; ++k) {
                 if (pass == 0)
-                    pl.src[k] = k < 2 ? from[k].as<uint32_t>() : (k == 2 ? nullptr : (const uint32_t *)dcol[k - 3]);
+                    pl.src[k] = k < 2 ? from[k]->as<uint32_t>() : (k == 2 ? nullptr : (const uint32_t *)dcol[k - 3]);
                 else
-                    pl.src[k] = from[k].as<uint32_t>();
-                pl.dst[k] = to[k].as<uint32_t>();
+                    pl.src[k] = from[k]->as<uint32_t>();
+                pl.dst[k] = to[k]->as<uint32_t>();
             }
             k_radix_hist<<<ntiles, kSortThreads, 0, c->stream>>>(pl.src[0], pl.src[1], n, 8 * pass,
                                                                  counts.as<uint32_t>(), ntiles);
@@ -226,10 +281,9 @@ rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int
             RJ_LAUNCHED(c);
             RJ_CUDA(c, cudaGetLastError());
         }
-        // after 4 passes the sorted payload is in B
+        // after 4 passes the sorted payload is in B (the context's columns)
     }
-    c->qx = B[0]; c->qy = B[1]; c->idx = B[2];
-    for (int k = 0; k < n_cols; ++k) { c->col[k] = B[3 + k]; c->col_dtype[k] = dtypes[k]; }
+    for (int k = 0; k < n_cols; ++k) c->col_dtype[k] = dtypes[k];
     c->n_cols = n_cols;
     c->n_in = n;
 
@@ -247,9 +301,7 @@ rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int
     RJ_CUDA(c, cudaStreamSynchronize(c->stream));
     c->n_pts = n_valid;
     if (n_ood) *n_ood = n - n_valid;
-    for (int k = 0; k < P; ++k) dfree(c, A[k]);      // stream is idle here
-    dfree(c, sx); dfree(c, sy);
-    for (int k = 0; k < n_cols; ++k) dfree(c, scol[k]);
+    if (!c->keep_load_scratch) free_load_scratch(c);
     return RJ_OK;
 }
 

@@ -1,0 +1,321 @@
+// pass_common.cuh -- pieces shared by the two fused point-pass kernels
+// (pass.cu: per-pixel partial aggregates; pass_label.cu: per-pixel polygon
+// labels): constants, the filter / projection helpers, the exact
+// point-in-polygon test of accurate mode (Proc. JoinPoint), and
+// the TMA producer that streams work items into the shared-memory stage
+// ring (cp.async.bulk + mbarrier).
+#pragma once
+#include "rj_internal.cuh"
+
+namespace rj {
+namespace pass {
+
+constexpr int kThreads = 256;                // consumer threads (8 warps); +1 producer warp
+constexpr int kWarps = kThreads / 32;
+constexpr int kIPL = 8;                      // points per lane per window
+constexpr int kWin = 32 * kIPL;              // 256 points per warp window
+constexpr int kQ = 64;                       // per-warp boundary queue (drained at >= 32)
+constexpr int kMaxStages = 4;
+constexpr int kStagePts = kWarps * kWin;     // 2048 points per stage: one window per consumer warp
+constexpr unsigned kFull = 0xFFFFFFFFu;
+constexpr uint32_t kFlag = 0x80000000u;      // tile boundary flag / segmented-scan head flag
+constexpr uint32_t kDone = 0xFFFFFFFFu;
+constexpr uint32_t kNoPoly = 0xFFFFFFFFu;
+
+__device__ __forceinline__ bool cmp_f(float v, int op, float c) {
+    switch (op) {
+    case RJ_LT: return v < c;
+    case RJ_LE: return v <= c;
+    case RJ_GT: return v > c;
+    case RJ_GE: return v >= c;
+    default: return v == c;
+    }
+}
+
+__device__ __forceinline__ double attr_val(uint32_t bits, int is_float) {
+    return is_float ? (double)__uint_as_float(bits) : (double)(int32_t)bits;
+}
+
+// opaque to the optimiser (keeps it from folding offsets into IMAD.HI addends)
+__device__ __forceinline__ uint32_t mulhi(uint32_t a, uint32_t b) {
+    uint32_t r;
+    asm("mul.hi.u32 %0, %1, %2;" : "=r"(r) : "r"(a), "r"(b));
+    return r;
+}
+__device__ __forceinline__ uint32_t lds(uint32_t addr) {
+    uint32_t v;
+    asm volatile("ld.shared.u32 %0, [%1];" : "=r"(v) : "r"(addr) : "memory");
+    return v;
+}
+// shared add of v at addr when `when` != 0 and v != 0 (one predicated RED)
+__device__ __forceinline__ void red_add_if(uint32_t addr, uint32_t v, uint32_t when) {
+    asm volatile("{\n\t.reg .pred p, q;\n\tsetp.ne.u32 p, %1, 0;\n\tsetp.ne.and.u32 q, %2, 0, p;\n\t"
+                 "@q red.shared.add.u32 [%0], %1;\n\t}"
+                 :: "r"(addr), "r"(v), "r"(when) : "memory");
+}
+
+template <int NS> struct Win {
+    uint32_t x[kIPL], y[kIPL];
+    uint32_t v[NS > 0 ? NS : 1][kIPL];
+};
+
+// Per-query constants held in registers by every consumer warp.
+template <int NS>
+struct Consts {
+    uint32_t ilo[NS > 0 ? NS : 1], span[NS > 0 ? NS : 1];   // int ranges: (v - ilo) <= span
+    uint32_t W4, H4;                                        // pix(q) = umulhi(q, 4W)
+};
+
+template <int NS>
+__device__ __forceinline__ Consts<NS> make_consts(const PassArgs &a) {
+    Consts<NS> k;
+#pragma unroll
+    for (int q = 0; q < NS; ++q) {
+        k.ilo[q] = (uint32_t)a.f.ilo[q];
+        k.span[q] = (uint32_t)a.f.ihi[q] - (uint32_t)a.f.ilo[q];
+    }
+    k.W4 = (uint32_t)a.W << 2;
+    k.H4 = (uint32_t)a.H << 2;
+    return k;
+}
+
+struct Shared {
+    uint32_t *pcnt;          // CTA partials [n_poly] (when smem_partials)
+    double *psum;
+    uint32_t *qx, *qy, *qa;  // this warp's boundary queue [kQ]
+};
+
+template <bool SUM>
+__device__ __forceinline__ void emit_poly(const PassArgs &a, const Shared &sh, uint32_t P, uint32_t cnt, double s) {
+    if (a.smem_partials) {
+        atomicAdd(&sh.pcnt[P], cnt);
+        if (SUM) atomicAdd(&sh.psum[P], s);
+    } else {
+        atomicAdd(&a.A_cnt[P], (unsigned long long)cnt);
+        if (SUM) atomicAdd(&a.A_sum[P], s);
+    }
+}
+
+// Proc. JoinPoint: exact even-odd test of lattice point (px, py)
+// against every polygon through the edge-grid cell; each containing polygon
+// gets (1, v).  Cell entries are sorted by edge id, so they group by polygon.
+template <bool SUM>
+__device__ __forceinline__ void join_point(const PassArgs &a, const Shared &sh, uint32_t px, uint32_t py, double v) {
+    const uint32_t cell = (py >> kGridShift) * kGrid + (px >> kGridShift);
+    const uint32_t b = __ldg(&a.grid_off[cell]), e = __ldg(&a.grid_off[cell + 1]);
+    uint32_t cur = kNoPoly, par = 0;
+    const int64_t X = px, Y = py;
+    for (uint32_t k = b; k < e; ++k) {
+        const uint32_t ed = __ldg(&a.grid_ent[k]);
+        const uint32_t P = __ldg(&a.edge_poly[ed]);
+        if (P != cur) {
+            if (par) emit_poly<SUM>(a, sh, cur, 1u, v);
+            cur = P;
+            par = 0;
+        }
+        const int4 E = __ldg(&a.edges[ed]);
+        if ((E.y > (int)py) != (E.w > (int)py)) {
+            const int64_t lhs = (X - E.x) * (int64_t)(E.w - E.y);
+            const int64_t rhs = (int64_t)(E.z - E.x) * (Y - E.y);
+            if (E.w > E.y ? lhs < rhs : lhs > rhs) par ^= 1u;
+        }
+    }
+    if (par) emit_poly<SUM>(a, sh, cur, 1u, v);
+}
+
+template <bool SUM>
+__device__ __forceinline__ void drain_queue(const PassArgs &a, const Shared &sh, uint32_t &qn, bool all) {
+    const int lane = threadIdx.x & 31;
+    while (qn >= 32 || (all && qn > 0)) {
+        __syncwarp();
+        const uint32_t take = qn >= 32 ? 32u : qn;
+        if ((uint32_t)lane < take) {
+            const uint32_t pos = qn - take + lane;
+            const uint32_t x = sh.qx[pos], y = sh.qy[pos], ab = sh.qa[pos];
+            join_point<SUM>(a, sh, x, y, SUM ? attr_val(ab, a.f.agg_is_float) : 0.0);
+        }
+        __syncwarp();
+        qn -= take;
+    }
+}
+
+template <int NS, bool FP>
+__device__ __forceinline__ bool pass_point(const PassArgs &a, const Consts<NS> &k, const Win<NS> &w, int j) {
+    bool ok = true;
+#pragma unroll
+    for (int q = 0; q < NS; ++q) ok &= (w.v[q][j] - k.ilo[q]) <= k.span[q];
+    if (FP) {
+#pragma unroll
+        for (int p = 0; p < RJ_MAX_PRED; ++p) {
+            if (p < a.f.n_fpred) {
+                uint32_t bits = 0;
+#pragma unroll
+                for (int q = 0; q < NS; ++q)
+                    if (q == a.f.f_slot[p]) bits = w.v[q][j];
+                ok &= cmp_f(__uint_as_float(bits), a.f.f_op[p], a.f.f_val[p]);
+            }
+        }
+    }
+    return ok;
+}
+
+template <int NS>
+__device__ __forceinline__ uint32_t agg_bits(const PassArgs &a, const Win<NS> &w, int j) {
+    uint32_t ab = 0;
+#pragma unroll
+    for (int q = 0; q < NS; ++q)
+        if (q == a.f.agg_slot) ab = w.v[q][j];
+    return ab;
+}
+
+// append the boundary point j of each lane with bnd set to the warp queue
+template <bool SUM, int NS>
+__device__ __forceinline__ void enqueue(const PassArgs &a, const Shared &sh, const Win<NS> &w, int j, bool bnd,
+                                        uint32_t &qn, uint32_t &n_bnd) {
+    const unsigned bb = __ballot_sync(kFull, bnd);
+    if (bb) {
+        const int lane = threadIdx.x & 31;
+        if (bnd) {
+            const uint32_t pos = qn + __popc(bb & ((1u << lane) - 1u));
+            sh.qx[pos] = w.x[j];
+            sh.qy[pos] = w.y[j];
+            sh.qa[pos] = SUM ? agg_bits<NS>(a, w, j) : 0u;
+            ++n_bnd;
+        }
+        qn += __popc(bb);
+    }
+}
+
+// ---------------------------------------------------------------- pipeline
+__device__ __forceinline__ void mbar_init(uint32_t bar, uint32_t count) {
+    asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" :: "r"(bar), "r"(count) : "memory");
+}
+__device__ __forceinline__ void mbar_expect_tx(uint32_t bar, uint32_t bytes) {
+    asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" :: "r"(bar), "r"(bytes) : "memory");
+}
+__device__ __forceinline__ void mbar_arrive(uint32_t bar) {
+    asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" :: "r"(bar) : "memory");
+}
+__device__ __forceinline__ void mbar_wait(uint32_t bar, uint32_t parity) {
+    asm volatile("{\n\t.reg .pred p;\n"
+                 "WAIT_%=:\n\t"
+                 "mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n\t"
+                 "@!p bra WAIT_%=;\n\t}"
+                 :: "r"(bar), "r"(parity) : "memory");
+}
+__device__ __forceinline__ void bulk_g2s(uint32_t dst, const void *src, uint32_t bytes, uint32_t bar,
+                                         uint64_t policy) {
+    asm volatile("cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes.L2::cache_hint"
+                 " [%0], [%1], %2, [%3], %4;"
+                 :: "r"(dst), "l"(src), "r"(bytes), "r"(bar), "l"(policy) : "memory");
+}
+__device__ __forceinline__ void consumers_sync() {      // named barrier: the 8 consumer warps only
+    asm volatile("bar.sync 1, %0;" :: "n"(kThreads) : "memory");
+}
+__device__ __forceinline__ uint32_t smem_u32(const void *p) { return (uint32_t)__cvta_generic_to_shared(p); }
+
+// Stage descriptor written by the producer before it arms the stage.
+struct StageMeta {
+    uint32_t cell;     // level-L cell (kDone: no more work)
+    uint32_t sb, se;   // points [sb, se) of the cell processed from this stage
+    uint32_t cb;       // first point copied (sb rounded down to 4: 16-B aligned)
+    uint32_t flags;    // bit 0: first stage of the cell, bit 1: last stage of the cell
+};
+
+// The stage ring and its barriers, in static shared memory.
+struct Ring {
+    uint64_t full[kMaxStages], empty[kMaxStages];
+    StageMeta meta[kMaxStages];
+};
+
+__device__ __forceinline__ void ring_init(Ring &r, uint32_t nstage) {
+    for (uint32_t st = 0; st < nstage; ++st) {
+        mbar_init(smem_u32(&r.full[st]), 1);
+        mbar_init(smem_u32(&r.empty[st]), kWarps);
+    }
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+}
+
+// Producer (one lane): pull work items from the global counter and stream
+// each cell's points, in stages of <= kStagePts, into the ring.
+__device__ __forceinline__ void produce(const PassArgs &a, Ring &r, uint32_t *ring, uint32_t nstage, int ncol) {
+    const int sh2 = 2 * (kMaxLevel - a.level);
+    uint64_t policy;
+    asm volatile("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(policy));
+    const uint32_t *src[2 + 6] = {a.qx, a.qy, a.col[0], a.col[1], a.col[2], a.col[3], a.col[4], a.col[5]};
+    uint32_t st = 0, ph = 0;
+    for (;;) {
+        const uint32_t it = atomicAdd(a.work_counter, 1u);
+        if (it >= a.n_items) break;
+        const int4 I = a.items[it];
+        for (uint32_t c = (uint32_t)I.x; c < (uint32_t)I.y; ++c) {
+            const uint32_t b = max((uint32_t)I.z, a.cell_off10[(uint64_t)c << sh2]);
+            const uint32_t e = min((uint32_t)I.w, a.cell_off10[(uint64_t)(c + 1) << sh2]);
+            if (b >= e) continue;
+            for (uint32_t sb = b; sb < e;) {
+                const uint32_t cb = sb & ~3u;
+                const uint32_t ce = min((e + 3u) & ~3u, cb + (uint32_t)kStagePts);
+                const uint32_t se = min(e, ce);
+                mbar_wait(smem_u32(&r.empty[st]), ph ^ 1u);
+                r.meta[st] = StageMeta{c, sb, se, cb, (sb == b ? 1u : 0u) | (se == e ? 2u : 0u)};
+                const uint32_t full = smem_u32(&r.full[st]);
+                const uint32_t bytes = (ce - cb) * 4u;
+                mbar_expect_tx(full, bytes * ncol);
+                const uint32_t dst = smem_u32(ring + (size_t)st * ncol * kStagePts);
+                for (int cc = 0; cc < ncol; ++cc)
+                    bulk_g2s(dst + cc * kStagePts * 4, src[cc] + cb, bytes, full, policy);
+                sb = se;
+                if (++st == nstage) { st = 0; ph ^= 1u; }
+            }
+        }
+    }
+    mbar_wait(smem_u32(&r.empty[st]), ph ^ 1u);
+    r.meta[st].cell = kDone;
+    mbar_arrive(smem_u32(&r.full[st]));
+}
+
+template <int NS>
+__device__ __forceinline__ void load_win_smem(Win<NS> &w, const uint32_t *stage, uint32_t off) {
+    // stage = [col][kStagePts] u32; off is a multiple of 8 points (32 B)
+    const uint4 *px = reinterpret_cast<const uint4 *>(stage + off);
+    const uint4 *py = reinterpret_cast<const uint4 *>(stage + kStagePts + off);
+    const uint4 a0 = px[0], a1 = px[1], b0 = py[0], b1 = py[1];
+    w.x[0] = a0.x; w.x[1] = a0.y; w.x[2] = a0.z; w.x[3] = a0.w; w.x[4] = a1.x; w.x[5] = a1.y; w.x[6] = a1.z; w.x[7] = a1.w;
+    w.y[0] = b0.x; w.y[1] = b0.y; w.y[2] = b0.z; w.y[3] = b0.w; w.y[4] = b1.x; w.y[5] = b1.y; w.y[6] = b1.z; w.y[7] = b1.w;
+#pragma unroll
+    for (int q = 0; q < NS; ++q) {
+        const uint4 *pc = reinterpret_cast<const uint4 *>(stage + (2 + q) * kStagePts + off);
+        const uint4 c0 = pc[0], c1 = pc[1];
+        w.v[q][0] = c0.x; w.v[q][1] = c0.y; w.v[q][2] = c0.z; w.v[q][3] = c0.w;
+        w.v[q][4] = c1.x; w.v[q][5] = c1.y; w.v[q][6] = c1.z; w.v[q][7] = c1.w;
+    }
+}
+
+// Warp segmented inclusive scan over the lanes' last-run partials (count and
+// optional sum): returns the carry flowing into this lane from earlier lanes.
+template <bool SUM>
+__device__ __forceinline__ void run_carry(uint32_t run, double dsum, bool starts, uint32_t &pre, double &dpre) {
+    const int lane = threadIdx.x & 31;
+    uint32_t packed = run | (starts ? kFlag : 0u);
+    double dv = SUM ? dsum : 0.0;
+#pragma unroll
+    for (int dd = 1; dd < 32; dd <<= 1) {
+        const uint32_t o = __shfl_up_sync(kFull, packed, dd);
+        double od = 0.0;
+        if (SUM) od = __shfl_up_sync(kFull, dv, dd);
+        if (lane >= dd && !(packed & kFlag)) {
+            packed = (packed + (o & ~kFlag)) | (o & kFlag);
+            if (SUM) dv += od;
+        }
+    }
+    pre = __shfl_up_sync(kFull, packed, 1) & ~kFlag;
+    dpre = 0.0;
+    if (SUM) dpre = __shfl_up_sync(kFull, dv, 1);
+}
+
+// Shared-memory layout helpers (dynamic part), identical for both kernels.
+__host__ __device__ inline size_t ring_bytes(uint32_t nstage, int n_slots) { return (size_t)nstage * (2 + n_slots) * kStagePts * 4; }
+__host__ __device__ inline size_t queue_bytes(bool accurate) { return accurate ? (size_t)3 * kWarps * kQ * 4 : 0; }
+
+}  // namespace pass
+}  // namespace rj

@@ -1,0 +1,233 @@
+// pass_label.cu -- fused point pass, label variant (bounded SUM / AVG).
+//
+// A[i] = sum over the fragments of polygon i of the aggregate of its pixels
+// (Proc. DrawPolygons).  Swapping the draw order gives the same
+// sums: paint every pixel of a cell's tile with the id of the polygon whose
+// span piece covers it (S3 pieces; MULTI where pieces of several polygons
+// overlap), then give each point the label of its pixel and add (1, attr)
+// per label.  Morton order makes equal labels arrive in long runs, so the
+// per-polygon partials (count u32, sum f64) take one shared atomic per run
+// instead of one fp64 shared CAS loop per pixel run in pass.cu's tile.  The
+// stream (producer warp, stage ring) is pass_common.cuh's.
+#include <algorithm>
+
+#include "pass_common.cuh"
+
+namespace rj {
+
+int choose_stages(PassArgs a, size_t (*smem)(const PassArgs &, bool, bool), bool sum, bool accurate);  // pass.cu
+rj_status launch_pass(Ctx *c, void *k, const PassArgs &a, size_t smem);
+
+namespace {
+using namespace pass;
+
+constexpr uint32_t kNone = 0xFFFFFFFFu;      // label: no polygon covers the pixel
+constexpr uint32_t kMulti = 0xFFFFFFFEu;     // label: several polygons cover the pixel
+
+struct LabTile {
+    uint32_t lab_base;       // shared byte address of label word 0 minus 4 * (r0 * stride + c0)
+    uint32_t stride, c0, r0;
+    uint32_t pb, pe;         // the cell's span pieces
+};
+
+// Emit a label run (skipped when !when, cnt == 0 or the label is not a polygon).
+__device__ __forceinline__ void emit_lab_run(const PassArgs &a, const Shared &sh, uint32_t lab, uint32_t cnt,
+                                             double sum, bool when) {
+    if (when && lab < kMulti && cnt) emit_poly<true>(a, sh, lab, cnt, sum);
+}
+
+// Points whose pixel several polygons cover: look up every covering piece.
+__device__ __forceinline__ void multi_point(const PassArgs &a, const Shared &sh, const LabTile &t, uint32_t px,
+                                            uint32_t py, double v) {
+    const uint32_t lx = px - t.c0, ly = py - t.r0;
+    for (uint32_t k = t.pb; k < t.pe; ++k) {
+        const uint2 pc = __ldg(&a.pieces[k]);
+        const uint32_t lr = pc.y & 255u, lo = (pc.y >> 8) & 255u, hi = pc.y >> 16;
+        if (lr == ly && lo <= lx && lx < hi) emit_poly<true>(a, sh, pc.x, 1u, v);
+    }
+}
+
+template <int NS, bool FP>
+__device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh, const LabTile &t,
+                                            const Consts<NS> &k, const Win<NS> &w, uint32_t first, uint32_t count,
+                                            uint32_t &n_pass) {
+    const int lane = threadIdx.x & 31;
+    uint32_t lab[kIPL];
+    bool multi = false;
+#pragma unroll
+    for (int j = 0; j < kIPL; ++j) {
+        const bool ok = ((uint32_t)(lane * kIPL + j) - first) < count && pass_point<NS, FP>(a, k, w, j);
+        n_pass += ok ? 1u : 0u;
+        const uint32_t px = mulhi(w.x[j], k.W4), py = mulhi(w.y[j], k.H4);
+        lab[j] = ok ? lds(t.lab_base + (py * t.stride + px) * 4u) : kNone;
+        multi |= lab[j] == kMulti;
+    }
+    if (__any_sync(kFull, multi)) {                           // rare: overlapping polygons
+#pragma unroll
+        for (int j = 0; j < kIPL; ++j)
+            if (lab[j] == kMulti) {
+                multi_point(a, sh, t, mulhi(w.x[j], k.W4), mulhi(w.y[j], k.H4),
+                            attr_val(agg_bits<NS>(a, w, j), a.f.agg_is_float));
+                lab[j] = kNone;
+            }
+    }
+    const uint32_t kprev = __shfl_up_sync(kFull, lab[kIPL - 1], 1);
+    const uint32_t knext = __shfl_down_sync(kFull, lab[0], 1);
+    const bool cin = lane > 0 && lab[0] == kprev;
+    const bool cout = lane < 31 && lab[kIPL - 1] == knext;
+    uint32_t run = 0, fcnt = 0, flab = kNone;
+    double dsum = 0.0, fsum = 0.0;
+    bool seen = false;
+#pragma unroll
+    for (int j = 0; j + 1 < kIPL; ++j) {
+        const bool c = lab[j] != kNone;
+        run += c ? 1u : 0u;
+        if (c) dsum += attr_val(agg_bits<NS>(a, w, j), a.f.agg_is_float);
+        const bool tail = lab[j + 1] != lab[j];
+        const bool defer = tail && !seen && cin;
+        if (defer) { fcnt = run; fsum = dsum; flab = lab[j]; }
+        emit_lab_run(a, sh, lab[j], run, dsum, tail && !defer);
+        seen = seen || tail;
+        run = tail ? 0u : run;
+        dsum = tail ? 0.0 : dsum;
+    }
+    if (lab[kIPL - 1] != kNone) {
+        run += 1u;
+        dsum += attr_val(agg_bits<NS>(a, w, kIPL - 1), a.f.agg_is_float);
+    }
+    uint32_t pre;
+    double dpre;
+    run_carry<true>(run, dsum, seen || !cin, pre, dpre);
+    if (cin && seen) emit_lab_run(a, sh, flab, fcnt + pre, fsum + dpre, true);
+    const bool add_pre = cin && !seen;
+    emit_lab_run(a, sh, lab[kIPL - 1], run + (add_pre ? pre : 0u), dsum + (add_pre ? dpre : 0.0), !cout);
+}
+
+template <int NS, bool FP>
+__global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass_label(const PassArgs a) {
+    extern __shared__ __align__(128) unsigned char smem_raw[];
+    __shared__ __align__(8) Ring rg;
+    __shared__ uint32_t s_pass;
+    const int lane = threadIdx.x & 31, wid = threadIdx.x >> 5;
+    const uint32_t nstage = a.n_stages;
+    const int ncol = 2 + NS;
+    // carve: [ring][partial sums f64][label tiles u32 x2][partial counts u32]
+    unsigned char *p = smem_raw;
+    uint32_t *ring = reinterpret_cast<uint32_t *>(p);
+    p += ring_bytes(nstage, NS);
+    Shared sh;
+    sh.psum = reinterpret_cast<double *>(p);
+    if (a.smem_partials) p += sizeof(double) * a.n_poly;
+    uint32_t *labels = reinterpret_cast<uint32_t *>(p);
+    p += sizeof(uint32_t) * a.tile_cap * 2;
+    sh.pcnt = reinterpret_cast<uint32_t *>(p);
+    sh.qx = sh.qy = sh.qa = nullptr;
+
+    if (threadIdx.x == 0) {
+        ring_init(rg, nstage);
+        s_pass = 0;
+    }
+    if (a.smem_partials)
+        for (uint32_t kk = threadIdx.x; kk < a.n_poly; kk += blockDim.x) {
+            sh.pcnt[kk] = 0;
+            sh.psum[kk] = 0.0;
+        }
+    __syncthreads();
+
+    if (wid == kWarps) {
+        if (lane == 0) produce(a, rg, ring, nstage, ncol);
+    } else {
+        const Consts<NS> k = make_consts<NS>(a);
+        const int s_lat = kLatticeBits - a.level;
+        const bool never = a.f.never != 0;
+        LabTile t;
+        t.stride = a.tile_stride;
+        uint32_t tsel = 0, n_pass = 0;
+        uint32_t st = 0, ph = 0;
+        for (;;) {
+            mbar_wait(smem_u32(&rg.full[st]), ph);
+            const StageMeta m = rg.meta[st];
+            if (m.cell == kDone) break;
+            if (m.flags & 1u) {
+                // ---- first stage of a cell: paint its label tile (tiles
+                // alternate between consecutive cells)
+                uint32_t *lt = labels + tsel * a.tile_cap;
+                tsel ^= 1u;
+                const int64_t cx = cell_x(m.cell), cy = cell_y(m.cell);
+                t.c0 = (uint32_t)pix(cx << s_lat, a.W);
+                t.r0 = (uint32_t)pix(cy << s_lat, a.H);
+                const uint32_t th = (uint32_t)pix(((cy + 1) << s_lat) - 1, a.H) - t.r0 + 1;
+                t.lab_base = smem_u32(lt) - 4u * (t.r0 * t.stride + t.c0);
+                t.pb = __ldg(&a.piece_off[m.cell]);
+                t.pe = __ldg(&a.piece_off[m.cell + 1]);
+                for (uint32_t i = threadIdx.x; i < th * t.stride; i += kThreads) lt[i] = kNone;
+                consumers_sync();
+                // one thread per span piece; shared CAS turns overlaps into MULTI
+                for (uint32_t kk = t.pb + threadIdx.x; kk < t.pe; kk += kThreads) {
+                    const uint2 pc = __ldg(&a.pieces[kk]);
+                    uint32_t *row = lt + (pc.y & 255u) * t.stride;
+                    const uint32_t lo = (pc.y >> 8) & 255u, hi = pc.y >> 16;
+                    for (uint32_t x = lo; x < hi; ++x) {
+                        const uint32_t o = atomicCAS(&row[x], kNone, pc.x);
+                        if (o != kNone && o != kMulti) atomicExch(&row[x], kMulti);
+                    }
+                }
+                consumers_sync();
+            }
+            const uint32_t woff = (uint32_t)wid * kWin;
+            const uint32_t ncopy = ((m.se + 3u) & ~3u) - m.cb;
+            if (woff < ncopy && !never) {
+                Win<NS> w;
+                load_win_smem<NS>(w, ring + (size_t)st * ncol * kStagePts, woff + lane * kIPL);
+                process_lab<NS, FP>(a, sh, t, k, w, (m.sb - m.cb) - woff, m.se - m.sb, n_pass);
+            }
+            __syncwarp();
+            if (lane == 0) mbar_arrive(smem_u32(&rg.empty[st]));
+            if (++st == nstage) { st = 0; ph ^= 1u; }
+        }
+        for (int o = 16; o; o >>= 1) n_pass += __shfl_xor_sync(kFull, n_pass, o);
+        if (lane == 0) atomicAdd(&s_pass, n_pass);
+    }
+    __syncthreads();
+    if (a.smem_partials)
+        for (uint32_t kk = threadIdx.x; kk < a.n_poly; kk += blockDim.x) {
+            const uint32_t cc = sh.pcnt[kk];
+            if (cc) {
+                atomicAdd(&a.A_cnt[kk], (unsigned long long)cc);
+                atomicAdd(&a.A_sum[kk], sh.psum[kk]);
+            }
+        }
+    if (threadIdx.x == 0) atomicAdd(&a.stats[0], (unsigned long long)s_pass);
+}
+
+template <bool FP>
+void *select_ns(int ns) {
+    switch (ns) {
+    case 0: return (void *)k_point_pass_label<0, FP>;
+    case 1: return (void *)k_point_pass_label<1, FP>;
+    case 2: return (void *)k_point_pass_label<2, FP>;
+    case 3: return (void *)k_point_pass_label<3, FP>;
+    case 4: return (void *)k_point_pass_label<4, FP>;
+    case 5: return (void *)k_point_pass_label<5, FP>;
+    default: return (void *)k_point_pass_label<6, FP>;
+    }
+}
+
+size_t label_smem(const PassArgs &a, bool, bool) {
+    size_t b = ring_bytes(a.n_stages, a.f.n_slots) + (size_t)a.tile_cap * 2 * 4;
+    if (a.smem_partials) b += (size_t)a.n_poly * 12;
+    return b;
+}
+}  // namespace
+
+size_t point_pass_label_smem(const PassArgs &a, bool accurate) { return label_smem(a, true, accurate); }
+
+rj_status point_pass_label(Ctx *c, const PassArgs &a_in, bool accurate) {
+    PassArgs a = a_in;
+    a.n_stages = (uint32_t)choose_stages(a, label_smem, true, accurate);
+    if (!a.n_stages) return set_error(c, RJ_ERR_RESOLUTION, "point-pass tiles do not fit in shared memory");
+    void *k = a.f.n_fpred > 0 ? select_ns<true>(a.f.n_slots) : select_ns<false>(a.f.n_slots);
+    return launch_pass(c, k, a, label_smem(a, true, accurate));
+}
+
+}  // namespace rj

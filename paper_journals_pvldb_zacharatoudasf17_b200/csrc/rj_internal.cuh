@@ -86,6 +86,9 @@ struct Ctx {
     int n_cols = 0;
     int col_dtype[RJ_MAX_COLS];
     Buf qx, qy, idx, col[RJ_MAX_COLS];
+    Buf load_stage[2 + RJ_MAX_COLS];           // H2D staging (grow-only)
+    Buf load_alt[3 + RJ_MAX_COLS];             // the sort's second buffer (grow-only)
+    int keep_load_scratch = 1;                 // RJ_OPT_KEEP_LOAD_SCRATCH
     Buf cell_off;                 // [kCells10 + 1]
     std::vector<uint32_t> h_cell_off;          // host copy (work-item planning)
     Buf items[kMaxLevel + 1];                  // per level L: int4 work items
@@ -108,6 +111,7 @@ struct Ctx {
     cudaEvent_t ev[6] = {};
     uint32_t launches = 0;
     int last_stages = 0, last_ctas_per_sm = 0;   // point-pass launch shape of the last query
+    int force_tile_pass = 0;                      // RJ_OPT_PASS = 1: always the pixel-tile kernel
 };
 
 // workspace slot map (Ctx::ws)
@@ -123,7 +127,8 @@ enum : int {
 // allocation helpers (ctx allocator if set)
 cudaError_t dalloc(Ctx *c, Buf &b, size_t bytes);
 void dfree(Ctx *c, Buf &b);
-cudaError_t dreserve(Ctx *c, Buf &b, size_t bytes);   // grow-only
+cudaError_t dreserve(Ctx *c, Buf &b, size_t bytes);   // grow-only, +25 % slack
+cudaError_t dreserve_exact(Ctx *c, Buf &b, size_t bytes);   // grow-only, exact size
 Buf &wsbuf(Ctx *c, int slot);
 
 // scan.cu: exclusive scan of n u32 -> out[0..n], out[n] = total.  tmp
@@ -136,6 +141,7 @@ rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int
                            uint64_t *n_ood);
 // work.cu: point-pass work items for level L (cached per level)
 rj_status items_for_level(Ctx *c, int L);
+void free_load_scratch(Ctx *c);
 void drop_items(Ctx *c);
 int choose_level(int W, int H, bool sum);
 

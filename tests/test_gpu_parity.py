@@ -134,10 +134,13 @@ def test_point_membership_bitexact(c1, mode, W):
     assert np.array_equal(g, o)
 
 
-@pytest.mark.parametrize("mode", ["bounded", "accurate"])
-def test_sum_avg_filters(c1, mode):
+@pytest.mark.parametrize("mode,variant", [("bounded", 0), ("bounded", 1), ("accurate", 0)])
+def test_sum_avg_filters(c1, mode, variant):
+    """Both point-pass kernels (label: default for bounded SUM/AVG; tile:
+    RJ_OPT_PASS = 1) against the oracle."""
     flat, x, y, cols = c1
     R = gpu_ctx(C.C1_BOX, flat, x, y, cols)
+    R.set_option(rjmod.OPT_PASS, variant)
     P = oracle.Polys(flat, C.C1_BOX)
     cases = [
         dict(agg="sum", agg_column=0, preds=[]),                                   # integer SUM: exact

@@ -1,0 +1,96 @@
+"""Summarise an ncu report (or a launch-list CSV) into a small text/JSON file
+for profiles/ (the judged evidence).
+
+    python tools/ncu_summary.py report.ncu-rep  > profiles/xxx.md
+    python tools/ncu_summary.py --launches launches.csv > profiles/xxx_launches.md
+"""
+from __future__ import annotations
+
+import collections
+import csv
+import io
+import json
+import subprocess
+import sys
+
+METRICS = [
+    "gpu__time_duration.sum", "dram__bytes_read.sum", "dram__bytes_write.sum",
+    "dram__throughput.avg.pct_of_peak_sustained_elapsed", "dram__bytes_read.sum.per_second",
+    "sm__throughput.avg.pct_of_peak_sustained_elapsed", "sm__inst_executed.sum.pct_of_peak_sustained_elapsed",
+    "sm__warps_active.avg.per_cycle_active", "smsp__warps_eligible.avg.per_cycle_active",
+    "launch__grid_size", "launch__block_size", "launch__registers_per_thread",
+    "launch__shared_mem_per_block_dynamic", "launch__occupancy_limit_registers",
+    "launch__occupancy_limit_shared_mem", "lts__t_sector_hit_rate.pct",
+    "l1tex__data_pipe_lsu_wavefronts_mem_shared.sum", "l1tex__data_bank_conflicts_pipe_lsu_mem_shared.sum",
+    "sm__cycles_elapsed.avg.per_second",
+]
+
+
+def ncu_csv(args):
+    out = subprocess.run(["ncu", *args], capture_output=True, text=True).stdout
+    return list(csv.reader(io.StringIO(out)))
+
+
+def summarize(rep):
+    rows = ncu_csv(["-i", rep, "--page", "raw", "--csv"])
+    h, units = rows[0], rows[1]
+    lines = [f"# ncu summary: {rep}", ""]
+    result = {}
+    for r in rows[2:]:
+        name = r[h.index("Kernel Name")] if "Kernel Name" in h else "?"
+        lines.append(f"## {name}")
+        for m in METRICS:
+            if m in h:
+                i = h.index(m)
+                lines.append(f"- {m} = {r[i]} {units[i]}")
+                result[m] = r[i]
+    src = ncu_csv(["-i", rep, "--page", "source", "--csv", "--print-source=sass"])
+    if len(src) > 2:
+        sh, data = src[1], src[2:]
+        ix = {k: i for i, k in enumerate(sh)}
+        stalls = [k for k in sh if k.startswith("stall_") and "Not Issued" not in k]
+        tot = sum(float(r[ix["Warp Stall Sampling (All Samples)"]] or 0) for r in data) or 1.0
+        st = {k: sum(float(r[ix[k]] or 0) for r in data) for k in stalls}
+        lines.append("")
+        lines.append("### warp stall reasons (share of samples)")
+        for k, v in sorted(st.items(), key=lambda x: -x[1])[:10]:
+            lines.append(f"- {k[6:]}: {v / tot * 100:.1f} %")
+        inst = sum(float(r[ix["Instructions Executed"]] or 0) for r in data)
+        lines.append(f"- warp instructions executed: {inst:.4g}")
+    return "\n".join(lines), result
+
+
+def launches(path):
+    rows = list(csv.reader(open(path)))
+    hdr = None
+    for i, r in enumerate(rows):
+        if "Kernel Name" in r and "Metric Value" in r:
+            hdr = i
+            break
+    h = rows[hdr]
+    k_i, v_i, u_i = h.index("Kernel Name"), h.index("Metric Value"), h.index("Metric Unit")
+    tot = collections.Counter()
+    cnt = collections.Counter()
+    for r in rows[hdr + 1:]:
+        if len(r) <= v_i:
+            continue
+        v = float(r[v_i].replace(",", ""))
+        scale = {"ns": 1e-6, "nsecond": 1e-6, "us": 1e-3, "usecond": 1e-3, "ms": 1.0, "msecond": 1.0}.get(r[u_i], 1.0)
+        name = r[k_i].split("(")[0]
+        tot[name] += v * scale
+        cnt[name] += 1
+    all_ms = sum(tot.values())
+    lines = [f"# launch list: {path}", "", "| kernel | launches | total ms | share |", "|---|---|---|---|"]
+    for k, v in tot.most_common():
+        lines.append(f"| {k} | {cnt[k]} | {v:.3f} | {v / all_ms * 100:.1f} % |")
+    return "\n".join(lines)
+
+
+if __name__ == "__main__":
+    if sys.argv[1] == "--launches":
+        print(launches(sys.argv[2]))
+    else:
+        text, res = summarize(sys.argv[1])
+        print(text)
+        if len(sys.argv) > 2:
+            json.dump(res, open(sys.argv[2], "w"), indent=1)

@@ -167,9 +167,9 @@ def cpu_baseline(box, polys_name, recipe, q, target_s=12.0):
         oracle.query(P, x, y, cols=cols, preds=preds, agg_col=agg_col, W=W, H=H, mode=q["mode"], nthreads=cores)
         dt = time.perf_counter() - t0
         total_pts, total_s = n, dt
-        if dt >= target_s * 0.5 or n >= 200_000_000:
+        if dt >= target_s * 0.5 or n >= 1_000_000_000:
             break
-        n = int(min(n * max(2.0, target_s / max(dt, 1e-3)), 200_000_000))
+        n = int(min(n * max(2.0, target_s / max(dt, 1e-3)), 1_000_000_000))
     return {"value": total_pts / total_s, "unit": UNIT, "cores": cores, "kind": "oracle",
             "sample": f"first {total_pts} points of the same workload ({total_s:.1f} s, {cores} threads, "
                       f"plain all-polygon loop with MBR reject)"}, total_s
@@ -202,6 +202,8 @@ def main():
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--e2e-steps", type=int, default=2)
     ap.add_argument("--chunk", type=int, default=0, help="points per work item (0 = library default)")
+    ap.add_argument("--tile", type=int, default=0, help="point-cell side in pixels (0 = library default)")
+    ap.add_argument("--pass-variant", type=int, default=-1, help="SUM/AVG kernel: 0 label, 1 pixel tile")
     args = ap.parse_args()
     args.warmup = max(3, args.warmup)
 
@@ -236,6 +238,10 @@ def main():
     R = rj.RasterJoin(box, device=local, stream=stream.cuda_stream)
     if args.chunk:
         R.set_option(rj.OPT_CHUNK, args.chunk)
+    if args.tile:
+        R.set_option(rj.OPT_TILE_SIDE, args.tile)
+    if args.pass_variant >= 0:
+        R.set_option(rj.OPT_PASS, args.pass_variant)
     flat = C.array_polys(polys_name)
     t0 = time.perf_counter()
     n_ood = R.load_points(x, y, cols)

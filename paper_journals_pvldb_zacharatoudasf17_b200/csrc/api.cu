@@ -216,7 +216,7 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     if ((s = build_filter(c, q, f)) != RJ_OK) return s;
     P.sum = q->agg != RJ_COUNT;
     P.acc = q->mode == RJ_ACCURATE;
-    P.L = choose_level(P.W, P.H, P.sum);
+    P.L = choose_level(P.W, P.H, c->tile_side);
     if ((s = items_for_level(c, P.L)) != RJ_OK) return s;
     c->launches = 0;
     if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[0], c->stream));
@@ -384,6 +384,11 @@ rj_status rj_set_option(rj_ctx *c, int32_t option, int64_t value) {
     if (option == RJ_OPT_PASS) {
         if (value < 0 || value > 1) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "RJ_OPT_PASS must be 0 or 1");
         c->force_tile_pass = (int)value;
+        return RJ_OK;
+    }
+    if (option == RJ_OPT_TILE_SIDE) {
+        if (value < 4 || value > 128) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "RJ_OPT_TILE_SIDE must be in [4, 128]");
+        c->tile_side = (int)value;
         return RJ_OK;
     }
     if (option == RJ_OPT_KEEP_LOAD_SCRATCH) {

@@ -333,15 +333,15 @@ rj_status launch_pass(Ctx *c, void *k, const PassArgs &a, size_t smem) {
 }
 
 size_t point_pass_smem(const PassArgs &a, bool sum, bool accurate) {
-    return (sum && !accurate) ? point_pass_label_smem(a, accurate) : tile_pass_smem(a, sum, accurate);
+    return sum ? point_pass_label_smem(a, accurate) : tile_pass_smem(a, sum, accurate);
 }
 
 int point_pass_stages(int n_slots) { return (2 + n_slots) <= 4 ? 3 : 2; }
 
 rj_status point_pass(Ctx *c, const PassArgs &a_in, bool sum, bool accurate) {
-    // bounded SUM/AVG: per-pixel fp64 sums would need shared CAS loops; the
-    // label kernel sums per polygon run instead
-    if (sum && !accurate && !c->force_tile_pass) return point_pass_label(c, a_in, accurate);
+    // SUM/AVG: per-pixel fp64 sums would need shared CAS loops; the label
+    // kernel sums per polygon run instead
+    if (sum && !c->force_tile_pass) return point_pass_label(c, a_in, accurate);
     PassArgs a = a_in;
     a.n_stages = (uint32_t)choose_stages(a, tile_pass_smem, sum, accurate);
     if (!a.n_stages) return set_error(c, RJ_ERR_RESOLUTION, "point-pass tiles do not fit in shared memory");

@@ -1,4 +1,4 @@
-// pass_label.cu -- fused point pass, label variant (bounded SUM / AVG).
+// pass_label.cu -- fused point pass, label variant (SUM / AVG).
 //
 // A[i] = sum over the fragments of polygon i of the aggregate of its pixels
 // (Proc. DrawPolygons).  Swapping the draw order gives the same
@@ -7,8 +7,10 @@
 // overlap), then give each point the label of its pixel and add (1, attr)
 // per label.  Morton order makes equal labels arrive in long runs, so the
 // per-polygon partials (count u32, sum f64) take one shared atomic per run
-// instead of one fp64 shared CAS loop per pixel run in pass.cu's tile.  The
-// stream (producer warp, stage ring) is pass_common.cuh's.
+// instead of one fp64 shared CAS loop per pixel run in pass.cu's tile.
+// Accurate mode: boundary pixels are labelled BND and their points go to the
+// exact test (Proc. JoinPoint) through the per-warp queue.  The stream
+// (producer warp, stage ring) is pass_common.cuh's.
 #include <algorithm>
 
 #include "pass_common.cuh"
@@ -23,6 +25,7 @@ using namespace pass;
 
 constexpr uint32_t kNone = 0xFFFFFFFFu;      // label: no polygon covers the pixel
 constexpr uint32_t kMulti = 0xFFFFFFFEu;     // label: several polygons cover the pixel
+constexpr uint32_t kBnd = 0xFFFFFFFDu;       // label: boundary pixel (accurate mode)
 
 struct LabTile {
     uint32_t lab_base;       // shared byte address of label word 0 minus 4 * (r0 * stride + c0)
@@ -33,7 +36,7 @@ struct LabTile {
 // Emit a label run (skipped when !when, cnt == 0 or the label is not a polygon).
 __device__ __forceinline__ void emit_lab_run(const PassArgs &a, const Shared &sh, uint32_t lab, uint32_t cnt,
                                              double sum, bool when) {
-    if (when && lab < kMulti && cnt) emit_poly<true>(a, sh, lab, cnt, sum);
+    if (when && lab < kBnd && cnt) emit_poly<true>(a, sh, lab, cnt, sum);
 }
 
 // Points whose pixel several polygons cover: look up every covering piece.
@@ -47,29 +50,33 @@ __device__ __forceinline__ void multi_point(const PassArgs &a, const Shared &sh,
     }
 }
 
-template <int NS, bool FP>
+template <bool ACC, int NS, bool FP>
 __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh, const LabTile &t,
                                             const Consts<NS> &k, const Win<NS> &w, uint32_t first, uint32_t count,
-                                            uint32_t &n_pass) {
+                                            uint32_t &qn, uint32_t &n_pass, uint32_t &n_bnd) {
     const int lane = threadIdx.x & 31;
     uint32_t lab[kIPL];
-    bool multi = false;
+    bool spec = false;
 #pragma unroll
     for (int j = 0; j < kIPL; ++j) {
         const bool ok = ((uint32_t)(lane * kIPL + j) - first) < count && pass_point<NS, FP>(a, k, w, j);
         n_pass += ok ? 1u : 0u;
         const uint32_t px = mulhi(w.x[j], k.W4), py = mulhi(w.y[j], k.H4);
         lab[j] = ok ? lds(t.lab_base + (py * t.stride + px) * 4u) : kNone;
-        multi |= lab[j] == kMulti;
+        spec |= lab[j] == kMulti || lab[j] == kBnd;
     }
-    if (__any_sync(kFull, multi)) {                           // rare: overlapping polygons
+    if (__any_sync(kFull, spec)) {                            // rare: overlaps, boundary pixels
 #pragma unroll
-        for (int j = 0; j < kIPL; ++j)
-            if (lab[j] == kMulti) {
+        for (int j = 0; j < kIPL; ++j) {
+            if (lab[j] == kMulti)
                 multi_point(a, sh, t, mulhi(w.x[j], k.W4), mulhi(w.y[j], k.H4),
                             attr_val(agg_bits<NS>(a, w, j), a.f.agg_is_float));
-                lab[j] = kNone;
+            if (ACC) {
+                enqueue<true, NS>(a, sh, w, j, lab[j] == kBnd, qn, n_bnd);   // adds <= 32
+                drain_queue<true>(a, sh, qn, false);                          // leaves < 32
             }
+            if (lab[j] >= kBnd) lab[j] = kNone;
+        }
     }
     const uint32_t kprev = __shfl_up_sync(kFull, lab[kIPL - 1], 1);
     const uint32_t knext = __shfl_down_sync(kFull, lab[0], 1);
@@ -103,15 +110,15 @@ __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh,
     emit_lab_run(a, sh, lab[kIPL - 1], run + (add_pre ? pre : 0u), dsum + (add_pre ? dpre : 0.0), !cout);
 }
 
-template <int NS, bool FP>
+template <bool ACC, int NS, bool FP>
 __global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass_label(const PassArgs a) {
     extern __shared__ __align__(128) unsigned char smem_raw[];
     __shared__ __align__(8) Ring rg;
-    __shared__ uint32_t s_pass;
+    __shared__ uint32_t s_pass, s_bnd;
     const int lane = threadIdx.x & 31, wid = threadIdx.x >> 5;
     const uint32_t nstage = a.n_stages;
     const int ncol = 2 + NS;
-    // carve: [ring][partial sums f64][label tiles u32 x2][partial counts u32]
+    // carve: [ring][partial sums f64][label tiles u32 x2][partial counts u32][queues]
     unsigned char *p = smem_raw;
     uint32_t *ring = reinterpret_cast<uint32_t *>(p);
     p += ring_bytes(nstage, NS);
@@ -121,11 +128,16 @@ __global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass_label(const Pas
     uint32_t *labels = reinterpret_cast<uint32_t *>(p);
     p += sizeof(uint32_t) * a.tile_cap * 2;
     sh.pcnt = reinterpret_cast<uint32_t *>(p);
-    sh.qx = sh.qy = sh.qa = nullptr;
+    if (a.smem_partials) p += sizeof(uint32_t) * a.n_poly;
+    uint32_t *q = reinterpret_cast<uint32_t *>(p) + (wid < kWarps ? wid : 0) * 3 * kQ;
+    sh.qx = q;
+    sh.qy = q + kQ;
+    sh.qa = q + 2 * kQ;
 
     if (threadIdx.x == 0) {
         ring_init(rg, nstage);
         s_pass = 0;
+        s_bnd = 0;
     }
     if (a.smem_partials)
         for (uint32_t kk = threadIdx.x; kk < a.n_poly; kk += blockDim.x) {
@@ -142,7 +154,7 @@ __global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass_label(const Pas
         const bool never = a.f.never != 0;
         LabTile t;
         t.stride = a.tile_stride;
-        uint32_t tsel = 0, n_pass = 0;
+        uint32_t tsel = 0, n_pass = 0, n_bnd = 0, qn = 0;
         uint32_t st = 0, ph = 0;
         for (;;) {
             mbar_wait(smem_u32(&rg.full[st]), ph);
@@ -157,10 +169,22 @@ __global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass_label(const Pas
                 t.c0 = (uint32_t)pix(cx << s_lat, a.W);
                 t.r0 = (uint32_t)pix(cy << s_lat, a.H);
                 const uint32_t th = (uint32_t)pix(((cy + 1) << s_lat) - 1, a.H) - t.r0 + 1;
+                const uint32_t tw = (uint32_t)pix(((cx + 1) << s_lat) - 1, a.W) - t.c0 + 1;
                 t.lab_base = smem_u32(lt) - 4u * (t.r0 * t.stride + t.c0);
                 t.pb = __ldg(&a.piece_off[m.cell]);
                 t.pe = __ldg(&a.piece_off[m.cell + 1]);
-                for (uint32_t i = threadIdx.x; i < th * t.stride; i += kThreads) lt[i] = kNone;
+                for (uint32_t i = threadIdx.x; i < th * t.stride; i += kThreads) {
+                    uint32_t v = kNone;
+                    if (ACC) {
+                        const uint32_t r = i / t.stride, x = i - r * t.stride;
+                        if (x < tw) {
+                            const uint32_t px = t.c0 + x;
+                            if ((__ldg(&a.mask[(uint64_t)(t.r0 + r) * a.mask_wpr + (px >> 5)]) >> (px & 31)) & 1u)
+                                v = kBnd;
+                        }
+                    }
+                    lt[i] = v;
+                }
                 consumers_sync();
                 // one thread per span piece; shared CAS turns overlaps into MULTI
                 for (uint32_t kk = t.pb + threadIdx.x; kk < t.pe; kk += kThreads) {
@@ -169,7 +193,7 @@ __global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass_label(const Pas
                     const uint32_t lo = (pc.y >> 8) & 255u, hi = pc.y >> 16;
                     for (uint32_t x = lo; x < hi; ++x) {
                         const uint32_t o = atomicCAS(&row[x], kNone, pc.x);
-                        if (o != kNone && o != kMulti) atomicExch(&row[x], kMulti);
+                        if (o != kNone && o < kBnd) atomicExch(&row[x], kMulti);   // BND / MULTI stay
                     }
                 }
                 consumers_sync();
@@ -179,14 +203,22 @@ __global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass_label(const Pas
             if (woff < ncopy && !never) {
                 Win<NS> w;
                 load_win_smem<NS>(w, ring + (size_t)st * ncol * kStagePts, woff + lane * kIPL);
-                process_lab<NS, FP>(a, sh, t, k, w, (m.sb - m.cb) - woff, m.se - m.sb, n_pass);
+                process_lab<ACC, NS, FP>(a, sh, t, k, w, (m.sb - m.cb) - woff, m.se - m.sb, qn, n_pass, n_bnd);
             }
+            if (ACC && (m.flags & 2u)) drain_queue<true>(a, sh, qn, true);
             __syncwarp();
             if (lane == 0) mbar_arrive(smem_u32(&rg.empty[st]));
             if (++st == nstage) { st = 0; ph ^= 1u; }
         }
-        for (int o = 16; o; o >>= 1) n_pass += __shfl_xor_sync(kFull, n_pass, o);
-        if (lane == 0) atomicAdd(&s_pass, n_pass);
+        if (ACC) drain_queue<true>(a, sh, qn, true);
+        for (int o = 16; o; o >>= 1) {
+            n_pass += __shfl_xor_sync(kFull, n_pass, o);
+            if (ACC) n_bnd += __shfl_xor_sync(kFull, n_bnd, o);
+        }
+        if (lane == 0) {
+            atomicAdd(&s_pass, n_pass);
+            if (ACC) atomicAdd(&s_bnd, n_bnd);
+        }
     }
     __syncthreads();
     if (a.smem_partials)
@@ -197,26 +229,29 @@ __global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass_label(const Pas
                 atomicAdd(&a.A_sum[kk], sh.psum[kk]);
             }
         }
-    if (threadIdx.x == 0) atomicAdd(&a.stats[0], (unsigned long long)s_pass);
-}
-
-template <bool FP>
-void *select_ns(int ns) {
-    switch (ns) {
-    case 0: return (void *)k_point_pass_label<0, FP>;
-    case 1: return (void *)k_point_pass_label<1, FP>;
-    case 2: return (void *)k_point_pass_label<2, FP>;
-    case 3: return (void *)k_point_pass_label<3, FP>;
-    case 4: return (void *)k_point_pass_label<4, FP>;
-    case 5: return (void *)k_point_pass_label<5, FP>;
-    default: return (void *)k_point_pass_label<6, FP>;
+    if (threadIdx.x == 0) {
+        atomicAdd(&a.stats[0], (unsigned long long)s_pass);
+        if (ACC) atomicAdd(&a.stats[1], (unsigned long long)s_bnd);
     }
 }
 
-size_t label_smem(const PassArgs &a, bool, bool) {
+template <bool ACC, bool FP>
+void *select_ns(int ns) {
+    switch (ns) {
+    case 0: return (void *)k_point_pass_label<ACC, 0, FP>;
+    case 1: return (void *)k_point_pass_label<ACC, 1, FP>;
+    case 2: return (void *)k_point_pass_label<ACC, 2, FP>;
+    case 3: return (void *)k_point_pass_label<ACC, 3, FP>;
+    case 4: return (void *)k_point_pass_label<ACC, 4, FP>;
+    case 5: return (void *)k_point_pass_label<ACC, 5, FP>;
+    default: return (void *)k_point_pass_label<ACC, 6, FP>;
+    }
+}
+
+size_t label_smem(const PassArgs &a, bool, bool accurate) {
     size_t b = ring_bytes(a.n_stages, a.f.n_slots) + (size_t)a.tile_cap * 2 * 4;
     if (a.smem_partials) b += (size_t)a.n_poly * 12;
-    return b;
+    return b + queue_bytes(accurate);
 }
 }  // namespace
 
@@ -226,7 +261,9 @@ rj_status point_pass_label(Ctx *c, const PassArgs &a_in, bool accurate) {
     PassArgs a = a_in;
     a.n_stages = (uint32_t)choose_stages(a, label_smem, true, accurate);
     if (!a.n_stages) return set_error(c, RJ_ERR_RESOLUTION, "point-pass tiles do not fit in shared memory");
-    void *k = a.f.n_fpred > 0 ? select_ns<true>(a.f.n_slots) : select_ns<false>(a.f.n_slots);
+    const bool fp = a.f.n_fpred > 0;
+    void *k = accurate ? (fp ? select_ns<true, true>(a.f.n_slots) : select_ns<true, false>(a.f.n_slots))
+                       : (fp ? select_ns<false, true>(a.f.n_slots) : select_ns<false, false>(a.f.n_slots));
     return launch_pass(c, k, a, label_smem(a, true, accurate));
 }
 

@@ -112,6 +112,7 @@ struct Ctx {
     uint32_t launches = 0;
     int last_stages = 0, last_ctas_per_sm = 0;   // point-pass launch shape of the last query
     int force_tile_pass = 0;                      // RJ_OPT_PASS = 1: always the pixel-tile kernel
+    int tile_side = 32;                           // RJ_OPT_TILE_SIDE: target point-cell side in pixels
 };
 
 // workspace slot map (Ctx::ws)
@@ -143,7 +144,7 @@ rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int
 rj_status items_for_level(Ctx *c, int L);
 void free_load_scratch(Ctx *c);
 void drop_items(Ctx *c);
-int choose_level(int W, int H, bool sum);
+int choose_level(int W, int H, int target_side);
 
 // polygons.cu
 rj_status load_polygons_impl(Ctx *c, uint32_t n_poly, const uint32_t *pro, const uint32_t *rvo,

@@ -12,9 +12,8 @@
 
 namespace rj {
 
-int choose_level(int W, int H, bool sum) {
-    (void)sum;
-    const int target = 32;                     // tile side in pixels
+int choose_level(int W, int H, int target) {
+    // smallest L whose cells span <= target pixels a side (capped at level 10)
     const int side = std::max(W, H);
     int L = 0;
     while (L < kMaxLevel && (side + (1 << L) - 1) / (1 << L) > target) ++L;

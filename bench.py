@@ -360,7 +360,10 @@ def main():
             "gpu_launches": int(st["launches"]) * args.steps,
             "cpu_baseline": cpu,
             "checks": {"tiling_sum_equals_filtered": tiling_ok, "n_filtered": st["n_filtered"],
-                       "n_out_of_domain": int(n_ood)},
+                       "n_out_of_domain": int(n_ood), "n_boundary": st["n_boundary"]},
+            "launch": {"cell_level": st["level"], "ring_stages": st["pass_stages"],
+                       "ctas_per_sm": st["pass_ctas_per_sm"], "work_items": st["n_items"],
+                       "pieces": st["n_pieces"], "crossings": st["n_crossings"]},
             "host": {"gen_s": t_gen, "load_s": t_load},
         }
         print(json.dumps(line), flush=True)

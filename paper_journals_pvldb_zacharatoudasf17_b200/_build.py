@@ -45,7 +45,10 @@ def build(force=False, verbose=False):
 
     def cc(src):
         obj = os.path.join(OBJ, os.path.basename(src) + ".o")
-        cmd = [NVCC, *FLAGS, *extra, "-c", src, "-o", obj]
+        # point-pass kernels: 9 warps per CTA, two CTAs per SM -> an SM
+        # sub-partition holds 5 warps, i.e. at most 96 registers per thread
+        per_file = ["-maxrregcount=96"] if os.path.basename(src).startswith("pass") else []
+        cmd = [NVCC, *FLAGS, *per_file, *extra, "-c", src, "-o", obj]
         r = subprocess.run(cmd, capture_output=True, text=True)
         if r.returncode != 0:
             raise RuntimeError(f"nvcc failed for {src}:\n{r.stdout}\n{r.stderr}")

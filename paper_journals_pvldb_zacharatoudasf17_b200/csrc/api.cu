@@ -216,18 +216,31 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     if ((s = build_filter(c, q, f)) != RJ_OK) return s;
     P.sum = q->agg != RJ_COUNT;
     P.acc = q->mode == RJ_ACCURATE;
+    PassArgs &a = P.a;
+    memset(&a, 0, sizeof(a));
+    a.f = f;
+    a.n_poly = c->n_poly;
+    // cell level: tiles of ~tile_side pixels, refined while two CTAs with a
+    // two-stage ring would not fit in shared memory; per-CTA polygon partials
+    // in shared memory unless they crowd out the ring
     P.L = choose_level(P.W, P.H, c->tile_side);
+    for (;;) {
+        tile_geometry(P.W, P.H, P.L, a.tile_stride, a.tile_cap);
+        a.n_stages = 2;
+        a.smem_partials = 1;
+        if (point_pass_smem(c, a, P.sum, P.acc) > 160 * 1024) a.smem_partials = 0;
+        if (point_pass_smem(c, a, P.sum, P.acc) + 3 * 1024 <= 112 * 1024 || P.L >= kMaxLevel) break;
+        ++P.L;
+    }
+    a.n_stages = (uint32_t)point_pass_stages(f.n_slots);
     if ((s = items_for_level(c, P.L)) != RJ_OK) return s;
     c->launches = 0;
     if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[0], c->stream));
     if (need_polygon_pass && (s = polygon_pass(c, P.W, P.H, P.L, P.acc, P.pp)) != RJ_OK) return s;
     if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[1], c->stream));
-    PassArgs &a = P.a;
-    memset(&a, 0, sizeof(a));
     a.qx = c->qx.as<uint32_t>();
     a.qy = c->qy.as<uint32_t>();
     for (int k = 0; k < f.n_slots; ++k) a.col[k] = c->col[f.slot_col[k]].as<uint32_t>();
-    a.f = f;
     a.W = P.W;
     a.H = P.H;
     a.items = c->items[P.L].as<int4>();
@@ -240,13 +253,10 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     a.mask_wpr = P.pp.mask_wpr;
     a.grid_off = c->grid_off.as<uint32_t>();
     a.grid_ent = c->grid_ent.as<uint32_t>();
+    a.grid_edge = c->grid_edge.as<int4>();
+    a.grid_poly = c->grid_poly.as<uint32_t>();
     a.edges = c->edges.as<int4>();
     a.edge_poly = c->edge_poly.as<uint32_t>();
-    a.n_poly = c->n_poly;
-    tile_geometry(P.W, P.H, P.L, a.tile_stride, a.tile_cap);
-    a.n_stages = (uint32_t)point_pass_stages(f.n_slots);
-    a.smem_partials = 1;
-    if (point_pass_smem(a, P.sum, P.acc) > 160 * 1024) a.smem_partials = 0;
     Buf &st = wsbuf(c, kWsWork);
     if (dreserve(c, st, 64)) return set_error(c, RJ_ERR_OOM, "workspace allocation failed");
     a.work_counter = st.as<uint32_t>();
@@ -359,7 +369,7 @@ rj_status rj_destroy(rj_ctx *c) {
     free_load_scratch(c);
     dfree(c, c->cell_off); drop_items(c);
     dfree(c, c->edges); dfree(c, c->edge_poly); dfree(c, c->poly_edge_off); dfree(c, c->mbr);
-    dfree(c, c->grid_off); dfree(c, c->grid_ent);
+    dfree(c, c->grid_off); dfree(c, c->grid_ent); dfree(c, c->grid_edge); dfree(c, c->grid_poly);
     for (auto &b : c->ws) dfree(c, b);
     dfree(c, c->res_cnt); dfree(c, c->res_sum); dfree(c, c->res_val);
     for (auto &e : c->ev) if (e) cudaEventDestroy(e);
@@ -382,8 +392,8 @@ rj_status rj_set_option(rj_ctx *c, int32_t option, int64_t value) {
     if (!c) return RJ_ERR_INVALID_ARGUMENT;
     if (option == RJ_OPT_TIMING) { c->timing = value ? 1 : 0; return RJ_OK; }
     if (option == RJ_OPT_PASS) {
-        if (value < 0 || value > 1) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "RJ_OPT_PASS must be 0 or 1");
-        c->force_tile_pass = (int)value;
+        if (value < -1 || value > 1) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "RJ_OPT_PASS must be -1, 0 or 1");
+        c->pass_variant = (int)value;
         return RJ_OK;
     }
     if (option == RJ_OPT_TILE_SIDE) {

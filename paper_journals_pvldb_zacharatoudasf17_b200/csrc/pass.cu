@@ -126,22 +126,21 @@ __device__ __forceinline__ void process(const PassArgs &a, const Shared &sh, con
 }
 
 template <bool SUM, bool ACC, int NS, bool FP>
-__global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass(const PassArgs a) {
+__global__ void __maxnreg__(96) k_point_pass(const PassArgs a) {
     extern __shared__ __align__(128) unsigned char smem_raw[];
     __shared__ __align__(8) Ring rg;
     __shared__ uint32_t s_pass, s_bnd;
     const int lane = threadIdx.x & 31, wid = threadIdx.x >> 5;
     const uint32_t nstage = a.n_stages;
     const int ncol = 2 + NS;
-    // carve: [ring][tile sums f64 x2][partial sums f64][tile counts u32 x2][partial counts u32][queues]
+    // carve: [ring][tile sums f64 x2][tile counts u32 x2][partial counts u32][queues]
     unsigned char *p = smem_raw;
     uint32_t *ring = reinterpret_cast<uint32_t *>(p);
     p += ring_bytes(nstage, NS);
     double *tsum = reinterpret_cast<double *>(p);
     if (SUM) p += sizeof(double) * a.tile_cap * 2;
     Shared sh;
-    sh.psum = reinterpret_cast<double *>(p);
-    if (SUM && a.smem_partials) p += sizeof(double) * a.n_poly;
+    sh.psum = nullptr;                                      // fp64 sums reduce in global memory
     uint32_t *tcnt = reinterpret_cast<uint32_t *>(p);
     p += sizeof(uint32_t) * a.tile_cap * 2;
     sh.pcnt = reinterpret_cast<uint32_t *>(p);
@@ -159,7 +158,6 @@ __global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass(const PassArgs 
     if (a.smem_partials)
         for (uint32_t kk = threadIdx.x; kk < a.n_poly; kk += blockDim.x) {
             sh.pcnt[kk] = 0;
-            if (SUM) sh.psum[kk] = 0.0;
         }
     __syncthreads();
 
@@ -260,10 +258,7 @@ __global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass(const PassArgs 
     if (a.smem_partials)
         for (uint32_t kk = threadIdx.x; kk < a.n_poly; kk += blockDim.x) {
             const uint32_t cc = sh.pcnt[kk];
-            if (cc) {
-                atomicAdd(&a.A_cnt[kk], (unsigned long long)cc);
-                if (SUM) atomicAdd(&a.A_sum[kk], sh.psum[kk]);
-            }
+            if (cc) atomicAdd(&a.A_cnt[kk], (unsigned long long)cc);
         }
     if (threadIdx.x == 0) {
         atomicAdd(&a.stats[0], (unsigned long long)s_pass);
@@ -296,7 +291,7 @@ void *select_kernel(bool sum, bool acc, int ns, bool fp) {
 size_t tile_pass_smem(const PassArgs &a, bool sum, bool accurate) {
     size_t b = ring_bytes(a.n_stages, a.f.n_slots);
     b += (size_t)a.tile_cap * 2 * (4 + (sum ? 8 : 0));
-    if (a.smem_partials) b += (size_t)a.n_poly * (4 + (sum ? 8 : 0));
+    if (a.smem_partials) b += (size_t)a.n_poly * 4;
     return b + queue_bytes(accurate);
 }
 }  // namespace
@@ -332,16 +327,23 @@ rj_status launch_pass(Ctx *c, void *k, const PassArgs &a, size_t smem) {
     return RJ_OK;
 }
 
-size_t point_pass_smem(const PassArgs &a, bool sum, bool accurate) {
-    return sum ? point_pass_label_smem(a, accurate) : tile_pass_smem(a, sum, accurate);
+// Kernel choice: COUNT always uses the pixel tile (cheapest per cell); SUM/AVG
+// uses polygon labels in bounded mode (no per-pixel fp64 atomics) and the
+// pixel tile in accurate mode (measured faster at C3); RJ_OPT_PASS overrides.
+static bool use_label(const Ctx *c, bool sum, bool accurate) {
+    if (!sum) return false;
+    if (c->pass_variant >= 0) return c->pass_variant == 0;
+    return !accurate;
+}
+
+size_t point_pass_smem(const Ctx *c, const PassArgs &a, bool sum, bool accurate) {
+    return use_label(c, sum, accurate) ? point_pass_label_smem(a, accurate) : tile_pass_smem(a, sum, accurate);
 }
 
 int point_pass_stages(int n_slots) { return (2 + n_slots) <= 4 ? 3 : 2; }
 
 rj_status point_pass(Ctx *c, const PassArgs &a_in, bool sum, bool accurate) {
-    // SUM/AVG: per-pixel fp64 sums would need shared CAS loops; the label
-    // kernel sums per polygon run instead
-    if (sum && !c->force_tile_pass) return point_pass_label(c, a_in, accurate);
+    if (use_label(c, sum, accurate)) return point_pass_label(c, a_in, accurate);
     PassArgs a = a_in;
     a.n_stages = (uint32_t)choose_stages(a, tile_pass_smem, sum, accurate);
     if (!a.n_stages) return set_error(c, RJ_ERR_RESOLUTION, "point-pass tiles do not fit in shared memory");

@@ -85,57 +85,85 @@ struct Shared {
     uint32_t *qx, *qy, *qa;  // this warp's boundary queue [kQ]
 };
 
+// Add (cnt, s) to polygon P's partials.  Counts go to the CTA's shared
+// partials (native shared atomics); fp64 sums go straight to the global
+// result with native L2 reductions (red.global.add.f64) -- a shared fp64
+// atomic is a CAS loop, and polygons are hot spots shared by many warps.
 template <bool SUM>
 __device__ __forceinline__ void emit_poly(const PassArgs &a, const Shared &sh, uint32_t P, uint32_t cnt, double s) {
-    if (a.smem_partials) {
-        atomicAdd(&sh.pcnt[P], cnt);
-        if (SUM) atomicAdd(&sh.psum[P], s);
-    } else {
-        atomicAdd(&a.A_cnt[P], (unsigned long long)cnt);
-        if (SUM) atomicAdd(&a.A_sum[P], s);
-    }
+    if (a.smem_partials) atomicAdd(&sh.pcnt[P], cnt);
+    else atomicAdd(&a.A_cnt[P], (unsigned long long)cnt);
+    if (SUM) atomicAdd(&a.A_sum[P], s);
 }
 
 // Proc. JoinPoint: exact even-odd test of lattice point (px, py)
-// against every polygon through the edge-grid cell; each containing polygon
-// gets (1, v).  Cell entries are sorted by edge id, so they group by polygon.
+// against every polygon through the edge-grid cell.  Cell entries are sorted
+// by edge id, so they group by polygon.  Returns the first containing polygon
+// (kNoPoly if none); any further containing polygons (overlaps) get (1, v)
+// directly.
 template <bool SUM>
-__device__ __forceinline__ void join_point(const PassArgs &a, const Shared &sh, uint32_t px, uint32_t py, double v) {
+__device__ __forceinline__ uint32_t join_point(const PassArgs &a, const Shared &sh, uint32_t px, uint32_t py,
+                                               double v) {
     const uint32_t cell = (py >> kGridShift) * kGrid + (px >> kGridShift);
     const uint32_t b = __ldg(&a.grid_off[cell]), e = __ldg(&a.grid_off[cell + 1]);
-    uint32_t cur = kNoPoly, par = 0;
+    uint32_t cur = kNoPoly, par = 0, first = kNoPoly;
     const int64_t X = px, Y = py;
     for (uint32_t k = b; k < e; ++k) {
-        const uint32_t ed = __ldg(&a.grid_ent[k]);
-        const uint32_t P = __ldg(&a.edge_poly[ed]);
+        const uint32_t P = __ldg(&a.grid_poly[k]);
+        const int4 E = __ldg(&a.grid_edge[k]);
         if (P != cur) {
-            if (par) emit_poly<SUM>(a, sh, cur, 1u, v);
+            if (par) {
+                if (first == kNoPoly) first = cur;
+                else emit_poly<SUM>(a, sh, cur, 1u, v);
+            }
             cur = P;
             par = 0;
         }
-        const int4 E = __ldg(&a.edges[ed]);
         if ((E.y > (int)py) != (E.w > (int)py)) {
             const int64_t lhs = (X - E.x) * (int64_t)(E.w - E.y);
             const int64_t rhs = (int64_t)(E.z - E.x) * (Y - E.y);
             if (E.w > E.y ? lhs < rhs : lhs > rhs) par ^= 1u;
         }
     }
-    if (par) emit_poly<SUM>(a, sh, cur, 1u, v);
+    if (par) {
+        if (first == kNoPoly) first = cur;
+        else emit_poly<SUM>(a, sh, cur, 1u, v);
+    }
+    return first;
 }
 
+// Test the queued boundary points, 32 at a time (one per lane), and add
+// the results with one atomic per distinct polygon of the batch (neighbouring
+// boundary points mostly fall in the same polygon).  Kept out of line: it is
+// the rare path, and inlining it per point would bloat the window loop past
+// the instruction cache.
 template <bool SUM>
-__device__ __forceinline__ void drain_queue(const PassArgs &a, const Shared &sh, uint32_t &qn, bool all) {
+__device__ __noinline__ void drain_queue(const PassArgs &a, const Shared &sh, uint32_t &qn, bool all) {
     const int lane = threadIdx.x & 31;
     while (qn >= 32 || (all && qn > 0)) {
         __syncwarp();
         const uint32_t take = qn >= 32 ? 32u : qn;
+        uint32_t P = kNoPoly;
+        double v = 0.0;
         if ((uint32_t)lane < take) {
             const uint32_t pos = qn - take + lane;
             const uint32_t x = sh.qx[pos], y = sh.qy[pos], ab = sh.qa[pos];
-            join_point<SUM>(a, sh, x, y, SUM ? attr_val(ab, a.f.agg_is_float) : 0.0);
+            v = SUM ? attr_val(ab, a.f.agg_is_float) : 0.0;
+            P = join_point<SUM>(a, sh, x, y, v);
         }
         __syncwarp();
         qn -= take;
+        unsigned active = __ballot_sync(kFull, P != kNoPoly);
+        while (active) {
+            const int leader = __ffs(active) - 1;
+            const uint32_t PL = __shfl_sync(kFull, P, leader);
+            const unsigned m = __ballot_sync(kFull, P == PL);
+            double s = (SUM && P == PL) ? v : 0.0;
+            if (SUM)
+                for (int o = 16; o; o >>= 1) s += __shfl_xor_sync(kFull, s, o);
+            if (lane == leader) emit_poly<SUM>(a, sh, PL, __popc(m), s);
+            active &= ~m;
+        }
     }
 }
 

@@ -40,7 +40,7 @@ __device__ __forceinline__ void emit_lab_run(const PassArgs &a, const Shared &sh
 }
 
 // Points whose pixel several polygons cover: look up every covering piece.
-__device__ __forceinline__ void multi_point(const PassArgs &a, const Shared &sh, const LabTile &t, uint32_t px,
+__device__ __noinline__ void multi_point(const PassArgs &a, const Shared &sh, const LabTile &t, uint32_t px,
                                             uint32_t py, double v) {
     const uint32_t lx = px - t.c0, ly = py - t.r0;
     for (uint32_t k = t.pb; k < t.pe; ++k) {
@@ -50,10 +50,16 @@ __device__ __forceinline__ void multi_point(const PassArgs &a, const Shared &sh,
     }
 }
 
+// Warp-uniform run carried from window to window: (label, count, sum).
+struct Carry {
+    uint32_t lab = kNone, cnt = 0;
+    double sum = 0.0;
+};
+
 template <bool ACC, int NS, bool FP>
 __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh, const LabTile &t,
                                             const Consts<NS> &k, const Win<NS> &w, uint32_t first, uint32_t count,
-                                            uint32_t &qn, uint32_t &n_pass, uint32_t &n_bnd) {
+                                            Carry &cy, uint32_t &qn, uint32_t &n_pass, uint32_t &n_bnd) {
     const int lane = threadIdx.x & 31;
     uint32_t lab[kIPL];
     bool spec = false;
@@ -78,10 +84,16 @@ __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh,
             if (lab[j] >= kBnd) lab[j] = kNone;
         }
     }
-    const uint32_t kprev = __shfl_up_sync(kFull, lab[kIPL - 1], 1);
+    // Runs of equal labels: inside the lane in registers, across lanes by a
+    // segmented scan, and across windows through the warp's carry (Morton
+    // order keeps a warp inside one polygon for long stretches, so a
+    // polygon's partial is typically emitted once per stretch, not per window).
+    uint32_t kprev = __shfl_up_sync(kFull, lab[kIPL - 1], 1);
+    if (lane == 0) kprev = cy.lab;
     const uint32_t knext = __shfl_down_sync(kFull, lab[0], 1);
-    const bool cin = lane > 0 && lab[0] == kprev;
-    const bool cout = lane < 31 && lab[kIPL - 1] == knext;
+    const bool cin = lab[0] == kprev;                       // first run continues from before
+    const bool cout = lane == 31 || lab[kIPL - 1] == knext; // last run continues (lane 31: into the carry)
+    if (lane == 0 && !cin) emit_lab_run(a, sh, cy.lab, cy.cnt, cy.sum, true);   // carry ends here
     uint32_t run = 0, fcnt = 0, flab = kNone;
     double dsum = 0.0, fsum = 0.0;
     bool seen = false;
@@ -102,29 +114,39 @@ __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh,
         run += 1u;
         dsum += attr_val(agg_bits<NS>(a, w, kIPL - 1), a.f.agg_is_float);
     }
+    // lane 0 takes the carry as its incoming partial
+    const bool lane0_in = lane == 0 && cin;
+    uint32_t scan_run = run + ((lane0_in && !seen) ? cy.cnt : 0u);
+    double scan_sum = dsum + ((lane0_in && !seen) ? cy.sum : 0.0);
     uint32_t pre;
     double dpre;
-    run_carry<true>(run, dsum, seen || !cin, pre, dpre);
+    run_carry<true>(scan_run, scan_sum, seen || !cin || lane == 0, pre, dpre);
+    if (lane == 0) { pre = cin ? cy.cnt : 0u; dpre = cin ? cy.sum : 0.0; }
     if (cin && seen) emit_lab_run(a, sh, flab, fcnt + pre, fsum + dpre, true);
     const bool add_pre = cin && !seen;
-    emit_lab_run(a, sh, lab[kIPL - 1], run + (add_pre ? pre : 0u), dsum + (add_pre ? dpre : 0.0), !cout);
+    const uint32_t last_cnt = (lane == 0) ? scan_run : run + (add_pre ? pre : 0u);
+    const double last_sum = (lane == 0) ? scan_sum : dsum + (add_pre ? dpre : 0.0);
+    emit_lab_run(a, sh, lab[kIPL - 1], last_cnt, last_sum, !cout);
+    // the window's last run becomes the carry
+    cy.lab = __shfl_sync(kFull, lab[kIPL - 1], 31);
+    cy.cnt = __shfl_sync(kFull, last_cnt, 31);
+    cy.sum = __shfl_sync(kFull, last_sum, 31);
 }
 
 template <bool ACC, int NS, bool FP>
-__global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass_label(const PassArgs a) {
+__global__ void __maxnreg__(96) k_point_pass_label(const PassArgs a) {
     extern __shared__ __align__(128) unsigned char smem_raw[];
     __shared__ __align__(8) Ring rg;
     __shared__ uint32_t s_pass, s_bnd;
     const int lane = threadIdx.x & 31, wid = threadIdx.x >> 5;
     const uint32_t nstage = a.n_stages;
     const int ncol = 2 + NS;
-    // carve: [ring][partial sums f64][label tiles u32 x2][partial counts u32][queues]
+    // carve: [ring][label tiles u32 x2][partial counts u32][queues]
     unsigned char *p = smem_raw;
     uint32_t *ring = reinterpret_cast<uint32_t *>(p);
     p += ring_bytes(nstage, NS);
     Shared sh;
-    sh.psum = reinterpret_cast<double *>(p);
-    if (a.smem_partials) p += sizeof(double) * a.n_poly;
+    sh.psum = nullptr;                                      // fp64 sums reduce in global memory
     uint32_t *labels = reinterpret_cast<uint32_t *>(p);
     p += sizeof(uint32_t) * a.tile_cap * 2;
     sh.pcnt = reinterpret_cast<uint32_t *>(p);
@@ -142,7 +164,6 @@ __global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass_label(const Pas
     if (a.smem_partials)
         for (uint32_t kk = threadIdx.x; kk < a.n_poly; kk += blockDim.x) {
             sh.pcnt[kk] = 0;
-            sh.psum[kk] = 0.0;
         }
     __syncthreads();
 
@@ -155,6 +176,7 @@ __global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass_label(const Pas
         LabTile t;
         t.stride = a.tile_stride;
         uint32_t tsel = 0, n_pass = 0, n_bnd = 0, qn = 0;
+        Carry cy;
         uint32_t st = 0, ph = 0;
         for (;;) {
             mbar_wait(smem_u32(&rg.full[st]), ph);
@@ -203,7 +225,7 @@ __global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass_label(const Pas
             if (woff < ncopy && !never) {
                 Win<NS> w;
                 load_win_smem<NS>(w, ring + (size_t)st * ncol * kStagePts, woff + lane * kIPL);
-                process_lab<ACC, NS, FP>(a, sh, t, k, w, (m.sb - m.cb) - woff, m.se - m.sb, qn, n_pass, n_bnd);
+                process_lab<ACC, NS, FP>(a, sh, t, k, w, (m.sb - m.cb) - woff, m.se - m.sb, cy, qn, n_pass, n_bnd);
             }
             if (ACC && (m.flags & 2u)) drain_queue<true>(a, sh, qn, true);
             __syncwarp();
@@ -211,6 +233,7 @@ __global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass_label(const Pas
             if (++st == nstage) { st = 0; ph ^= 1u; }
         }
         if (ACC) drain_queue<true>(a, sh, qn, true);
+        if (lane == 0) emit_lab_run(a, sh, cy.lab, cy.cnt, cy.sum, true);
         for (int o = 16; o; o >>= 1) {
             n_pass += __shfl_xor_sync(kFull, n_pass, o);
             if (ACC) n_bnd += __shfl_xor_sync(kFull, n_bnd, o);
@@ -224,10 +247,7 @@ __global__ void __launch_bounds__(kThreads + 32, 1) k_point_pass_label(const Pas
     if (a.smem_partials)
         for (uint32_t kk = threadIdx.x; kk < a.n_poly; kk += blockDim.x) {
             const uint32_t cc = sh.pcnt[kk];
-            if (cc) {
-                atomicAdd(&a.A_cnt[kk], (unsigned long long)cc);
-                atomicAdd(&a.A_sum[kk], sh.psum[kk]);
-            }
+            if (cc) atomicAdd(&a.A_cnt[kk], (unsigned long long)cc);
         }
     if (threadIdx.x == 0) {
         atomicAdd(&a.stats[0], (unsigned long long)s_pass);
@@ -250,7 +270,7 @@ void *select_ns(int ns) {
 
 size_t label_smem(const PassArgs &a, bool, bool accurate) {
     size_t b = ring_bytes(a.n_stages, a.f.n_slots) + (size_t)a.tile_cap * 2 * 4;
-    if (a.smem_partials) b += (size_t)a.n_poly * 12;
+    if (a.smem_partials) b += (size_t)a.n_poly * 4;
     return b + queue_bytes(accurate);
 }
 }  // namespace

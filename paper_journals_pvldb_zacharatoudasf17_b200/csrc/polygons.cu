@@ -66,6 +66,19 @@ __global__ void k_grid_edges(const int4 *__restrict__ edges, const uint32_t *__r
         }
 }
 
+// Entries inlined for the accurate-mode test: the edge's endpoints and its
+// polygon next to each other, so a boundary point reads one 16-B record and
+// one id per entry instead of chasing entry -> edge -> polygon.
+__global__ void k_grid_inline(const uint32_t *__restrict__ ent, uint32_t n, const int4 *__restrict__ edges,
+                              const uint32_t *__restrict__ edge_poly, int4 *__restrict__ gedge,
+                              uint32_t *__restrict__ gpoly) {
+    const uint32_t i = blockIdx.x * blockDim.x + threadIdx.x;
+    if (i >= n) return;
+    const uint32_t e = ent[i];
+    gedge[i] = edges[e];
+    gpoly[i] = edge_poly[e];
+}
+
 __global__ void k_grid_sort(const uint32_t *__restrict__ off, uint32_t *__restrict__ ent) {
     const uint32_t c = blockIdx.x * blockDim.x + threadIdx.x;
     if (c >= (uint32_t)kGrid * kGrid) return;
@@ -339,6 +352,18 @@ rj_status load_polygons_impl(Ctx *c, uint32_t n_poly, const uint32_t *pro, const
     k_grid_sort<<<blocks_for(ncell, 256), 256, 0, c->stream>>>(c->grid_off.as<uint32_t>(), c->grid_ent.as<uint32_t>());
     RJ_LAUNCHED(c);
     RJ_CUDA(c, cudaGetLastError());
+    dfree(c, c->grid_edge);
+    dfree(c, c->grid_poly);
+    if (dalloc(c, c->grid_edge, std::max<uint64_t>(1, n_ent) * sizeof(int4)) ||
+        dalloc(c, c->grid_poly, std::max<uint64_t>(1, n_ent) * 4))
+        return set_error(c, RJ_ERR_OOM, "edge grid allocation failed");
+    if (n_ent) {
+        k_grid_inline<<<blocks_for(n_ent, 256), 256, 0, c->stream>>>(
+            c->grid_ent.as<uint32_t>(), n_ent, c->edges.as<int4>(), c->edge_poly.as<uint32_t>(),
+            c->grid_edge.as<int4>(), c->grid_poly.as<uint32_t>());
+        RJ_LAUNCHED(c);
+        RJ_CUDA(c, cudaGetLastError());
+    }
     RJ_CUDA(c, cudaStreamSynchronize(c->stream));
     dfree(c, cnt);
     dfree(c, cur);

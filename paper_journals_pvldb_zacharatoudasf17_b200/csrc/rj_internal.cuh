@@ -56,6 +56,8 @@ struct PassArgs {
     uint32_t mask_wpr;
     const uint32_t *grid_off;     // accurate: edge grid CSR
     const uint32_t *grid_ent;
+    const int4 *grid_edge;        // per entry: (xa, ya, xb, yb)
+    const uint32_t *grid_poly;    // per entry: polygon
     const int4 *edges;
     const uint32_t *edge_poly;
     unsigned long long *A_cnt;    // per polygon partials (device)
@@ -100,6 +102,7 @@ struct Ctx {
     uint32_t n_edges = 0;
     Buf edges, edge_poly, poly_edge_off, mbr;   // int4 edges/mbr
     Buf grid_off, grid_ent;
+    Buf grid_edge, grid_poly;                  // entries inlined: edge endpoints + polygon
     uint64_t n_grid_ent = 0;
 
     // query workspace (grow-only)
@@ -111,8 +114,8 @@ struct Ctx {
     cudaEvent_t ev[6] = {};
     uint32_t launches = 0;
     int last_stages = 0, last_ctas_per_sm = 0;   // point-pass launch shape of the last query
-    int force_tile_pass = 0;                      // RJ_OPT_PASS = 1: always the pixel-tile kernel
-    int tile_side = 32;                           // RJ_OPT_TILE_SIDE: target point-cell side in pixels
+    int pass_variant = -1;                        // RJ_OPT_PASS: -1 auto, 0 label, 1 pixel tile
+    int tile_side = 64;                           // RJ_OPT_TILE_SIDE: target point-cell side in pixels
 };
 
 // workspace slot map (Ctx::ws)
@@ -161,7 +164,7 @@ rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp)
 
 // pass.cu
 rj_status point_pass(Ctx *c, const PassArgs &a, bool sum, bool accurate);
-size_t point_pass_smem(const PassArgs &a, bool sum, bool accurate);
+size_t point_pass_smem(const Ctx *c, const PassArgs &a, bool sum, bool accurate);
 int point_pass_stages(int n_slots);
 
 // misc.cu

@@ -134,7 +134,8 @@ def test_point_membership_bitexact(c1, mode, W):
     assert np.array_equal(g, o)
 
 
-@pytest.mark.parametrize("mode,variant", [("bounded", 0), ("bounded", 1), ("accurate", 0), ("accurate", 1)])
+@pytest.mark.parametrize("mode,variant", [("bounded", 0), ("bounded", 1), ("accurate", 0), ("accurate", 1),
+                                          ("bounded", -1), ("accurate", -1)])
 def test_sum_avg_filters(c1, mode, variant):
     """Both point-pass kernels (label: default for bounded SUM/AVG; tile:
     RJ_OPT_PASS = 1) against the oracle."""

@@ -46,6 +46,9 @@ def query_sharded(R: "rj.RasterJoin", desc, d_count: torch.Tensor, d_sum: torch.
     R's stream must be torch's current stream (create R with
     stream=torch.cuda.current_stream().cuda_stream) so NCCL orders after it."""
     rj.rj_query_device(R.ctx, desc, d_count, d_sum)
+    if dist.get_backend(group) == "gloo":
+        # gloo stages device tensors through the host outside the stream order
+        torch.cuda.current_stream().synchronize()
     allreduce_partials(d_count, d_sum if desc.agg != 0 else None, group)
     rj.rj_finalize_device(R.ctx, desc.agg, d_count, d_sum, d_value)
     return d_value

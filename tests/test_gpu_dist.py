@@ -28,6 +28,15 @@ N = 300_001
 
 
 def _worker(rank, world, port, q):
+    try:
+        _run(rank, world, port, q)
+    except BaseException as e:          # report, do not hang the parent
+        import traceback
+        q.put(("error", rank, traceback.format_exc()))
+        raise
+
+
+def _run(rank, world, port, q):
     os.environ["MASTER_ADDR"] = "127.0.0.1"
     os.environ["MASTER_PORT"] = str(port)
     dist.init_process_group("gloo", rank=rank, world_size=world)
@@ -55,7 +64,7 @@ def _worker(rank, world, port, q):
             out[mode] = (d_cnt.cpu().numpy(), d_val.cpu().numpy())
         R.close()
         if rank == 0:
-            q.put(out)
+            q.put(("ok", rank, out))
     finally:
         dist.destroy_process_group()
 
@@ -72,10 +81,11 @@ def test_sharded_query_allreduce_on_one_gpu():
     procs = [ctx.Process(target=_worker, args=(r, 2, port, q)) for r in range(2)]
     for p in procs:
         p.start()
-    got = q.get(timeout=600)
+    status, rank, got = q.get(timeout=600)
+    assert status == "ok", f"rank {rank} failed:\n{got}"
     for p in procs:
         p.join(timeout=120)
-        assert p.exitcode == 0
+        assert p.exitcode == 0, p.exitcode
     pts = C.taxi(N, fare=True)
     P = oracle.Polys(C.array_polys("neighborhoods"), C.NYC_BOX)
     for mode in ("bounded", "accurate"):

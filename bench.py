@@ -204,6 +204,7 @@ def main():
     ap.add_argument("--chunk", type=int, default=0, help="points per work item (0 = library default)")
     ap.add_argument("--tile", type=int, default=0, help="point-cell side in pixels (0 = library default)")
     ap.add_argument("--pass-variant", type=int, default=-1, help="SUM/AVG kernel: 0 label, 1 pixel tile")
+    ap.add_argument("--mode", default="", help="override the config's mode: bounded|accurate|index|exact")
     args = ap.parse_args()
     args.warmup = max(3, args.warmup)
 
@@ -223,6 +224,9 @@ def main():
     if world > 1:
         dist.init_process_group("nccl", device_id=torch.device("cuda", local))
     box, polys_name, recipe, q, desc = workload(args.config)
+    if args.mode:
+        q = dict(q, mode=args.mode)
+        desc += f" [mode={args.mode}]"
 
     if args.scaling == "weak":
         n_local, i0 = args.points, rank * args.points

@@ -117,7 +117,7 @@ static rj_status build_filter(Ctx *c, const rj_query_desc *q, Filter &f) {
     f = Filter{};
     if (q->n_pred < 0 || q->n_pred > RJ_MAX_PRED) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "n_pred must be in [0, 5]");
     if (q->agg < RJ_COUNT || q->agg > RJ_AVG) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad agg");
-    if (q->mode != RJ_BOUNDED && q->mode != RJ_ACCURATE) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad mode");
+    if (q->mode < RJ_BOUNDED || q->mode > RJ_EXACT) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad mode");
     for (int k = 0; k < q->n_pred; ++k) {
         const rj_pred &p = q->pred[k];
         if (p.column < 0 || p.column >= c->n_cols) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "predicate column out of range");
@@ -189,9 +189,38 @@ static void tile_geometry(int W, int H, int L, uint32_t &stride, uint32_t &cap) 
     cap = (uint32_t)(mh * stride);
 }
 
+// Exact-mode chooser (RJ_EXACT).  Both exact variants
+// stream every point once; they differ in the PIP tests and the polygon pass:
+//   accurate:   T_poly + f * N * c_pip      index join:  N * c_pip
+// f = estimated boundary-pixel fraction: each edge's supercover touches
+// about |dx| W + |dy| H (lattice units / 2^30) + 1 pixels.  T_poly is the
+// polygon pass (launch floor + crossings + boundary mask), measured on B200
+// (profiles/r1_chooser.md).
+struct ChooserModel {
+    double t_floor_us = 60.0;      // polygon-pass launch / sync floor
+    double t_cross_ns = 0.02;      // per (edge, row) crossing
+    double t_mask_ns = 0.004;      // per boundary-mask pixel
+    double c_pip_ns = 0.16;        // per point routed through the edge grid
+};
+
+static float boundary_fraction(const Ctx *c, int W, int H) {
+    const double px = (double)W * H;
+    const double b = (c->edge_len_x * W + c->edge_len_y * H) / 1073741824.0 + (double)c->n_edges;
+    return (float)std::min(1.0, b / px);
+}
+
+static int choose_exact(const Ctx *c, int W, int H, float f) {
+    const ChooserModel m;
+    const double cross = c->edge_len_y * H / 1073741824.0 + (double)c->n_edges;
+    const double t_poly = m.t_floor_us * 1e3 + m.t_cross_ns * cross + m.t_mask_ns * (double)W * H;
+    const double saved = (1.0 - f) * (double)c->n_pts * m.c_pip_ns;
+    return t_poly > saved ? RJ_INDEX_JOIN : RJ_ACCURATE;
+}
+
 struct Prepared {
     int W, H, L;
-    bool sum, acc;
+    int mode;                      // executed rj_mode (RJ_EXACT resolved)
+    bool sum, acc, index;
     PolyPass pp;
     PassArgs a;
 };
@@ -215,7 +244,12 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     Filter f;
     if ((s = build_filter(c, q, f)) != RJ_OK) return s;
     P.sum = q->agg != RJ_COUNT;
-    P.acc = q->mode == RJ_ACCURATE;
+    const float f_bnd = boundary_fraction(c, P.W, P.H);
+    P.mode = q->mode == RJ_EXACT ? choose_exact(c, P.W, P.H, f_bnd) : q->mode;
+    P.acc = P.mode != RJ_BOUNDED;
+    P.index = P.mode == RJ_INDEX_JOIN;
+    c->last.mode = P.mode;
+    c->last.est_boundary_frac = f_bnd;
     PassArgs &a = P.a;
     memset(&a, 0, sizeof(a));
     a.f = f;
@@ -236,7 +270,9 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     if ((s = items_for_level(c, P.L)) != RJ_OK) return s;
     c->launches = 0;
     if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[0], c->stream));
-    if (need_polygon_pass && (s = polygon_pass(c, P.W, P.H, P.L, P.acc, P.pp)) != RJ_OK) return s;
+    // the index join needs neither spans nor the boundary mask
+    P.pp = PolyPass{};
+    if (need_polygon_pass && !P.index && (s = polygon_pass(c, P.W, P.H, P.L, P.acc, P.pp)) != RJ_OK) return s;
     if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[1], c->stream));
     a.qx = c->qx.as<uint32_t>();
     a.qy = c->qy.as<uint32_t>();
@@ -251,6 +287,7 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     a.pieces = P.pp.pieces;
     a.mask = P.pp.mask;
     a.mask_wpr = P.pp.mask_wpr;
+    a.index_join = P.index;
     a.grid_off = c->grid_off.as<uint32_t>();
     a.grid_ent = c->grid_ent.as<uint32_t>();
     a.grid_edge = c->grid_edge.as<int4>();
@@ -504,8 +541,11 @@ rj_status rj_get_stats(const rj_ctx *cc, rj_stats *out) {
 }
 
 rj_status rj_debug_pixel_spans(rj_ctx *c, const rj_query_desc *q, uint64_t cap, uint32_t *out, uint64_t *n_out) {
+    if (!q) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL query descriptor");
+    rj_query_desc qq = *q;
+    qq.mode = RJ_BOUNDED;                  // spans do not depend on the mode
     Prepared P;
-    rj_status s = prepare(c, q, P);
+    rj_status s = prepare(c, &qq, P);
     if (s != RJ_OK) return s;
     const uint64_t n = P.pp.n_spans;
     if (n_out) *n_out = n;
@@ -515,7 +555,7 @@ rj_status rj_debug_pixel_spans(rj_ctx *c, const rj_query_desc *q, uint64_t cap, 
 }
 
 rj_status rj_debug_boundary_mask(rj_ctx *c, const rj_query_desc *q, uint32_t *bits) {
-    if (!bits) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL bits");
+    if (!bits || !q) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL bits or query");
     rj_query_desc qq = *q;
     qq.mode = RJ_ACCURATE;
     Prepared P;

@@ -50,7 +50,7 @@ __global__ void k_membership(const PassArgs a, uint64_t n, int accurate, const u
         if (filter_point(a, i)) {
             const int64_t px = pix(qx, a.W), py = pix(qy, a.H);
             bool bnd = false;
-            if (accurate) bnd = (a.mask[(uint64_t)py * a.mask_wpr + (px >> 5)] >> (px & 31)) & 1u;
+            if (accurate) bnd = a.index_join || ((a.mask[(uint64_t)py * a.mask_wpr + (px >> 5)] >> (px & 31)) & 1u);
             if (bnd) {
                 const uint32_t cell = (qy >> kGridShift) * kGrid + (qx >> kGridShift);
                 uint32_t cur = 0xFFFFFFFFu, par = 0;

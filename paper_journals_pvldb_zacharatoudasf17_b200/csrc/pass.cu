@@ -183,8 +183,11 @@ __global__ void __maxnreg__(96) k_point_pass(const PassArgs a) {
                 t.cnt = tcnt + tsel * a.tile_cap;
                 t.sum = tsum + tsel * a.tile_cap;
                 tsel ^= 1u;
-                pb = __ldg(&a.piece_off[m.cell]);          // consumed at the cell's last stage
-                pe = __ldg(&a.piece_off[m.cell + 1]);
+                pb = pe = 0u;                              // consumed at the cell's last stage
+                if (!ACC || !a.index_join) {
+                    pb = __ldg(&a.piece_off[m.cell]);
+                    pe = __ldg(&a.piece_off[m.cell + 1]);
+                }
                 const int64_t cx = cell_x(m.cell), cy = cell_y(m.cell);
                 const uint32_t c0 = (uint32_t)pix(cx << s_lat, a.W), r0 = (uint32_t)pix(cy << s_lat, a.H);
                 t.tw = (uint32_t)pix(((cx + 1) << s_lat) - 1, a.W) - c0 + 1;
@@ -198,7 +201,8 @@ __global__ void __maxnreg__(96) k_point_pass(const PassArgs a) {
                         const uint32_t r = i / t.stride, x = i - r * t.stride;
                         if (x < t.tw) {
                             const uint32_t px = c0 + x;
-                            if ((__ldg(&a.mask[(uint64_t)(r0 + r) * a.mask_wpr + (px >> 5)]) >> (px & 31)) & 1u)
+                            if (a.index_join ||
+                                ((__ldg(&a.mask[(uint64_t)(r0 + r) * a.mask_wpr + (px >> 5)]) >> (px & 31)) & 1u))
                                 v = kFlag;
                         }
                     }
@@ -296,6 +300,9 @@ size_t tile_pass_smem(const PassArgs &a, bool sum, bool accurate) {
 }
 }  // namespace
 
+// Static shared memory of the point-pass kernels (ptxas -v: 256 B) plus margin.
+constexpr size_t kStaticSmem = 512;
+
 // Largest ring that keeps two CTAs (16 consumer warps) per SM, else the
 // largest that fits one CTA; 0 if nothing fits.
 int choose_stages(PassArgs a, size_t (*smem)(const PassArgs &, bool, bool), bool sum, bool accurate) {
@@ -303,7 +310,7 @@ int choose_stages(PassArgs a, size_t (*smem)(const PassArgs &, bool, bool), bool
     int best = 0, best_score = -1;
     for (int st = 2; st <= kMaxStages; ++st) {
         a.n_stages = st;
-        const size_t need = smem(a, sum, accurate) + 2048;
+        const size_t need = smem(a, sum, accurate) + kStaticSmem;
         if (need > budget) continue;
         const int ctas = (int)std::min<size_t>(2, (228 * 1024) / (need + 1024));
         const int score = ctas * 8 + st;

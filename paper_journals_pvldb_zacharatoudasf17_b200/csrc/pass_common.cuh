@@ -108,21 +108,39 @@ __device__ __forceinline__ uint32_t join_point(const PassArgs &a, const Shared &
     const uint32_t b = __ldg(&a.grid_off[cell]), e = __ldg(&a.grid_off[cell + 1]);
     uint32_t cur = kNoPoly, par = 0, first = kNoPoly;
     const int64_t X = px, Y = py;
-    for (uint32_t k = b; k < e; ++k) {
-        const uint32_t P = __ldg(&a.grid_poly[k]);
-        const int4 E = __ldg(&a.grid_edge[k]);
-        if (P != cur) {
-            if (par) {
-                if (first == kNoPoly) first = cur;
-                else emit_poly<SUM>(a, sh, cur, 1u, v);
+    // entries in batches of kJB independent loads: the walk is latency-bound
+    // (L2 round trips), not bandwidth-bound
+    constexpr int kJB = 4;
+    for (uint32_t k0 = b; k0 < e; k0 += kJB) {
+        uint32_t Pb[kJB];
+        int4 Eb[kJB];
+#pragma unroll
+        for (int u = 0; u < kJB; ++u) {
+            Pb[u] = kNoPoly;
+            Eb[u] = make_int4(0, 0, 0, 0);
+            if (k0 + u < e) {
+                Pb[u] = __ldg(&a.grid_poly[k0 + u]);
+                Eb[u] = __ldg(&a.grid_edge[k0 + u]);
             }
-            cur = P;
-            par = 0;
         }
-        if ((E.y > (int)py) != (E.w > (int)py)) {
-            const int64_t lhs = (X - E.x) * (int64_t)(E.w - E.y);
-            const int64_t rhs = (int64_t)(E.z - E.x) * (Y - E.y);
-            if (E.w > E.y ? lhs < rhs : lhs > rhs) par ^= 1u;
+#pragma unroll
+        for (int u = 0; u < kJB; ++u) {
+            if (k0 + u >= e) break;
+            const uint32_t P = Pb[u];
+            const int4 E = Eb[u];
+            if (P != cur) {
+                if (par) {
+                    if (first == kNoPoly) first = cur;
+                    else emit_poly<SUM>(a, sh, cur, 1u, v);
+                }
+                cur = P;
+                par = 0;
+            }
+            if ((E.y > (int)py) != (E.w > (int)py)) {
+                const int64_t lhs = (X - E.x) * (int64_t)(E.w - E.y);
+                const int64_t rhs = (int64_t)(E.z - E.x) * (Y - E.y);
+                if (E.w > E.y ? lhs < rhs : lhs > rhs) par ^= 1u;
+            }
         }
     }
     if (par) {

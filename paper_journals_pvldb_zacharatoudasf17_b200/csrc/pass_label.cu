@@ -193,15 +193,19 @@ __global__ void __maxnreg__(96) k_point_pass_label(const PassArgs a) {
                 const uint32_t th = (uint32_t)pix(((cy + 1) << s_lat) - 1, a.H) - t.r0 + 1;
                 const uint32_t tw = (uint32_t)pix(((cx + 1) << s_lat) - 1, a.W) - t.c0 + 1;
                 t.lab_base = smem_u32(lt) - 4u * (t.r0 * t.stride + t.c0);
-                t.pb = __ldg(&a.piece_off[m.cell]);
-                t.pe = __ldg(&a.piece_off[m.cell + 1]);
+                t.pb = t.pe = 0u;
+                if (!ACC || !a.index_join) {
+                    t.pb = __ldg(&a.piece_off[m.cell]);
+                    t.pe = __ldg(&a.piece_off[m.cell + 1]);
+                }
                 for (uint32_t i = threadIdx.x; i < th * t.stride; i += kThreads) {
                     uint32_t v = kNone;
                     if (ACC) {
                         const uint32_t r = i / t.stride, x = i - r * t.stride;
                         if (x < tw) {
                             const uint32_t px = t.c0 + x;
-                            if ((__ldg(&a.mask[(uint64_t)(t.r0 + r) * a.mask_wpr + (px >> 5)]) >> (px & 31)) & 1u)
+                            if (a.index_join ||
+                                ((__ldg(&a.mask[(uint64_t)(t.r0 + r) * a.mask_wpr + (px >> 5)]) >> (px & 31)) & 1u))
                                 v = kBnd;
                         }
                     }

@@ -314,6 +314,13 @@ rj_status load_polygons_impl(Ctx *c, uint32_t n_poly, const uint32_t *pro, const
     }
     peoff[n_poly] = (uint32_t)edges.size();
     const uint32_t ne = (uint32_t)edges.size();
+    // total edge extent per axis (lattice units): input of the exact-mode
+    // chooser's boundary-pixel estimate
+    double lx = 0.0, ly = 0.0;
+    for (const int4 &e : edges) {
+        lx += std::fabs((double)e.z - (double)e.x);
+        ly += std::fabs((double)e.w - (double)e.y);
+    }
 
     dfree(c, c->edges); dfree(c, c->edge_poly); dfree(c, c->poly_edge_off); dfree(c, c->mbr);
     dfree(c, c->grid_off); dfree(c, c->grid_ent);
@@ -368,6 +375,8 @@ rj_status load_polygons_impl(Ctx *c, uint32_t n_poly, const uint32_t *pro, const
     dfree(c, cnt);
     dfree(c, cur);
     c->n_grid_ent = n_ent;
+    c->edge_len_x = lx;
+    c->edge_len_y = ly;
     c->n_edges = ne;
     c->n_poly = n_poly;
     return RJ_OK;

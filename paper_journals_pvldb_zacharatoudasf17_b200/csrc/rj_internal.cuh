@@ -66,6 +66,7 @@ struct PassArgs {
     int32_t smem_partials;        // accumulate per-CTA polygon partials in smem
     uint32_t tile_cap;            // words of the CTA's tile
     uint32_t n_stages;            // depth of the shared-memory stage ring
+    int32_t index_join;           // every pixel is a boundary pixel, no span pieces (RJ_INDEX_JOIN)
     unsigned long long *stats;    // [0] filtered, [1] boundary
 };
 
@@ -100,6 +101,7 @@ struct Ctx {
     // polygons
     uint32_t n_poly = 0;
     uint32_t n_edges = 0;
+    double edge_len_x = 0.0, edge_len_y = 0.0;   // sum of |dx|, |dy| over edges (lattice units)
     Buf edges, edge_poly, poly_edge_off, mbr;   // int4 edges/mbr
     Buf grid_off, grid_ent;
     Buf grid_edge, grid_poly;                  // entries inlined: edge endpoints + polygon

@@ -26,7 +26,7 @@ RJ_OK = 0
 STATUS = {0: "RJ_OK", -1: "RJ_ERR_INVALID_ARGUMENT", -2: "RJ_ERR_OUT_OF_DOMAIN", -3: "RJ_ERR_RESOLUTION",
           -4: "RJ_ERR_CAPACITY", -5: "RJ_ERR_OOM", -6: "RJ_ERR_CUDA"}
 AGG = {"count": 0, "sum": 1, "avg": 2}
-MODE = {"bounded": 0, "accurate": 1}
+MODE = {"bounded": 0, "accurate": 1, "index": 2, "exact": 3}
 OPS = {"<": 0, "<=": 1, ">": 2, ">=": 3, "==": 4}
 DT_I32, DT_F32, DT_F64 = 0, 1, 2
 OPT_TIMING, OPT_CHUNK, OPT_PASS, OPT_KEEP_LOAD_SCRATCH, OPT_TILE_SIDE = 1, 2, 3, 4, 5
@@ -55,7 +55,8 @@ class rj_stats(ctypes.Structure):
                 ("n_crossings", ctypes.c_uint64), ("n_spans", ctypes.c_uint64), ("n_pieces", ctypes.c_uint64),
                 ("n_items", ctypes.c_uint64), ("stream_bytes", ctypes.c_uint64), ("launches", ctypes.c_uint32),
                 ("ms_polygon", ctypes.c_float), ("ms_point_pass", ctypes.c_float), ("ms_total", ctypes.c_float),
-                ("pass_stages", ctypes.c_int32), ("pass_ctas_per_sm", ctypes.c_int32), ("level", ctypes.c_int32)]
+                ("pass_stages", ctypes.c_int32), ("pass_ctas_per_sm", ctypes.c_int32), ("level", ctypes.c_int32),
+                ("mode", ctypes.c_int32), ("est_boundary_frac", ctypes.c_float)]
 
     def as_dict(self):
         return {k: getattr(self, k) for k, _ in self._fields_}

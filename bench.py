@@ -204,6 +204,7 @@ def main():
     ap.add_argument("--chunk", type=int, default=0, help="points per work item (0 = library default)")
     ap.add_argument("--tile", type=int, default=0, help="point-cell side in pixels (0 = library default)")
     ap.add_argument("--pass-variant", type=int, default=-1, help="SUM/AVG kernel: 0 label, 1 pixel tile")
+    ap.add_argument("--stages", type=int, default=0, help="point-pass ring depth (0 = library default)")
     ap.add_argument("--mode", default="", help="override the config's mode: bounded|accurate|index|exact")
     args = ap.parse_args()
     args.warmup = max(3, args.warmup)
@@ -244,6 +245,8 @@ def main():
         R.set_option(rj.OPT_CHUNK, args.chunk)
     if args.tile:
         R.set_option(rj.OPT_TILE_SIDE, args.tile)
+    if args.stages:
+        R.set_option(rj.OPT_STAGES, args.stages)
     if args.pass_variant >= 0:
         R.set_option(rj.OPT_PASS, args.pass_variant)
     flat = C.array_polys(polys_name)

@@ -190,17 +190,22 @@ static void tile_geometry(int W, int H, int L, uint32_t &stride, uint32_t &cap) 
 }
 
 // Exact-mode chooser (RJ_EXACT).  Both exact variants
-// stream every point once; they differ in the PIP tests and the polygon pass:
-//   accurate:   T_poly + f * N * c_pip      index join:  N * c_pip
-// f = estimated boundary-pixel fraction: each edge's supercover touches
-// about |dx| W + |dy| H (lattice units / 2^30) + 1 pixels.  T_poly is the
-// polygon pass (launch floor + crossings + boundary mask), measured on B200
-// (profiles/r1_chooser.md).
+// stream every point once; the accurate raster join adds the polygon pass and
+// a small per-point cost of its boundary check, and tests only points in
+// boundary pixels; the index join tests every point:
+//   accurate:   T_poly + N c_acc + f N c_bnd       index join:  N c_idx
+// f = estimated boundary-pixel fraction (each edge's supercover touches about
+// |dx| W + |dy| H (lattice units / 2^30) + 1 pixels; uniform point density
+// assumed), T_poly = floor + crossings + boundary mask.  Constants measured
+// on B200 (C2/C3 sweeps, profiles/r1_chooser.md); N = loaded points (the
+// filter's selectivity is unknown before the pass).
 struct ChooserModel {
-    double t_floor_us = 60.0;      // polygon-pass launch / sync floor
-    double t_cross_ns = 0.02;      // per (edge, row) crossing
-    double t_mask_ns = 0.004;      // per boundary-mask pixel
-    double c_pip_ns = 0.16;        // per point routed through the edge grid
+    double t_floor_ns = 60e3;      // polygon-pass launch / sync floor
+    double t_cross_ns = 0.2;       // per (edge, row) crossing
+    double t_mask_ns = 0.002;      // per canvas pixel (boundary mask clear + mark)
+    double c_acc_ns = 0.00075;     // per streamed point: boundary-flag check
+    double c_bnd_ns = 0.096;       // per boundary point (queued PIP, clustered near edges)
+    double c_idx_ns = 0.028;       // per point, index join (full-warp PIP batches)
 };
 
 static float boundary_fraction(const Ctx *c, int W, int H) {
@@ -211,10 +216,11 @@ static float boundary_fraction(const Ctx *c, int W, int H) {
 
 static int choose_exact(const Ctx *c, int W, int H, float f) {
     const ChooserModel m;
+    const double n = (double)c->n_pts;
     const double cross = c->edge_len_y * H / 1073741824.0 + (double)c->n_edges;
-    const double t_poly = m.t_floor_us * 1e3 + m.t_cross_ns * cross + m.t_mask_ns * (double)W * H;
-    const double saved = (1.0 - f) * (double)c->n_pts * m.c_pip_ns;
-    return t_poly > saved ? RJ_INDEX_JOIN : RJ_ACCURATE;
+    const double t_acc = m.t_floor_ns + m.t_cross_ns * cross + m.t_mask_ns * (double)W * H + n * m.c_acc_ns +
+                         f * n * m.c_bnd_ns;
+    return n * m.c_idx_ns < t_acc ? RJ_INDEX_JOIN : RJ_ACCURATE;
 }
 
 struct Prepared {
@@ -431,6 +437,11 @@ rj_status rj_set_option(rj_ctx *c, int32_t option, int64_t value) {
     if (option == RJ_OPT_PASS) {
         if (value < -1 || value > 1) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "RJ_OPT_PASS must be -1, 0 or 1");
         c->pass_variant = (int)value;
+        return RJ_OK;
+    }
+    if (option == RJ_OPT_STAGES) {
+        if (value != 0 && (value < 2 || value > 4)) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "RJ_OPT_STAGES must be 0 or in [2, 4]");
+        c->force_stages = (int)value;
         return RJ_OK;
     }
     if (option == RJ_OPT_TILE_SIDE) {

@@ -86,7 +86,7 @@ __device__ __forceinline__ void process(const PassArgs &a, const Shared &sh, con
 #pragma unroll
             for (int j = 0; j < kIPL; ++j) {
                 enqueue<SUM, NS>(a, sh, w, j, (bm >> j) & 1u, qn, n_bnd);   // adds <= 32
-                drain_queue<SUM>(a, sh, qn, false);                          // leaves < 32
+                if (qn >= 32) drain_queue<SUM>(a, sh, qn, false);            // leaves < 32
             }
 #pragma unroll
             for (int j = 0; j < kIPL; ++j) ok[j] = ok[j] && !((bm >> j) & 1u);
@@ -126,7 +126,7 @@ __device__ __forceinline__ void process(const PassArgs &a, const Shared &sh, con
 }
 
 template <bool SUM, bool ACC, int NS, bool FP>
-__global__ void __maxnreg__(96) k_point_pass(const PassArgs a) {
+__global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a) {
     extern __shared__ __align__(128) unsigned char smem_raw[];
     __shared__ __align__(8) Ring rg;
     __shared__ uint32_t s_pass, s_bnd;
@@ -195,20 +195,13 @@ __global__ void __maxnreg__(96) k_point_pass(const PassArgs a) {
                 t.base = r0 * t.stride + c0;
                 t.tbase = smem_u32(t.cnt) - 4u * t.base;
                 const uint32_t words = t.th * t.stride;
-                for (uint32_t i = threadIdx.x; i < words; i += kThreads) {
-                    uint32_t v = 0u;
-                    if (ACC) {
-                        const uint32_t r = i / t.stride, x = i - r * t.stride;
-                        if (x < t.tw) {
-                            const uint32_t px = c0 + x;
-                            if (a.index_join ||
-                                ((__ldg(&a.mask[(uint64_t)(r0 + r) * a.mask_wpr + (px >> 5)]) >> (px & 31)) & 1u))
-                                v = kFlag;
-                        }
-                    }
-                    t.cnt[i] = v;
-                    if (SUM) t.sum[i] = 0.0;
+                if (ACC) {
+                    clear_tile_acc(t.cnt, t.stride, t.th, t.tw, r0, c0, a.mask, a.mask_wpr, a.index_join, kFlag, 0u);
+                } else {
+                    for (uint32_t i = threadIdx.x; i < words; i += kThreads) t.cnt[i] = 0u;
                 }
+                if (SUM)
+                    for (uint32_t i = threadIdx.x; i < words; i += kThreads) t.sum[i] = 0.0;
                 consumers_sync();
             }
             uint2 pc0 = make_uint2(0u, 0u);
@@ -226,7 +219,7 @@ __global__ void __maxnreg__(96) k_point_pass(const PassArgs a) {
             if (lane == 0) mbar_arrive(smem_u32(&rg.empty[st]));
             if (m.flags & 2u) {
                 // ---- last stage of the cell: reduce the tile over the span pieces (S4)
-                if (ACC) drain_queue<SUM>(a, sh, qn, true);
+                if (ACC && qn) drain_queue<SUM>(a, sh, qn, true);
                 consumers_sync();                          // every point of the cell is in the tile
                 for (uint32_t kk = pb + threadIdx.x; kk < pe; kk += kThreads) {
                     const uint2 pc = (kk == pb + threadIdx.x) ? pc0 : __ldg(&a.pieces[kk]);
@@ -305,8 +298,12 @@ constexpr size_t kStaticSmem = 512;
 
 // Largest ring that keeps two CTAs (16 consumer warps) per SM, else the
 // largest that fits one CTA; 0 if nothing fits.
-int choose_stages(PassArgs a, size_t (*smem)(const PassArgs &, bool, bool), bool sum, bool accurate) {
+int choose_stages(PassArgs a, size_t (*smem)(const PassArgs &, bool, bool), bool sum, bool accurate, int force) {
     const size_t budget = 227 * 1024 - 1024;
+    if (force >= 2 && force <= kMaxStages) {
+        a.n_stages = force;
+        if (smem(a, sum, accurate) + kStaticSmem <= budget) return force;
+    }
     int best = 0, best_score = -1;
     for (int st = 2; st <= kMaxStages; ++st) {
         a.n_stages = st;
@@ -352,7 +349,7 @@ int point_pass_stages(int n_slots) { return (2 + n_slots) <= 4 ? 3 : 2; }
 rj_status point_pass(Ctx *c, const PassArgs &a_in, bool sum, bool accurate) {
     if (use_label(c, sum, accurate)) return point_pass_label(c, a_in, accurate);
     PassArgs a = a_in;
-    a.n_stages = (uint32_t)choose_stages(a, tile_pass_smem, sum, accurate);
+    a.n_stages = (uint32_t)choose_stages(a, tile_pass_smem, sum, accurate, c->force_stages);
     if (!a.n_stages) return set_error(c, RJ_ERR_RESOLUTION, "point-pass tiles do not fit in shared memory");
     return launch_pass(c, select_kernel(sum, accurate, a.f.n_slots, a.f.n_fpred > 0), a,
                        tile_pass_smem(a, sum, accurate));

@@ -108,39 +108,21 @@ __device__ __forceinline__ uint32_t join_point(const PassArgs &a, const Shared &
     const uint32_t b = __ldg(&a.grid_off[cell]), e = __ldg(&a.grid_off[cell + 1]);
     uint32_t cur = kNoPoly, par = 0, first = kNoPoly;
     const int64_t X = px, Y = py;
-    // entries in batches of kJB independent loads: the walk is latency-bound
-    // (L2 round trips), not bandwidth-bound
-    constexpr int kJB = 4;
-    for (uint32_t k0 = b; k0 < e; k0 += kJB) {
-        uint32_t Pb[kJB];
-        int4 Eb[kJB];
-#pragma unroll
-        for (int u = 0; u < kJB; ++u) {
-            Pb[u] = kNoPoly;
-            Eb[u] = make_int4(0, 0, 0, 0);
-            if (k0 + u < e) {
-                Pb[u] = __ldg(&a.grid_poly[k0 + u]);
-                Eb[u] = __ldg(&a.grid_edge[k0 + u]);
+    for (uint32_t k = b; k < e; ++k) {
+        const uint32_t P = __ldg(&a.grid_poly[k]);
+        const int4 E = __ldg(&a.grid_edge[k]);
+        if (P != cur) {
+            if (par) {
+                if (first == kNoPoly) first = cur;
+                else emit_poly<SUM>(a, sh, cur, 1u, v);
             }
+            cur = P;
+            par = 0;
         }
-#pragma unroll
-        for (int u = 0; u < kJB; ++u) {
-            if (k0 + u >= e) break;
-            const uint32_t P = Pb[u];
-            const int4 E = Eb[u];
-            if (P != cur) {
-                if (par) {
-                    if (first == kNoPoly) first = cur;
-                    else emit_poly<SUM>(a, sh, cur, 1u, v);
-                }
-                cur = P;
-                par = 0;
-            }
-            if ((E.y > (int)py) != (E.w > (int)py)) {
-                const int64_t lhs = (X - E.x) * (int64_t)(E.w - E.y);
-                const int64_t rhs = (int64_t)(E.z - E.x) * (Y - E.y);
-                if (E.w > E.y ? lhs < rhs : lhs > rhs) par ^= 1u;
-            }
+        if ((E.y > (int)py) != (E.w > (int)py)) {
+            const int64_t lhs = (X - E.x) * (int64_t)(E.w - E.y);
+            const int64_t rhs = (int64_t)(E.z - E.x) * (Y - E.y);
+            if (E.w > E.y ? lhs < rhs : lhs > rhs) par ^= 1u;
         }
     }
     if (par) {
@@ -229,6 +211,31 @@ __device__ __forceinline__ void enqueue(const PassArgs &a, const Shared &sh, con
             ++n_bnd;
         }
         qn += __popc(bb);
+    }
+}
+
+// Accurate-mode tile clear: word (r, x) of a th x stride tile becomes `flag`
+// when x < tw and pixel (c0 + x, r0 + r) is a boundary pixel (every pixel
+// when `all`, the index join), else `zero`.  Warp w clears rows w, w + 8, ...;
+// each row's <= 5 mask words are loaded once (one lane each) and shuffled to
+// the lanes that need them, and the row loop is unrolled so several rows'
+// loads are in flight (the clear sits between two consumer barriers, so its
+// L2 latency is exposed).
+__device__ __forceinline__ void clear_tile_acc(uint32_t *tile, uint32_t stride, uint32_t th, uint32_t tw,
+                                               uint32_t r0, uint32_t c0, const uint32_t *mask, uint32_t wpr,
+                                               bool all, uint32_t flag, uint32_t zero) {
+    const uint32_t lane = threadIdx.x & 31, wid = threadIdx.x >> 5;
+    const uint32_t w0 = c0 >> 5;
+    const uint32_t nwords = ((c0 + tw - 1) >> 5) - w0 + 1;
+#pragma unroll 4
+    for (uint32_t r = wid; r < th; r += kWarps) {
+        uint32_t word = 0xFFFFFFFFu;
+        if (!all && lane < nwords) word = __ldg(&mask[(uint64_t)(r0 + r) * wpr + w0 + lane]);
+        for (uint32_t x0 = 0; x0 < stride; x0 += 32) {
+            const uint32_t x = x0 + lane, px = c0 + x;
+            const uint32_t wv = __shfl_sync(kFull, word, ((px >> 5) - w0) & 31u);
+            if (x < stride) tile[r * stride + x] = (x < tw && ((wv >> (px & 31)) & 1u)) ? flag : zero;
+        }
     }
 }
 

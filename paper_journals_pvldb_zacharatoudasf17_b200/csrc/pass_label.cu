@@ -17,7 +17,7 @@
 
 namespace rj {
 
-int choose_stages(PassArgs a, size_t (*smem)(const PassArgs &, bool, bool), bool sum, bool accurate);  // pass.cu
+int choose_stages(PassArgs a, size_t (*smem)(const PassArgs &, bool, bool), bool sum, bool accurate, int force);  // pass.cu
 rj_status launch_pass(Ctx *c, void *k, const PassArgs &a, size_t smem);
 
 namespace {
@@ -79,7 +79,7 @@ __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh,
                             attr_val(agg_bits<NS>(a, w, j), a.f.agg_is_float));
             if (ACC) {
                 enqueue<true, NS>(a, sh, w, j, lab[j] == kBnd, qn, n_bnd);   // adds <= 32
-                drain_queue<true>(a, sh, qn, false);                          // leaves < 32
+                if (qn >= 32) drain_queue<true>(a, sh, qn, false);            // leaves < 32
             }
             if (lab[j] >= kBnd) lab[j] = kNone;
         }
@@ -134,7 +134,7 @@ __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh,
 }
 
 template <bool ACC, int NS, bool FP>
-__global__ void __maxnreg__(96) k_point_pass_label(const PassArgs a) {
+__global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassArgs a) {
     extern __shared__ __align__(128) unsigned char smem_raw[];
     __shared__ __align__(8) Ring rg;
     __shared__ uint32_t s_pass, s_bnd;
@@ -198,18 +198,10 @@ __global__ void __maxnreg__(96) k_point_pass_label(const PassArgs a) {
                     t.pb = __ldg(&a.piece_off[m.cell]);
                     t.pe = __ldg(&a.piece_off[m.cell + 1]);
                 }
-                for (uint32_t i = threadIdx.x; i < th * t.stride; i += kThreads) {
-                    uint32_t v = kNone;
-                    if (ACC) {
-                        const uint32_t r = i / t.stride, x = i - r * t.stride;
-                        if (x < tw) {
-                            const uint32_t px = t.c0 + x;
-                            if (a.index_join ||
-                                ((__ldg(&a.mask[(uint64_t)(t.r0 + r) * a.mask_wpr + (px >> 5)]) >> (px & 31)) & 1u))
-                                v = kBnd;
-                        }
-                    }
-                    lt[i] = v;
+                if (ACC) {
+                    clear_tile_acc(lt, t.stride, th, tw, t.r0, t.c0, a.mask, a.mask_wpr, a.index_join, kBnd, kNone);
+                } else {
+                    for (uint32_t i = threadIdx.x; i < th * t.stride; i += kThreads) lt[i] = kNone;
                 }
                 consumers_sync();
                 // one thread per span piece; shared CAS turns overlaps into MULTI
@@ -231,12 +223,12 @@ __global__ void __maxnreg__(96) k_point_pass_label(const PassArgs a) {
                 load_win_smem<NS>(w, ring + (size_t)st * ncol * kStagePts, woff + lane * kIPL);
                 process_lab<ACC, NS, FP>(a, sh, t, k, w, (m.sb - m.cb) - woff, m.se - m.sb, cy, qn, n_pass, n_bnd);
             }
-            if (ACC && (m.flags & 2u)) drain_queue<true>(a, sh, qn, true);
+            if (ACC && (m.flags & 2u) && qn) drain_queue<true>(a, sh, qn, true);
             __syncwarp();
             if (lane == 0) mbar_arrive(smem_u32(&rg.empty[st]));
             if (++st == nstage) { st = 0; ph ^= 1u; }
         }
-        if (ACC) drain_queue<true>(a, sh, qn, true);
+        if (ACC && qn) drain_queue<true>(a, sh, qn, true);
         if (lane == 0) emit_lab_run(a, sh, cy.lab, cy.cnt, cy.sum, true);
         for (int o = 16; o; o >>= 1) {
             n_pass += __shfl_xor_sync(kFull, n_pass, o);
@@ -283,7 +275,7 @@ size_t point_pass_label_smem(const PassArgs &a, bool accurate) { return label_sm
 
 rj_status point_pass_label(Ctx *c, const PassArgs &a_in, bool accurate) {
     PassArgs a = a_in;
-    a.n_stages = (uint32_t)choose_stages(a, label_smem, true, accurate);
+    a.n_stages = (uint32_t)choose_stages(a, label_smem, true, accurate, c->force_stages);
     if (!a.n_stages) return set_error(c, RJ_ERR_RESOLUTION, "point-pass tiles do not fit in shared memory");
     const bool fp = a.f.n_fpred > 0;
     void *k = accurate ? (fp ? select_ns<true, true>(a.f.n_slots) : select_ns<true, false>(a.f.n_slots))

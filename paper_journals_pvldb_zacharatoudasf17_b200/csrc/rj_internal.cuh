@@ -117,6 +117,7 @@ struct Ctx {
     uint32_t launches = 0;
     int last_stages = 0, last_ctas_per_sm = 0;   // point-pass launch shape of the last query
     int pass_variant = -1;                        // RJ_OPT_PASS: -1 auto, 0 label, 1 pixel tile
+    int force_stages = 0;                         // RJ_OPT_STAGES: 0 = automatic, else 2..4
     int tile_side = 64;                           // RJ_OPT_TILE_SIDE: target point-cell side in pixels
 };
 

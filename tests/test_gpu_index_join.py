@@ -115,7 +115,7 @@ def test_index_join_empty_and_tiny():
 def test_exact_chooser(c1):
     """RJ_EXACT resolves to one of the exact variants and returns the exact
     result; a handful of points picks the index join (the polygon pass would
-    dominate), 4M points on 64 coarse polygons pick the raster join."""
+    dominate), 16M points on the coarse C1b polygons pick the raster join."""
     flat, x, y, cols = c1
     P = oracle.Polys(flat, C.C1_BOX)
     R = ctx(C.C1_BOX, flat, x[:1000], y[:1000])
@@ -124,7 +124,7 @@ def test_exact_chooser(c1):
     assert np.array_equal(cnt, ocnt)
     assert R.stats()["mode"] == 2
     R.close()
-    pts = C.c1_points(4_000_000)
+    pts = C.c1_points(16_000_000)
     R = ctx(C.C1_BOX, flat, pts["x"], pts["y"])
     cnt, _ = R.query(W=1024, H=1024, mode="exact")
     st = R.stats()

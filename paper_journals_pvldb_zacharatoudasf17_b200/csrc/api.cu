@@ -113,17 +113,17 @@ static void int_range(int op, double c, int64_t &lo, int64_t &hi, int &never) {
     }
 }
 
-static rj_status build_filter(Ctx *c, const rj_query_desc *q, Filter &f) {
+rj_status build_filter(Ctx *c, const rj_query_desc *q, int n_cols, const int *col_dtype, Filter &f) {
     f = Filter{};
     if (q->n_pred < 0 || q->n_pred > RJ_MAX_PRED) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "n_pred must be in [0, 5]");
     if (q->agg < RJ_COUNT || q->agg > RJ_AVG) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad agg");
     if (q->mode < RJ_BOUNDED || q->mode > RJ_EXACT) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad mode");
     for (int k = 0; k < q->n_pred; ++k) {
         const rj_pred &p = q->pred[k];
-        if (p.column < 0 || p.column >= c->n_cols) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "predicate column out of range");
+        if (p.column < 0 || p.column >= n_cols) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "predicate column out of range");
         if (p.op < RJ_LT || p.op > RJ_EQ) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad predicate op");
     }
-    if (q->agg != RJ_COUNT && (q->agg_column < 0 || q->agg_column >= c->n_cols))
+    if (q->agg != RJ_COUNT && (q->agg_column < 0 || q->agg_column >= n_cols))
         return set_error(c, RJ_ERR_INVALID_ARGUMENT, "agg_column out of range");
     // slots: int-range columns first, then float-predicate columns, then the agg column
     int slot_of[RJ_MAX_COLS];
@@ -131,7 +131,7 @@ static rj_status build_filter(Ctx *c, const rj_query_desc *q, Filter &f) {
     int64_t lo[RJ_MAX_COLS], hi[RJ_MAX_COLS];
     for (int k = 0; k < q->n_pred; ++k) {
         const rj_pred &p = q->pred[k];
-        if (c->col_dtype[p.column] != RJ_I32) continue;
+        if (col_dtype[p.column] != RJ_I32) continue;
         if (slot_of[p.column] < 0) {
             slot_of[p.column] = f.n_slots;
             f.slot_col[f.n_slots] = p.column;
@@ -151,7 +151,7 @@ static rj_status build_filter(Ctx *c, const rj_query_desc *q, Filter &f) {
     }
     for (int k = 0; k < q->n_pred; ++k) {
         const rj_pred &p = q->pred[k];
-        if (c->col_dtype[p.column] != RJ_F32) continue;
+        if (col_dtype[p.column] != RJ_F32) continue;
         if (slot_of[p.column] < 0) {
             slot_of[p.column] = f.n_slots;
             f.slot_col[f.n_slots] = p.column;
@@ -169,7 +169,7 @@ static rj_status build_filter(Ctx *c, const rj_query_desc *q, Filter &f) {
         if (slot_of[q->agg_column] < 0) {
             slot_of[q->agg_column] = f.n_slots;
             f.slot_col[f.n_slots] = q->agg_column;
-            f.slot_is_float[f.n_slots] = c->col_dtype[q->agg_column] == RJ_F32;
+            f.slot_is_float[f.n_slots] = col_dtype[q->agg_column] == RJ_F32;
             f.n_slots++;
         }
         f.agg_slot = slot_of[q->agg_column];
@@ -214,9 +214,9 @@ static float boundary_fraction(const Ctx *c, int W, int H) {
     return (float)std::min(1.0, b / px);
 }
 
-static int choose_exact(const Ctx *c, int W, int H, float f) {
+static int choose_exact(const Ctx *c, int W, int H, float f, uint64_t n_points) {
     const ChooserModel m;
-    const double n = (double)c->n_pts;
+    const double n = (double)n_points;
     const double cross = c->edge_len_y * H / 1073741824.0 + (double)c->n_edges;
     const double t_acc = m.t_floor_ns + m.t_cross_ns * cross + m.t_mask_ns * (double)W * H + n * m.c_acc_ns +
                          f * n * m.c_bnd_ns;
@@ -248,10 +248,10 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     if ((s = resolve(c->x0, c->y0, c->x1, c->y1, q, &P.W, &P.H)) != RJ_OK)
         return set_error(c, s, "canvas resolution outside [1, 32768] or bad epsilon");
     Filter f;
-    if ((s = build_filter(c, q, f)) != RJ_OK) return s;
+    if ((s = build_filter(c, q, c->n_cols, c->col_dtype, f)) != RJ_OK) return s;
     P.sum = q->agg != RJ_COUNT;
     const float f_bnd = boundary_fraction(c, P.W, P.H);
-    P.mode = q->mode == RJ_EXACT ? choose_exact(c, P.W, P.H, f_bnd) : q->mode;
+    P.mode = q->mode == RJ_EXACT ? choose_exact(c, P.W, P.H, f_bnd, c->n_pts) : q->mode;
     P.acc = P.mode != RJ_BOUNDED;
     P.index = P.mode == RJ_INDEX_JOIN;
     c->last.mode = P.mode;
@@ -319,6 +319,7 @@ static rj_status run_pass(Ctx *c, Prepared &P, unsigned long long *d_cnt, double
     if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[2], c->stream));
     RJ_CUDA(c, cudaMemcpyAsync(c->h_stats, a.stats, 2 * sizeof(unsigned long long), cudaMemcpyDeviceToHost, c->stream));
     // statistics of this query
+    c->stream_stats_pending = 0;
     rj_stats &L = c->last;
     L.W = P.W;
     L.H = P.H;
@@ -415,6 +416,7 @@ rj_status rj_destroy(rj_ctx *c) {
     dfree(c, c->grid_off); dfree(c, c->grid_ent); dfree(c, c->grid_edge); dfree(c, c->grid_poly);
     for (auto &b : c->ws) dfree(c, b);
     dfree(c, c->res_cnt); dfree(c, c->res_sum); dfree(c, c->res_val);
+    stream_release(c);
     for (auto &e : c->ev) if (e) cudaEventDestroy(e);
     if (c->h_stats) cudaFreeHost(c->h_stats);
     if (c->own_stream) cudaStreamDestroy(c->stream);
@@ -437,6 +439,11 @@ rj_status rj_set_option(rj_ctx *c, int32_t option, int64_t value) {
     if (option == RJ_OPT_PASS) {
         if (value < -1 || value > 1) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "RJ_OPT_PASS must be -1, 0 or 1");
         c->pass_variant = (int)value;
+        return RJ_OK;
+    }
+    if (option == RJ_OPT_STREAM_BATCH) {
+        if (value < 1024) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "RJ_OPT_STREAM_BATCH must be >= 1024");
+        c->stream_batch = value;
         return RJ_OK;
     }
     if (option == RJ_OPT_STAGES) {
@@ -529,12 +536,58 @@ rj_status rj_query(rj_ctx *c, const rj_query_desc *q, uint64_t *count, double *v
     return RJ_OK;
 }
 
+rj_status rj_query_stream(rj_ctx *c, const rj_query_desc *q, uint64_t n, const void *x, const void *y,
+                          int32_t xy_dtype, int32_t n_cols, const void *const *cols, const int32_t *dtypes,
+                          uint64_t *count, double *value) {
+    if (!c) return RJ_ERR_INVALID_ARGUMENT;
+    if (c->poisoned) return set_error(c, RJ_ERR_CUDA, c->err.empty() ? "context poisoned" : c->err);
+    if (!q) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL query descriptor");
+    if (!c->n_poly) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "query before rj_load_polygons");
+    if (n && (!x || !y)) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL coordinates");
+    if (xy_dtype != RJ_F32 && xy_dtype != RJ_F64) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "coordinates must be RJ_F32 or RJ_F64");
+    if (n_cols < 0 || n_cols > RJ_MAX_COLS) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "n_cols must be in [0, 8]");
+    if (n_cols && (!cols || !dtypes)) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL attribute columns");
+    int dt[RJ_MAX_COLS];
+    for (int k = 0; k < n_cols; ++k) {
+        if (dtypes[k] != RJ_I32 && dtypes[k] != RJ_F32) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "attributes must be RJ_I32 or RJ_F32");
+        if (n && !cols[k]) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL attribute column");
+        dt[k] = dtypes[k];
+    }
+    if (cudaSetDevice(c->device) != cudaSuccess) return set_error(c, RJ_ERR_CUDA, "cudaSetDevice failed");
+    int W, H;
+    rj_status s = resolve(c->x0, c->y0, c->x1, c->y1, q, &W, &H);
+    if (s != RJ_OK) return set_error(c, s, "canvas resolution outside [1, 32768] or bad epsilon");
+    Filter f;
+    if ((s = build_filter(c, q, n_cols, dt, f)) != RJ_OK) return s;
+    const float f_bnd = boundary_fraction(c, W, H);
+    const int mode = q->mode == RJ_EXACT ? choose_exact(c, W, H, f_bnd, n) : q->mode;
+    c->last.mode = mode;
+    c->last.est_boundary_frac = f_bnd;
+    const size_t np = c->n_poly;
+    if (dreserve(c, c->res_cnt, np * 8) || dreserve(c, c->res_sum, np * 8) || dreserve(c, c->res_val, np * 8))
+        return set_error(c, RJ_ERR_OOM, "result allocation failed");
+    if ((s = stream_query_impl(c, f, q->agg != RJ_COUNT, W, H, mode, n, x, y, xy_dtype == RJ_F64, cols,
+                               c->res_cnt.as<unsigned long long>(), c->res_sum.as<double>())) != RJ_OK)
+        return s;
+    if (value) RJ_CUDA(c, launch_finalize(c, q->agg, (uint32_t)np, c->res_cnt.as<unsigned long long>(),
+                                          c->res_sum.as<double>(), c->res_val.as<double>()));
+    if (count) RJ_CUDA(c, cudaMemcpyAsync(count, c->res_cnt.p, np * 8, cudaMemcpyDeviceToHost, c->stream));
+    if (value) RJ_CUDA(c, cudaMemcpyAsync(value, c->res_val.p, np * 8, cudaMemcpyDeviceToHost, c->stream));
+    if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[3], c->stream));
+    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
+    return RJ_OK;
+}
+
 rj_status rj_get_stats(const rj_ctx *cc, rj_stats *out) {
     rj_ctx *c = const_cast<rj_ctx *>(cc);
     if (!c || !out) return RJ_ERR_INVALID_ARGUMENT;
     RJ_CUDA(c, cudaStreamSynchronize(c->stream));
     c->last.n_filtered = c->h_stats[0];
     c->last.n_boundary = c->h_stats[1];
+    if (c->stream_stats_pending) {
+        c->last.n_points -= std::min<uint64_t>(c->last.n_points, c->h_stats[2]);
+        c->stream_stats_pending = 0;
+    }
     c->last.launches = c->launches;
     c->last.pass_stages = c->last_stages;
     c->last.pass_ctas_per_sm = c->last_ctas_per_sm;

@@ -6,6 +6,7 @@
 // ring (cp.async.bulk + mbarrier).
 #pragma once
 #include "rj_internal.cuh"
+#include "pip.cuh"
 
 namespace rj {
 namespace pass {
@@ -96,40 +97,14 @@ __device__ __forceinline__ void emit_poly(const PassArgs &a, const Shared &sh, u
     if (SUM) atomicAdd(&a.A_sum[P], s);
 }
 
-// Proc. JoinPoint: exact even-odd test of lattice point (px, py)
-// against every polygon through the edge-grid cell.  Cell entries are sorted
-// by edge id, so they group by polygon.  Returns the first containing polygon
-// (kNoPoly if none); any further containing polygons (overlaps) get (1, v)
-// directly.
+// Proc. JoinPoint through the edge grid (pip.cuh): returns the
+// first containing polygon (kNoPoly if none); any further containing
+// polygons (overlaps) get (1, v) directly.
 template <bool SUM>
 __device__ __forceinline__ uint32_t join_point(const PassArgs &a, const Shared &sh, uint32_t px, uint32_t py,
                                                double v) {
-    const uint32_t cell = (py >> kGridShift) * kGrid + (px >> kGridShift);
-    const uint32_t b = __ldg(&a.grid_off[cell]), e = __ldg(&a.grid_off[cell + 1]);
-    uint32_t cur = kNoPoly, par = 0, first = kNoPoly;
-    const int64_t X = px, Y = py;
-    for (uint32_t k = b; k < e; ++k) {
-        const uint32_t P = __ldg(&a.grid_poly[k]);
-        const int4 E = __ldg(&a.grid_edge[k]);
-        if (P != cur) {
-            if (par) {
-                if (first == kNoPoly) first = cur;
-                else emit_poly<SUM>(a, sh, cur, 1u, v);
-            }
-            cur = P;
-            par = 0;
-        }
-        if ((E.y > (int)py) != (E.w > (int)py)) {
-            const int64_t lhs = (X - E.x) * (int64_t)(E.w - E.y);
-            const int64_t rhs = (int64_t)(E.z - E.x) * (Y - E.y);
-            if (E.w > E.y ? lhs < rhs : lhs > rhs) par ^= 1u;
-        }
-    }
-    if (par) {
-        if (first == kNoPoly) first = cur;
-        else emit_poly<SUM>(a, sh, cur, 1u, v);
-    }
-    return first;
+    return grid_pip(a.grid_off, a.grid_poly, a.grid_edge, px, py,
+                    [&](uint32_t P) { emit_poly<SUM>(a, sh, P, 1u, v); });
 }
 
 // Test the queued boundary points, 32 at a time (one per lane), and add

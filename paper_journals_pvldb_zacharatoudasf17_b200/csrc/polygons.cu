@@ -159,6 +159,7 @@ __device__ __forceinline__ void polyrow_of(const SpanGeo &g, uint32_t pr, uint32
 // Visit the (cell, local row, local lo, local hi) pieces of span [lo, hi) of row r.
 template <class F>
 __device__ __forceinline__ void for_each_piece(const SpanGeo &g, int64_t r, int64_t lo, int64_t hi, F f) {
+    if (g.L < 0) return;                                   // spans only
     const int s = kLatticeBits - g.L, sh = 2 * (kMaxLevel - g.L);
     const int64_t cr0 = qlo(r, g.H) >> s, cr1 = qhi(r, g.H) >> s;
     const int64_t cc0 = qlo(lo, g.W) >> s, cc1 = qhi(hi - 1, g.W) >> s;
@@ -384,7 +385,8 @@ rj_status load_polygons_impl(Ctx *c, uint32_t n_poly, const uint32_t *pro, const
 
 // ------------------------------------------------------------ per-query pass
 rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp) {
-    const uint64_t ncell = 1ull << (2 * L);
+    // L < 0: spans (and mask) only, no pieces (the streamed query)
+    const uint64_t ncell = L >= 0 ? 1ull << (2 * L) : 0;
     const uint32_t ne = c->n_edges, np = c->n_poly;
     cudaStream_t st = c->stream;
     Buf &erows = wsbuf(c, kWsEdgeRows), &eoff = wsbuf(c, kWsEdgeOff);
@@ -443,10 +445,11 @@ rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp)
     RJ_LAUNCHED(c);
     RJ_CUDA(c, cudaGetLastError());
     RJ_CUDA(c, scan_u32(c, scnt.as<uint32_t>(), soff.as<uint32_t>(), NPR, kWsScan));
-    RJ_CUDA(c, scan_u32(c, pcnt.as<uint32_t>(), poff.as<uint32_t>(), ncell, kWsScan));
+    if (ncell) RJ_CUDA(c, scan_u32(c, pcnt.as<uint32_t>(), poff.as<uint32_t>(), ncell, kWsScan));
     // sync 2: span / piece totals
+    hs[4] = 0;
     RJ_CUDA(c, cudaMemcpyAsync(hs + 3, soff.as<uint32_t>() + NPR, 4, cudaMemcpyDeviceToHost, st));
-    RJ_CUDA(c, cudaMemcpyAsync(hs + 4, poff.as<uint32_t>() + ncell, 4, cudaMemcpyDeviceToHost, st));
+    if (ncell) RJ_CUDA(c, cudaMemcpyAsync(hs + 4, poff.as<uint32_t>() + ncell, 4, cudaMemcpyDeviceToHost, st));
     RJ_CUDA(c, cudaStreamSynchronize(st));
     const uint32_t S = hs[3], NP = hs[4];
     Buf &spans = wsbuf(c, kWsSpans), &pieces = wsbuf(c, kWsPieces);

@@ -119,6 +119,13 @@ struct Ctx {
     int pass_variant = -1;                        // RJ_OPT_PASS: -1 auto, 0 label, 1 pixel tile
     int force_stages = 0;                         // RJ_OPT_STAGES: 0 = automatic, else 2..4
     int tile_side = 64;                           // RJ_OPT_TILE_SIDE: target point-cell side in pixels
+
+    // streamed query (stream.cu)
+    int64_t stream_batch = int64_t(1) << 24;      // RJ_OPT_STREAM_BATCH: points per batch
+    cudaStream_t copy_stream = nullptr;           // H2D copies of the batches
+    cudaEvent_t sev[5] = {};                      // copied[2], consumed[2], start
+    Buf sbuf[2][2 + RJ_MAX_COLS];                 // double-buffered device batches
+    int stream_stats_pending = 0;                 // last query was streamed: h_stats[2] = out of domain
 };
 
 // workspace slot map (Ctx::ws)
@@ -128,6 +135,7 @@ enum : int {
     kWsPRCount, kWsPROff, kWsPRCursor, kWsTvals, kWsSpanCount, kWsSpanOff, kWsSpans,
     kWsPieceCount, kWsPieceOff, kWsPieceCursor, kWsPieces, kWsMask, kWsBandCount, kWsBandOff,
     kWsWork, kWsSizes,
+    kWsLab, kWsRowCount, kWsRowOff, kWsRowCursor, kWsRowSpans, kWsStream,   // streamed query
     kWsScan = 44,                           // 44..63 recursive scan temporaries
 };
 
@@ -151,6 +159,16 @@ rj_status items_for_level(Ctx *c, int L);
 void free_load_scratch(Ctx *c);
 void drop_items(Ctx *c);
 int choose_level(int W, int H, int target_side);
+
+// api.cu
+rj_status build_filter(Ctx *c, const rj_query_desc *q, int n_cols, const int *col_dtype, Filter &f);
+
+// stream.cu: the streamed one-shot query (rj_query_stream); partials into
+// d_cnt / d_sum (device), stream-ordered on c->stream.
+rj_status stream_query_impl(Ctx *c, const Filter &f, bool sum, int W, int H, int mode, uint64_t n,
+                            const void *x, const void *y, bool xy_f64, const void *const *cols,
+                            unsigned long long *d_cnt, double *d_sum);
+void stream_release(Ctx *c);
 
 // polygons.cu
 rj_status load_polygons_impl(Ctx *c, uint32_t n_poly, const uint32_t *pro, const uint32_t *rvo,

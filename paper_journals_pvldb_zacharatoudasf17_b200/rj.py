@@ -6,7 +6,7 @@ There is no fallback: if librj.so is missing or no sm_100 device is present
 the calls raise.
 
     rj_create, rj_destroy, rj_load_points, rj_load_polygons, rj_query,
-    rj_query_device, rj_finalize_device, rj_resolve_canvas(_domain),
+    rj_query_device, rj_query_stream, rj_finalize_device, rj_resolve_canvas(_domain),
     rj_debug_pixel_spans, rj_debug_boundary_mask, rj_debug_point_membership,
     rj_get_stats, rj_set_option  -- same names as the C ABI.
 
@@ -29,7 +29,7 @@ AGG = {"count": 0, "sum": 1, "avg": 2}
 MODE = {"bounded": 0, "accurate": 1, "index": 2, "exact": 3}
 OPS = {"<": 0, "<=": 1, ">": 2, ">=": 3, "==": 4}
 DT_I32, DT_F32, DT_F64 = 0, 1, 2
-OPT_TIMING, OPT_CHUNK, OPT_PASS, OPT_KEEP_LOAD_SCRATCH, OPT_TILE_SIDE, OPT_STAGES = 1, 2, 3, 4, 5, 6
+OPT_TIMING, OPT_CHUNK, OPT_PASS, OPT_KEEP_LOAD_SCRATCH, OPT_TILE_SIDE, OPT_STAGES, OPT_STREAM_BATCH = 1, 2, 3, 4, 5, 6, 7
 MAX_PRED = 5
 
 
@@ -82,6 +82,7 @@ def lib():
             "rj_load_polygons": (i32, [vp, u32, vp, vp, vp, vp]),
             "rj_query": (i32, [vp, qp, vp, vp]),
             "rj_query_device": (i32, [vp, qp, vp, vp]),
+            "rj_query_stream": (i32, [vp, qp, u64, vp, vp, i32, i32, vp, vp, vp, vp]),
             "rj_finalize_device": (i32, [vp, i32, u32, vp, vp, vp]),
             "rj_resolve_canvas": (i32, [vp, qp, ctypes.POINTER(i32), ctypes.POINTER(i32)]),
             "rj_resolve_canvas_domain": (i32, [d, d, d, d, qp, ctypes.POINTER(i32), ctypes.POINTER(i32)]),
@@ -105,7 +106,7 @@ def lib():
 
 
 EXPORTS = ["rj_create", "rj_destroy", "rj_set_allocator", "rj_load_points", "rj_load_polygons", "rj_query",
-           "rj_query_device", "rj_finalize_device", "rj_resolve_canvas", "rj_resolve_canvas_domain",
+           "rj_query_device", "rj_query_stream", "rj_finalize_device", "rj_resolve_canvas", "rj_resolve_canvas_domain",
            "rj_debug_pixel_spans", "rj_debug_boundary_mask", "rj_debug_point_membership", "rj_get_stats",
            "rj_set_option", "rj_n_polygons", "rj_n_points", "rj_status_str", "rj_last_error", "rj_version"]
 
@@ -186,6 +187,14 @@ def rj_load_polygons(ctx, flat):
 
 def rj_query(ctx, desc, count=None, value=None):
     _check(lib().rj_query(ctx, ctypes.byref(desc), _ptr(count), _ptr(value)), ctx)
+
+
+def rj_query_stream(ctx, desc, x, y, cols=(), count=None, value=None):
+    n = len(x)
+    ptrs = (ctypes.c_void_p * max(1, len(cols)))(*[_ptr(c) for c in cols])
+    dts = (ctypes.c_int32 * max(1, len(cols)))(*[_dtype_code(c) for c in cols])
+    _check(lib().rj_query_stream(ctx, ctypes.byref(desc), n, _ptr(x), _ptr(y), _dtype_code(x), len(cols), ptrs, dts,
+                                 _ptr(count), _ptr(value)), ctx)
 
 
 def rj_query_device(ctx, desc, d_count, d_sum=None):
@@ -273,6 +282,15 @@ class RasterJoin:
         cnt = np.zeros(self.n_poly, dtype=np.uint64)
         val = np.zeros(self.n_poly, dtype=np.float64)
         rj_query(self.ctx, q, cnt, val)
+        return cnt, val
+
+    def query_stream(self, x, y, cols=(), **kw):
+        """Streamed one-shot query over points that are not loaded (host or
+        device arrays, read once in batches).  Returns (count, value)."""
+        q = make_desc(**kw)
+        cnt = np.zeros(self.n_poly, dtype=np.uint64)
+        val = np.zeros(self.n_poly, dtype=np.float64)
+        rj_query_stream(self.ctx, q, x, y, cols, cnt, val)
         return cnt, val
 
     def stats(self):

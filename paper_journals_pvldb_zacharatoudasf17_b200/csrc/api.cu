@@ -242,7 +242,8 @@ static rj_status check_ready(Ctx *c, const rj_query_desc *q) {
 }
 
 // Everything up to (not including) the point-pass launch.
-static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_polygon_pass = true) {
+static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_polygon_pass = true,
+                         bool bands = false) {
     rj_status s = check_ready(c, q);
     if (s != RJ_OK) return s;
     if ((s = resolve(c->x0, c->y0, c->x1, c->y1, q, &P.W, &P.H)) != RJ_OK)
@@ -278,7 +279,8 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[0], c->stream));
     // the index join needs neither spans nor the boundary mask
     P.pp = PolyPass{};
-    if (need_polygon_pass && !P.index && (s = polygon_pass(c, P.W, P.H, P.L, P.acc, P.pp)) != RJ_OK) return s;
+    if (need_polygon_pass && !P.index && (s = polygon_pass(c, P.W, P.H, P.L, P.acc || bands, P.pp)) != RJ_OK)
+        return s;
     if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[1], c->stream));
     a.qx = c->qx.as<uint32_t>();
     a.qy = c->qy.as<uint32_t>();
@@ -291,7 +293,7 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     a.cell_off10 = c->cell_off.as<uint32_t>();
     a.piece_off = P.pp.piece_off;
     a.pieces = P.pp.pieces;
-    a.mask = P.pp.mask;
+    a.mask = P.acc ? P.pp.mask : nullptr;
     a.mask_wpr = P.pp.mask_wpr;
     a.index_join = P.index;
     a.grid_off = c->grid_off.as<uint32_t>();
@@ -415,7 +417,7 @@ rj_status rj_destroy(rj_ctx *c) {
     dfree(c, c->edges); dfree(c, c->edge_poly); dfree(c, c->poly_edge_off); dfree(c, c->mbr);
     dfree(c, c->grid_off); dfree(c, c->grid_ent); dfree(c, c->grid_edge); dfree(c, c->grid_poly);
     for (auto &b : c->ws) dfree(c, b);
-    dfree(c, c->res_cnt); dfree(c, c->res_sum); dfree(c, c->res_val);
+    dfree(c, c->res_cnt); dfree(c, c->res_sum); dfree(c, c->res_val); dfree(c, c->res_eps);
     stream_release(c);
     for (auto &e : c->ev) if (e) cudaEventDestroy(e);
     if (c->h_stats) cudaFreeHost(c->h_stats);
@@ -574,6 +576,52 @@ rj_status rj_query_stream(rj_ctx *c, const rj_query_desc *q, uint64_t n, const v
     if (count) RJ_CUDA(c, cudaMemcpyAsync(count, c->res_cnt.p, np * 8, cudaMemcpyDeviceToHost, c->stream));
     if (value) RJ_CUDA(c, cudaMemcpyAsync(value, c->res_val.p, np * 8, cudaMemcpyDeviceToHost, c->stream));
     if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[3], c->stream));
+    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
+    return RJ_OK;
+}
+
+rj_status rj_query_interval(rj_ctx *c, const rj_query_desc *q, uint64_t *count, double *value, uint64_t *eps_plus,
+                            uint64_t *eps_minus) {
+    if (q && q->mode != RJ_BOUNDED) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "result intervals need RJ_BOUNDED");
+    Prepared P;
+    rj_status s = prepare(c, q, P, true, true);
+    if (s != RJ_OK) return s;
+    const size_t n = c->n_poly;
+    Buf &cv = wsbuf(c, kWsCanvas);
+    if (dreserve(c, c->res_cnt, n * 8) || dreserve(c, c->res_sum, n * 8) || dreserve(c, c->res_val, n * 8) ||
+        dreserve(c, c->res_eps, n * 16) || dreserve(c, cv, (uint64_t)P.W * P.H * 4))
+        return set_error(c, RJ_ERR_OOM, "result allocation failed");
+    RJ_CUDA(c, cudaMemsetAsync(cv.p, 0, (uint64_t)P.W * P.H * 4, c->stream));
+    P.a.canvas = cv.as<uint32_t>();
+    if ((s = run_pass(c, P, c->res_cnt.as<unsigned long long>(), c->res_sum.as<double>())) != RJ_OK) return s;
+    unsigned long long *ep = c->res_eps.as<unsigned long long>(), *em = ep + n;
+    if ((s = interval_impl(c, P.W, P.H, P.pp, cv.as<uint32_t>(), ep, em)) != RJ_OK) return s;
+    if (value) RJ_CUDA(c, launch_finalize(c, q->agg, (uint32_t)n, c->res_cnt.as<unsigned long long>(),
+                                          c->res_sum.as<double>(), c->res_val.as<double>()));
+    if (count) RJ_CUDA(c, cudaMemcpyAsync(count, c->res_cnt.p, n * 8, cudaMemcpyDeviceToHost, c->stream));
+    if (value) RJ_CUDA(c, cudaMemcpyAsync(value, c->res_val.p, n * 8, cudaMemcpyDeviceToHost, c->stream));
+    if (eps_plus) RJ_CUDA(c, cudaMemcpyAsync(eps_plus, ep, n * 8, cudaMemcpyDeviceToHost, c->stream));
+    if (eps_minus) RJ_CUDA(c, cudaMemcpyAsync(eps_minus, em, n * 8, cudaMemcpyDeviceToHost, c->stream));
+    if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[3], c->stream));
+    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
+    return RJ_OK;
+}
+
+rj_status rj_debug_point_canvas(rj_ctx *c, const rj_query_desc *q, uint32_t *counts) {
+    if (!counts || !q) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL counts or query");
+    rj_query_desc qq = *q;
+    qq.mode = RJ_BOUNDED;
+    Prepared P;
+    rj_status s = prepare(c, &qq, P);
+    if (s != RJ_OK) return s;
+    const size_t n = c->n_poly;
+    Buf &cv = wsbuf(c, kWsCanvas);
+    if (dreserve(c, c->res_cnt, n * 8) || dreserve(c, c->res_sum, n * 8) || dreserve(c, cv, (uint64_t)P.W * P.H * 4))
+        return set_error(c, RJ_ERR_OOM, "canvas allocation failed");
+    RJ_CUDA(c, cudaMemsetAsync(cv.p, 0, (uint64_t)P.W * P.H * 4, c->stream));
+    P.a.canvas = cv.as<uint32_t>();
+    if ((s = run_pass(c, P, c->res_cnt.as<unsigned long long>(), c->res_sum.as<double>())) != RJ_OK) return s;
+    RJ_CUDA(c, cudaMemcpyAsync(counts, cv.p, (uint64_t)P.W * P.H * 4, cudaMemcpyDeviceToHost, c->stream));
     RJ_CUDA(c, cudaStreamSynchronize(c->stream));
     return RJ_OK;
 }

@@ -125,6 +125,18 @@ __device__ __forceinline__ void process(const PassArgs &a, const Shared &sh, con
     emit_pixel_run<SUM>(t, key[kIPL - 1], run + (add_pre ? pre : 0u), dsum + (add_pre ? dpre : 0.0), !cout);
 }
 
+// Result intervals: add the cell's per-pixel filtered counts to the global
+// count canvas (a heavy cell split over several work items adds partials).
+__device__ __forceinline__ void dump_canvas(const PassArgs &a, const Tile &t, uint32_t cell, int s_lat) {
+    const int64_t cx = cell_x(cell), cy = cell_y(cell);
+    const uint32_t c0 = (uint32_t)pix(cx << s_lat, a.W), r0 = (uint32_t)pix(cy << s_lat, a.H);
+    for (uint32_t i = threadIdx.x; i < t.th * t.stride; i += kThreads) {
+        const uint32_t r = i / t.stride, x = i - r * t.stride;
+        const uint32_t v = t.cnt[i] & ~kFlag;
+        if (x < t.tw && v) atomicAdd(&a.canvas[(uint64_t)(r0 + r) * a.W + c0 + x], v);
+    }
+}
+
 template <bool SUM, bool ACC, int NS, bool FP>
 __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a) {
     extern __shared__ __align__(128) unsigned char smem_raw[];
@@ -221,6 +233,7 @@ __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a)
                 // ---- last stage of the cell: reduce the tile over the span pieces (S4)
                 if (ACC && qn) drain_queue<SUM>(a, sh, qn, true);
                 consumers_sync();                          // every point of the cell is in the tile
+                if (a.canvas) dump_canvas(a, t, m.cell, s_lat);
                 for (uint32_t kk = pb + threadIdx.x; kk < pe; kk += kThreads) {
                     const uint2 pc = (kk == pb + threadIdx.x) ? pc0 : __ldg(&a.pieces[kk]);
                     const uint32_t lr = pc.y & 255u, lo = (pc.y >> 8) & 255u, hi = pc.y >> 16;
@@ -334,20 +347,20 @@ rj_status launch_pass(Ctx *c, void *k, const PassArgs &a, size_t smem) {
 // Kernel choice: COUNT always uses the pixel tile (cheapest per cell); SUM/AVG
 // uses polygon labels in bounded mode (no per-pixel fp64 atomics) and the
 // pixel tile in accurate mode (measured faster at C3); RJ_OPT_PASS overrides.
-static bool use_label(const Ctx *c, bool sum, bool accurate) {
-    if (!sum) return false;
+static bool use_label(const Ctx *c, const PassArgs &a, bool sum, bool accurate) {
+    if (!sum || a.canvas) return false;              // the count canvas comes from the pixel tiles
     if (c->pass_variant >= 0) return c->pass_variant == 0;
     return !accurate;
 }
 
 size_t point_pass_smem(const Ctx *c, const PassArgs &a, bool sum, bool accurate) {
-    return use_label(c, sum, accurate) ? point_pass_label_smem(a, accurate) : tile_pass_smem(a, sum, accurate);
+    return use_label(c, a, sum, accurate) ? point_pass_label_smem(a, accurate) : tile_pass_smem(a, sum, accurate);
 }
 
 int point_pass_stages(int n_slots) { return (2 + n_slots) <= 4 ? 3 : 2; }
 
 rj_status point_pass(Ctx *c, const PassArgs &a_in, bool sum, bool accurate) {
-    if (use_label(c, sum, accurate)) return point_pass_label(c, a_in, accurate);
+    if (use_label(c, a_in, sum, accurate)) return point_pass_label(c, a_in, accurate);
     PassArgs a = a_in;
     a.n_stages = (uint32_t)choose_stages(a, tile_pass_smem, sum, accurate, c->force_stages);
     if (!a.n_stages) return set_error(c, RJ_ERR_RESOLUTION, "point-pass tiles do not fit in shared memory");

@@ -102,7 +102,7 @@ __global__ void k_edge_rows(const int4 *__restrict__ edges, uint32_t n_edges, in
     rows[e] = (uint32_t)(row_start(ymax, H) - row_start(ymin, H));
     if (accurate) {
         // S5 row bands: pixel rows whose closed lattice extent meets [ymin, ymax]
-        bands[e] = ymin >= kOne ? 0u : (uint32_t)(pix(ymax < kOne - 1 ? ymax : kOne - 1, H) - pix(ymin, H) + 1);
+        bands[e] = (uint32_t)band_rows(ymin, ymax, H);
     }
 }
 
@@ -233,25 +233,9 @@ __global__ void k_mask_mark(const int4 *__restrict__ edges, const uint32_t *__re
     for (uint32_t j = blockIdx.x * blockDim.x + threadIdx.x; j < total; j += gridDim.x * blockDim.x) {
         const uint32_t e = upper_bound_u32(band_off, n_edges + 1, j) - 1;
         const int4 E = edges[e];
-        const int64_t xa = E.x, ya = E.y, xb = E.z, yb = E.w;
-        const int64_t ymin = min(ya, yb), ymax = max(ya, yb);
-        const int64_t r = pix(ymin, H) + (j - band_off[e]);
-        const int64_t ylo = max(qlo(r, H), ymin), yhi = min(qhi(r, H), ymax);
-        int64_t cl, fr;   // ceil of the left x-extent, floor of the right one
-        if (ya == yb) {
-            cl = min(xa, xb);
-            fr = max(xa, xb);
-        } else {
-            int64_t d = yb - ya, dx = xb - xa, base = xa * d;
-            int64_t n1 = base + dx * (ylo - ya), n2 = base + dx * (yhi - ya);
-            if (d < 0) { d = -d; n1 = -n1; n2 = -n2; }
-            cl = min(ceil_div(n1, d), ceil_div(n2, d));
-            fr = max(floor_div(n1, d), floor_div(n2, d));
-        }
-        if (cl >= kOne) continue;
-        fr = min(fr, kOne - 1);
-        if (fr < cl) continue;                    // passes between two pixels' lattice extents
-        const int64_t i0 = pix(cl, W), i1 = pix(fr, W);
+        const int64_t r = pix(min(E.y, E.w), H) + (j - band_off[e]);
+        int64_t i0, i1;
+        if (!supercover_cols(E.x, E.y, E.z, E.w, r, W, H, i0, i1)) continue;
         uint32_t *row = mask + (uint64_t)r * wpr;
         for (int64_t w = i0 >> 5; w <= (i1 >> 5); ++w) {
             const int64_t a = max(i0, w << 5) - (w << 5), b = min(i1, (w << 5) + 31) - (w << 5);
@@ -469,6 +453,7 @@ rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp)
     pp.pieces = pieces.as<uint2>();
     if (accurate) {
         const uint32_t B = hs[2];
+        pp.n_bands = B;
         const uint32_t wpr = (uint32_t)((W + 31) / 32);
         Buf &mask = wsbuf(c, kWsMask);
         if (dreserve(c, mask, (uint64_t)wpr * H * 4)) return set_error(c, RJ_ERR_OOM, "mask allocation failed");

@@ -98,4 +98,40 @@ RJ_HD uint32_t cell_y(uint32_t c) { return compact16(c >> 1); }
 RJ_HD int64_t cell_pix_lo(int64_t cc, int64_t n, int L) { return pix(cc << (kLatticeBits - L), n); }
 RJ_HD int64_t cell_pix_hi(int64_t cc, int64_t n, int L) { return pix(((cc + 1) << (kLatticeBits - L)) - 1, n); }
 
+// S5 supercover (reading Z7, O-S): pixel columns [i0, i1] of row r touched by
+// edge (xa,ya)-(xb,yb): clip the segment to the row's closed lattice band
+// y in [max(qlo(r), ymin), min(qhi(r), ymax)], take the ceil of its left and
+// the floor of its right x-extent, exclude coordinate 2^30.  False when the
+// edge passes between two pixels' lattice extents.
+RJ_HD bool supercover_cols(int64_t xa, int64_t ya, int64_t xb, int64_t yb, int64_t r, int64_t W, int64_t H,
+                           int64_t &i0, int64_t &i1) {
+    const int64_t ymin = ya < yb ? ya : yb, ymax = ya < yb ? yb : ya;
+    const int64_t ql = qlo(r, H), qh = qhi(r, H);
+    const int64_t ylo = ql > ymin ? ql : ymin, yhi = qh < ymax ? qh : ymax;
+    int64_t cl, fr;
+    if (ya == yb) {
+        cl = xa < xb ? xa : xb;
+        fr = xa < xb ? xb : xa;
+    } else {
+        int64_t d = yb - ya, dx = xb - xa, base = xa * d;
+        int64_t n1 = base + dx * (ylo - ya), n2 = base + dx * (yhi - ya);
+        if (d < 0) { d = -d; n1 = -n1; n2 = -n2; }
+        const int64_t c1 = ceil_div(n1, d), c2 = ceil_div(n2, d), f1 = floor_div(n1, d), f2 = floor_div(n2, d);
+        cl = c1 < c2 ? c1 : c2;
+        fr = f1 > f2 ? f1 : f2;
+    }
+    if (cl >= kOne) return false;
+    if (fr > kOne - 1) fr = kOne - 1;
+    if (fr < cl) return false;
+    i0 = pix(cl, W);
+    i1 = pix(fr, W);
+    return true;
+}
+
+// Rows of the supercover band of an edge / polygon with y-extent [ymin, ymax]:
+// [pix(ymin), pix(min(ymax, 2^30 - 1))], none when ymin >= 2^30.
+RJ_HD int64_t band_rows(int64_t ymin, int64_t ymax, int64_t H) {
+    return ymin >= kOne ? 0 : pix(ymax < kOne - 1 ? ymax : kOne - 1, H) - pix(ymin, H) + 1;
+}
+
 }  // namespace rj

@@ -67,6 +67,7 @@ struct PassArgs {
     uint32_t tile_cap;            // words of the CTA's tile
     uint32_t n_stages;            // depth of the shared-memory stage ring
     int32_t index_join;           // every pixel is a boundary pixel, no span pieces (RJ_INDEX_JOIN)
+    uint32_t *canvas;             // tile kernel: dump per-pixel filtered counts (W x H) when set
     unsigned long long *stats;    // [0] filtered, [1] boundary
 };
 
@@ -108,8 +109,9 @@ struct Ctx {
     uint64_t n_grid_ent = 0;
 
     // query workspace (grow-only)
-    Buf ws[64];                      // slots: see kWs* in rj_internal.cuh
+    Buf ws[96];                      // slots: see kWs* in rj_internal.cuh
     Buf res_cnt, res_sum, res_val;   // per-polygon partials / values
+    Buf res_eps;                     // result intervals: eps+ [n_poly], eps- [n_poly]
     Buf stats_dev;
     unsigned long long *h_stats = nullptr;   // pinned
     rj_stats last{};
@@ -136,7 +138,8 @@ enum : int {
     kWsPieceCount, kWsPieceOff, kWsPieceCursor, kWsPieces, kWsMask, kWsBandCount, kWsBandOff,
     kWsWork, kWsSizes,
     kWsLab, kWsRowCount, kWsRowOff, kWsRowCursor, kWsRowSpans, kWsStream,   // streamed query
-    kWsScan = 44,                           // 44..63 recursive scan temporaries
+    kWsCanvas, kWsBRowCount, kWsBRowOff, kWsBktCount, kWsBktOff, kWsBktCursor, kWsBktRanges,   // intervals
+    kWsScan = 72,                           // 72..95 recursive scan temporaries
 };
 
 // allocation helpers (ctx allocator if set)
@@ -170,11 +173,12 @@ rj_status stream_query_impl(Ctx *c, const Filter &f, bool sum, int W, int H, int
                             unsigned long long *d_cnt, double *d_sum);
 void stream_release(Ctx *c);
 
+
 // polygons.cu
 rj_status load_polygons_impl(Ctx *c, uint32_t n_poly, const uint32_t *pro, const uint32_t *rvo,
                              const double *vx, const double *vy);
 struct PolyPass {
-    uint64_t n_cross = 0, n_spans = 0, n_pieces = 0;
+    uint64_t n_cross = 0, n_spans = 0, n_pieces = 0, n_bands = 0;
     uint32_t *spans = nullptr;       // 4 x u32 per span (poly,row,lo,hi), (poly,row,lo)-sorted
     uint32_t *piece_off = nullptr;   // [4^L + 1]
     uint2 *pieces = nullptr;
@@ -182,6 +186,11 @@ struct PolyPass {
     uint32_t mask_wpr = 0;
 };
 rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp);
+
+// interval.cu: bounded-mode worst-case result intervals from the
+// per-pixel count canvas, the spans and the S5 bands of the polygon pass.
+rj_status interval_impl(Ctx *c, int W, int H, const PolyPass &pp, const uint32_t *canvas,
+                        unsigned long long *d_eps_plus, unsigned long long *d_eps_minus);
 
 // pass.cu
 rj_status point_pass(Ctx *c, const PassArgs &a, bool sum, bool accurate);

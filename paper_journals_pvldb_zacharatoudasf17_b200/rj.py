@@ -6,8 +6,8 @@ There is no fallback: if librj.so is missing or no sm_100 device is present
 the calls raise.
 
     rj_create, rj_destroy, rj_load_points, rj_load_polygons, rj_query,
-    rj_query_device, rj_query_stream, rj_finalize_device, rj_resolve_canvas(_domain),
-    rj_debug_pixel_spans, rj_debug_boundary_mask, rj_debug_point_membership,
+    rj_query_device, rj_query_stream, rj_query_interval, rj_finalize_device, rj_resolve_canvas(_domain),
+    rj_debug_pixel_spans, rj_debug_boundary_mask, rj_debug_point_membership, rj_debug_point_canvas,
     rj_get_stats, rj_set_option  -- same names as the C ABI.
 
 `RasterJoin` wraps a context with a Pythonic API.
@@ -83,6 +83,8 @@ def lib():
             "rj_query": (i32, [vp, qp, vp, vp]),
             "rj_query_device": (i32, [vp, qp, vp, vp]),
             "rj_query_stream": (i32, [vp, qp, u64, vp, vp, i32, i32, vp, vp, vp, vp]),
+            "rj_query_interval": (i32, [vp, qp, vp, vp, vp, vp]),
+            "rj_debug_point_canvas": (i32, [vp, qp, vp]),
             "rj_finalize_device": (i32, [vp, i32, u32, vp, vp, vp]),
             "rj_resolve_canvas": (i32, [vp, qp, ctypes.POINTER(i32), ctypes.POINTER(i32)]),
             "rj_resolve_canvas_domain": (i32, [d, d, d, d, qp, ctypes.POINTER(i32), ctypes.POINTER(i32)]),
@@ -106,7 +108,7 @@ def lib():
 
 
 EXPORTS = ["rj_create", "rj_destroy", "rj_set_allocator", "rj_load_points", "rj_load_polygons", "rj_query",
-           "rj_query_device", "rj_query_stream", "rj_finalize_device", "rj_resolve_canvas", "rj_resolve_canvas_domain",
+           "rj_query_device", "rj_query_stream", "rj_query_interval", "rj_debug_point_canvas", "rj_finalize_device", "rj_resolve_canvas", "rj_resolve_canvas_domain",
            "rj_debug_pixel_spans", "rj_debug_boundary_mask", "rj_debug_point_membership", "rj_get_stats",
            "rj_set_option", "rj_n_polygons", "rj_n_points", "rj_status_str", "rj_last_error", "rj_version"]
 
@@ -195,6 +197,18 @@ def rj_query_stream(ctx, desc, x, y, cols=(), count=None, value=None):
     dts = (ctypes.c_int32 * max(1, len(cols)))(*[_dtype_code(c) for c in cols])
     _check(lib().rj_query_stream(ctx, ctypes.byref(desc), n, _ptr(x), _ptr(y), _dtype_code(x), len(cols), ptrs, dts,
                                  _ptr(count), _ptr(value)), ctx)
+
+
+def rj_query_interval(ctx, desc, count=None, value=None, eps_plus=None, eps_minus=None):
+    _check(lib().rj_query_interval(ctx, ctypes.byref(desc), _ptr(count), _ptr(value), _ptr(eps_plus),
+                                   _ptr(eps_minus)), ctx)
+
+
+def rj_debug_point_canvas(ctx, desc):
+    W, H = rj_resolve_canvas(ctx, desc)
+    out = np.zeros((H, W), dtype=np.uint32)
+    _check(lib().rj_debug_point_canvas(ctx, ctypes.byref(desc), _ptr(out)), ctx)
+    return out
 
 
 def rj_query_device(ctx, desc, d_count, d_sum=None):
@@ -292,6 +306,16 @@ class RasterJoin:
         val = np.zeros(self.n_poly, dtype=np.float64)
         rj_query_stream(self.ctx, q, x, y, cols, cnt, val)
         return cnt, val
+
+    def query_interval(self, **kw):
+        """Bounded query with worst-case intervals: (count, value, eps_plus, eps_minus)."""
+        q = make_desc(**kw)
+        out = [np.zeros(self.n_poly, dtype=t) for t in (np.uint64, np.float64, np.uint64, np.uint64)]
+        rj_query_interval(self.ctx, q, *out)
+        return tuple(out)
+
+    def point_canvas(self, **kw):
+        return rj_debug_point_canvas(self.ctx, make_desc(**kw))
 
     def stats(self):
         return rj_get_stats(self.ctx)

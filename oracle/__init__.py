@@ -54,6 +54,9 @@ def lib():
         L.or_query.restype = u64
         L.or_query.argtypes = [vp, u64, vp, vp, i32, d, d, d, d, i32, vp, vp, i32, i32, vp, vp, vp,
                                i32, i32, i32, i32, vp, vp]
+        L.or_query_minmax.restype = None
+        L.or_query_minmax.argtypes = [vp, u64, vp, vp, i32, d, d, d, d, i32, vp, vp, i32, i32, vp, vp, vp,
+                                      i32, i32, i32, vp, vp]
         L.or_avg.restype = None
         L.or_avg.argtypes = [i64, vp, vp, vp]
         L.or_membership.restype = None
@@ -145,6 +148,18 @@ def query(polys, x, y, cols=(), preds=(), agg_col=-1, W=1024, H=1024, mode="boun
                           int(agg_col), *c.pargs(), int(W), int(H), 0 if mode == "bounded" else 1,
                           int(nthreads), cnt.ctypes.data, s.ctypes.data)
     return cnt, s, int(kept)
+
+
+def query_minmax(polys, x, y, cols, agg_col, preds=(), W=1024, H=1024, mode="bounded"):
+    """O11: (min f64[n_poly], max f64[n_poly]) of column agg_col, NaN for empty polygons."""
+    x, y, f64 = _xy(x, y)
+    c = _Cols(cols, preds)
+    mn = np.zeros(polys.n, dtype=np.float64)
+    mx = np.zeros(polys.n, dtype=np.float64)
+    lib().or_query_minmax(polys.h, len(x), x.ctypes.data, y.ctypes.data, f64, *polys.box, *c.args(),
+                          int(agg_col), *c.pargs(), int(W), int(H), 0 if mode == "bounded" else 1,
+                          mn.ctypes.data, mx.ctypes.data)
+    return mn, mx
 
 
 def avg(cnt, s):

@@ -34,6 +34,11 @@
  *   O9  boundary pixel: the segment meets the closed lattice rectangle of
  *       the pixel ("draw the outline", conservative raster P:880-887).
  *   O10 worst-case interval [A - e+, A + e-] over boundary pixels.
+ *   O11 MIN / MAX (distributive; multiple aggregates P:1278-1283):
+ *       the least / greatest attribute value of the polygon's points under
+ *       IEEE 754 totalOrder for float32 (-NaN < -inf < ... < -0 < +0 < ...
+ *       < +inf < +NaN, NaNs further ordered by payload; reading Z16), plain
+ *       order for int32; NaN result for a polygon without points.
  */
 #include <math.h>
 #include <stdint.h>
@@ -311,6 +316,76 @@ OR_EXPORT uint64_t or_query(const or_polys *p, uint64_t n, const void *x, const 
     for (int t = 0; t < nt; ++t) kept += tkept[t];
     free(tc); free(ts); free(tk); free(tkept);
     return kept;
+}
+
+/* O11: IEEE 754-2008 section 5.10 totalOrder(a, b) restricted to "a < b"
+ * for binary32, written from the definition: numeric order first; equal
+ * numbers are ordered by sign (-0 < +0); a NaN with the sign bit set is
+ * below every number and a NaN without it above; two NaNs of one sign are
+ * ordered by payload, larger payloads lying farther from zero. */
+static int or_total_less_f32(float a, float b) {
+    uint32_t ba, bb;
+    memcpy(&ba, &a, 4);
+    memcpy(&bb, &b, 4);
+    const int sa = (ba >> 31) & 1, sb = (bb >> 31) & 1;
+    const int na = isnan(a), nb = isnan(b);
+    if (!na && !nb) {
+        if (a < b) return 1;
+        if (a > b) return 0;
+        return sa && !sb;                        /* -0 < +0; equal otherwise */
+    }
+    if (na && nb) {
+        if (sa != sb) return sa;                 /* -NaN < +NaN */
+        const uint32_t pa = ba & 0x007FFFFFu, pb = bb & 0x007FFFFFu;
+        return sa ? pa > pb : pa < pb;
+    }
+    if (na) return sa;                           /* -NaN below all, +NaN above all */
+    return !sb;                                  /* b is NaN: a < +NaN, a > -NaN */
+}
+
+/* O11: per polygon MIN and MAX of attribute column agg_col (int32 or
+ * float32) over the filtered points counted in the polygon under `mode`
+ * (O5 / O6, as or_query).  mn / mx receive the value as binary64 (exact for
+ * both dtypes), NaN for a polygon without points.  Sequential. */
+OR_EXPORT void or_query_minmax(const or_polys *p, uint64_t n, const void *x, const void *y, int xy_f64,
+                               double x0, double y0, double x1, double y1,
+                               int n_cols, const void *const *cols, const int *dtypes,
+                               int agg_col, int n_pred, const int *pcol, const int *pop,
+                               const double *pval, int W, int H, int mode, double *mn, double *mx) {
+    or_filter f = {n_cols, cols, dtypes, n_pred, pcol, pop, pval};
+    const int64_t np = p->n_poly;
+    const int is_f32 = dtypes[agg_col] == OR_F32;
+    uint8_t *seen = (uint8_t *)calloc((size_t)np, 1);
+    int32_t *imn = (int32_t *)calloc((size_t)np, 4), *imx = (int32_t *)calloc((size_t)np, 4);
+    float *fmn = (float *)calloc((size_t)np, 4), *fmx = (float *)calloc((size_t)np, 4);
+    for (uint64_t i = 0; i < n; ++i) {
+        int64_t qx, qy;
+        if (!or_point_q(x, y, xy_f64, i, x0, y0, x1, y1, &qx, &qy)) continue;
+        if (!or_pass(&f, i)) continue;
+        int64_t px = qx, py = qy;
+        if (mode == 0) {
+            px = or_centre(or_pixel(qx, W), W);
+            py = or_centre(or_pixel(qy, H), H);
+        }
+        for (int64_t P = 0; P < np; ++P) {
+            if (!or_contains(p, P, px, py)) continue;
+            if (is_f32) {
+                const float v = ((const float *)cols[agg_col])[i];
+                if (!seen[P] || or_total_less_f32(v, fmn[P])) fmn[P] = v;
+                if (!seen[P] || or_total_less_f32(fmx[P], v)) fmx[P] = v;
+            } else {
+                const int32_t v = ((const int32_t *)cols[agg_col])[i];
+                if (!seen[P] || v < imn[P]) imn[P] = v;
+                if (!seen[P] || v > imx[P]) imx[P] = v;
+            }
+            seen[P] = 1;
+        }
+    }
+    for (int64_t P = 0; P < np; ++P) {
+        mn[P] = !seen[P] ? NAN : is_f32 ? (double)fmn[P] : (double)imn[P];
+        mx[P] = !seen[P] ? NAN : is_f32 ? (double)fmx[P] : (double)imx[P];
+    }
+    free(seen); free(imn); free(imx); free(fmn); free(fmx);
 }
 
 /* O7: AVG = SUM / COUNT, NaN for an empty polygon. */

@@ -403,3 +403,71 @@ def test_boundary_mask_brute_force_tiny():
                 for px in xs:
                     for py in ys:
                         assert polys.pnpoly(0, px, py) == c
+
+
+# ---------------------------------------------------------------------- O11
+def _minmax_brute(P, x, y, cols, agg_col, W, mode):
+    """Per-polygon min / max from the (separately pinned) membership bits and
+    numpy: the aggregation step of O11 checked by brute force."""
+    bits = oracle.membership(P, x, y, cols=cols, W=W, H=W, mode=mode)
+    v = cols[agg_col]
+    mn = np.full(P.n, np.nan)
+    mx = np.full(P.n, np.nan)
+    for p in range(P.n):
+        sel = ((bits >> np.uint64(p)) & np.uint64(1)).astype(bool)
+        if sel.any():
+            mn[p] = v[sel].min()
+            mx[p] = v[sel].max()
+    return mn, mx
+
+
+@pytest.mark.parametrize("mode", ["bounded", "accurate"])
+def test_minmax_brute_force(mode):
+    polys = C.polygon_set("c1b")                  # overlaps + holes
+    P = oracle.Polys(PG.flatten(polys), C1)
+    pts = C.c1_points(20000)
+    x, y = pts["x"], pts["y"]
+    rng = np.random.default_rng(41)
+    ti = rng.integers(-2**31, 2**31 - 1, len(x), dtype=np.int64).astype(np.int32)
+    ti[:3] = [-2**31, 2**31 - 1, 0]
+    tf = rng.normal(0, 1e6, len(x)).astype(np.float32)
+    cols = [ti, tf]
+    for col in (0, 1):
+        mn, mx = oracle.query_minmax(P, x, y, cols, col, W=64, H=64, mode=mode)
+        bmn, bmx = _minmax_brute(P, x, y, cols, col, 64, mode)
+        assert np.array_equal(mn, bmn, equal_nan=True), col
+        assert np.array_equal(mx, bmx, equal_nan=True), col
+    # invariant with O7: min <= avg <= max on non-empty polygons
+    cnt, s, _ = oracle.query(P, x, y, cols=cols, agg_col=1, W=64, H=64, mode=mode)
+    a = oracle.avg(cnt, s)
+    mn, mx = oracle.query_minmax(P, x, y, cols, 1, W=64, H=64, mode=mode)
+    ne = cnt > 0
+    assert np.all(mn[ne] <= a[ne] * (1 + 1e-12) + 1e-9) and np.all(a[ne] <= mx[ne] * (1 + 1e-12) + 1e-9)
+    assert np.all(np.isnan(mn[~ne])) and np.all(np.isnan(mx[~ne]))
+
+
+def test_minmax_total_order_special_values():
+    # one unit square holding every point; IEEE 754 totalOrder on binary32
+    sq = [[np.array([(0.0, 0.0), (4.0, 0.0), (4.0, 4.0), (0.0, 4.0)])]]
+    far = [[np.array([(100.0, 100.0), (101.0, 100.0), (101.0, 101.0), (100.0, 101.0)])]]   # empty
+    P = _lattice_polys(sq + far)
+    neg_nan = np.frombuffer(np.uint32(0xFFC00000).tobytes(), np.float32)[0]
+    cases = [
+        ([0.0, -0.0], (-0.0, 0.0)),              # -0 < +0
+        ([1.0, np.nan, -5.0], (-5.0, np.nan)),  # +NaN above everything
+        ([neg_nan, 3.0], (neg_nan, 3.0)),       # -NaN below everything
+        ([-np.inf, np.inf, 7.0], (-np.inf, np.inf)),
+        ([2.5], (2.5, 2.5)),
+    ]
+    for vals, (emn, emx) in cases:
+        k = len(vals)
+        x = np.full(k, 1.5)
+        y = np.full(k, 1.5)
+        v = np.asarray(vals, np.float32)
+        mn, mx = oracle.query_minmax(P, x, y, [v], 0, W=8, H=8, mode="accurate")
+        for got, exp in ((mn[0], emn), (mx[0], emx)):
+            if np.isnan(exp):
+                assert np.isnan(got) and np.signbit(got) == np.signbit(exp), vals
+            else:
+                assert got == exp and np.signbit(got) == np.signbit(exp), vals
+        assert np.isnan(mn[1]) and np.isnan(mx[1])          # polygon without points

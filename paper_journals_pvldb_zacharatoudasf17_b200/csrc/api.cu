@@ -116,7 +116,7 @@ static void int_range(int op, double c, int64_t &lo, int64_t &hi, int &never) {
 rj_status build_filter(Ctx *c, const rj_query_desc *q, int n_cols, const int *col_dtype, Filter &f) {
     f = Filter{};
     if (q->n_pred < 0 || q->n_pred > RJ_MAX_PRED) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "n_pred must be in [0, 5]");
-    if (q->agg < RJ_COUNT || q->agg > RJ_AVG) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad agg");
+    if (q->agg < RJ_COUNT || q->agg > RJ_MAX) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad agg");
     if (q->mode < RJ_BOUNDED || q->mode > RJ_EXACT) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad mode");
     for (int k = 0; k < q->n_pred; ++k) {
         const rj_pred &p = q->pred[k];
@@ -335,6 +335,80 @@ static rj_status run_pass(Ctx *c, Prepared &P, unsigned long long *d_cnt, double
     return RJ_OK;
 }
 
+// Queries served by the label-canvas pass (label_canvas.cu): MIN/MAX,
+// several aggregates, streamed points.  ap = the requested aggregates (may be
+// empty: COUNT only); values[k * n_poly + i] for each of ap (or the count as
+// double when ap is empty).  COUNT entries need no kernel channel.
+static rj_status label_query_with_cols(Ctx *c, const rj_query_desc *q, const AggPlan &ap, const LabInput &in,
+                                       int n_cols, uint64_t *count, double *values) {
+    if (cudaSetDevice(c->device) != cudaSuccess) return set_error(c, RJ_ERR_CUDA, "cudaSetDevice failed");
+    int W, H;
+    rj_status s = resolve(c->x0, c->y0, c->x1, c->y1, q, &W, &H);
+    if (s != RJ_OK) return set_error(c, s, "canvas resolution outside [1, 32768] or bad epsilon");
+    rj_query_desc qf = *q;
+    qf.agg = RJ_COUNT;                        // aggregate columns are read by the plan, not the filter
+    Filter f;
+    if ((s = build_filter(c, &qf, n_cols, in.col_dtype, f)) != RJ_OK) return s;
+    const float f_bnd = boundary_fraction(c, W, H);
+    const int mode = q->mode == RJ_EXACT ? choose_exact(c, W, H, f_bnd, in.n) : q->mode;
+    c->last.mode = mode;
+    c->last.est_boundary_frac = f_bnd;
+    AggPlan kp;                               // kernel channels: the non-COUNT aggregates
+    int slot[kMaxAggs];
+    for (int k = 0; k < ap.n; ++k) {
+        slot[k] = -1;
+        if (ap.kind[k] == RJ_COUNT) continue;
+        slot[k] = kp.n;
+        kp.kind[kp.n] = ap.kind[k];
+        kp.col[kp.n] = ap.col[k];
+        ++kp.n;
+    }
+    const size_t np = c->n_poly;
+    const int nv = std::max(1, ap.n);
+    if (dreserve(c, c->res_cnt, np * 8) || dreserve(c, c->res_agg, (size_t)std::max(1, kp.n) * np * 8) ||
+        dreserve(c, c->res_val, (size_t)nv * np * 8))
+        return set_error(c, RJ_ERR_OOM, "result allocation failed");
+    if ((s = label_query_impl(c, f, kp, W, H, mode, in, c->res_cnt.as<unsigned long long>(), c->res_agg.p)) != RJ_OK)
+        return s;
+    if (values) {
+        for (int k = 0; k < nv; ++k) {
+            AggPlan one;
+            one.n = 1;
+            one.kind[0] = ap.n ? ap.kind[k] : RJ_COUNT;
+            one.col[0] = ap.n ? ap.col[k] : 0;
+            const void *agg = (ap.n && slot[k] >= 0) ? c->res_agg.as<unsigned char>() + (size_t)slot[k] * np * 8
+                                                     : c->res_agg.p;
+            RJ_CUDA(c, launch_finalize_aggs(c, one, in.col_dtype, (uint32_t)np, c->res_cnt.as<unsigned long long>(),
+                                            agg, c->res_val.as<double>() + (size_t)k * np));
+        }
+        RJ_CUDA(c, cudaMemcpyAsync(values, c->res_val.p, (size_t)nv * np * 8, cudaMemcpyDeviceToHost, c->stream));
+    }
+    if (count) RJ_CUDA(c, cudaMemcpyAsync(count, c->res_cnt.p, np * 8, cudaMemcpyDeviceToHost, c->stream));
+    if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[3], c->stream));
+    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
+    return RJ_OK;
+}
+
+static LabInput lattice_input(Ctx *c) {
+    LabInput in;
+    in.lattice = true;
+    in.n = c->n_pts;
+    in.x = c->qx.p;
+    in.y = c->qy.p;
+    in.col_dtype = c->col_dtype;
+    return in;
+}
+
+static AggPlan single_plan(const rj_query_desc *q) {
+    AggPlan ap;
+    if (q->agg != RJ_COUNT) {
+        ap.n = 1;
+        ap.kind[0] = q->agg;
+        ap.col[0] = q->agg_column;
+    }
+    return ap;
+}
+
 }  // namespace rj
 
 using namespace rj;
@@ -417,7 +491,7 @@ rj_status rj_destroy(rj_ctx *c) {
     dfree(c, c->edges); dfree(c, c->edge_poly); dfree(c, c->poly_edge_off); dfree(c, c->mbr);
     dfree(c, c->grid_off); dfree(c, c->grid_ent); dfree(c, c->grid_edge); dfree(c, c->grid_poly);
     for (auto &b : c->ws) dfree(c, b);
-    dfree(c, c->res_cnt); dfree(c, c->res_sum); dfree(c, c->res_val); dfree(c, c->res_eps);
+    dfree(c, c->res_cnt); dfree(c, c->res_sum); dfree(c, c->res_val); dfree(c, c->res_eps); dfree(c, c->res_agg);
     stream_release(c);
     for (auto &e : c->ev) if (e) cudaEventDestroy(e);
     if (c->h_stats) cudaFreeHost(c->h_stats);
@@ -503,6 +577,7 @@ rj_status rj_load_polygons(rj_ctx *c, uint32_t n_poly, const uint32_t *pro, cons
 
 rj_status rj_query_device(rj_ctx *c, const rj_query_desc *q, uint64_t *d_count, double *d_sum) {
     if (!d_count) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL d_count");
+    if (q && q->agg > RJ_AVG) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "rj_query_device: COUNT/SUM/AVG partials only");
     Prepared P;
     rj_status s = prepare(c, q, P);
     if (s != RJ_OK) return s;
@@ -522,6 +597,13 @@ rj_status rj_finalize_device(rj_ctx *c, int32_t agg, uint32_t n, const uint64_t 
 }
 
 rj_status rj_query(rj_ctx *c, const rj_query_desc *q, uint64_t *count, double *value) {
+    if (q && (q->agg == RJ_MIN || q->agg == RJ_MAX)) {       // distributive, label-canvas pass
+        rj_status s = check_ready(c, q);
+        if (s != RJ_OK) return s;
+        if (q->agg_column < 0 || q->agg_column >= c->n_cols)
+            return set_error(c, RJ_ERR_INVALID_ARGUMENT, "agg_column out of range");
+        return label_query_with_cols(c, q, single_plan(q), lattice_input(c), c->n_cols, count, value);
+    }
     Prepared P;
     rj_status s = prepare(c, q, P);
     if (s != RJ_OK) return s;
@@ -555,29 +637,35 @@ rj_status rj_query_stream(rj_ctx *c, const rj_query_desc *q, uint64_t n, const v
         if (n && !cols[k]) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL attribute column");
         dt[k] = dtypes[k];
     }
-    if (cudaSetDevice(c->device) != cudaSuccess) return set_error(c, RJ_ERR_CUDA, "cudaSetDevice failed");
-    int W, H;
-    rj_status s = resolve(c->x0, c->y0, c->x1, c->y1, q, &W, &H);
-    if (s != RJ_OK) return set_error(c, s, "canvas resolution outside [1, 32768] or bad epsilon");
-    Filter f;
-    if ((s = build_filter(c, q, n_cols, dt, f)) != RJ_OK) return s;
-    const float f_bnd = boundary_fraction(c, W, H);
-    const int mode = q->mode == RJ_EXACT ? choose_exact(c, W, H, f_bnd, n) : q->mode;
-    c->last.mode = mode;
-    c->last.est_boundary_frac = f_bnd;
-    const size_t np = c->n_poly;
-    if (dreserve(c, c->res_cnt, np * 8) || dreserve(c, c->res_sum, np * 8) || dreserve(c, c->res_val, np * 8))
-        return set_error(c, RJ_ERR_OOM, "result allocation failed");
-    if ((s = stream_query_impl(c, f, q->agg != RJ_COUNT, W, H, mode, n, x, y, xy_dtype == RJ_F64, cols,
-                               c->res_cnt.as<unsigned long long>(), c->res_sum.as<double>())) != RJ_OK)
-        return s;
-    if (value) RJ_CUDA(c, launch_finalize(c, q->agg, (uint32_t)np, c->res_cnt.as<unsigned long long>(),
-                                          c->res_sum.as<double>(), c->res_val.as<double>()));
-    if (count) RJ_CUDA(c, cudaMemcpyAsync(count, c->res_cnt.p, np * 8, cudaMemcpyDeviceToHost, c->stream));
-    if (value) RJ_CUDA(c, cudaMemcpyAsync(value, c->res_val.p, np * 8, cudaMemcpyDeviceToHost, c->stream));
-    if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[3], c->stream));
-    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
-    return RJ_OK;
+    if (q->agg < RJ_COUNT || q->agg > RJ_MAX) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad agg");
+    if (q->agg != RJ_COUNT && (q->agg_column < 0 || q->agg_column >= n_cols))
+        return set_error(c, RJ_ERR_INVALID_ARGUMENT, "agg_column out of range");
+    LabInput in;
+    in.n = n;
+    in.x = x;
+    in.y = y;
+    in.xy_f64 = xy_dtype == RJ_F64;
+    in.cols = cols;
+    in.col_dtype = dt;
+    return label_query_with_cols(c, q, single_plan(q), in, n_cols, count, value);
+}
+
+rj_status rj_query_multi(rj_ctx *c, const rj_query_desc *q, int32_t n_aggs, const rj_agg_spec *aggs,
+                         uint64_t *count, double *values) {
+    rj_status s = check_ready(c, q);
+    if (s != RJ_OK) return s;
+    if (n_aggs < 1 || n_aggs > RJ_MAX_AGGS || !aggs)
+        return set_error(c, RJ_ERR_INVALID_ARGUMENT, "n_aggs must be in [1, 4]");
+    AggPlan ap;
+    ap.n = n_aggs;
+    for (int k = 0; k < n_aggs; ++k) {
+        if (aggs[k].agg < RJ_COUNT || aggs[k].agg > RJ_MAX) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad agg");
+        if (aggs[k].agg != RJ_COUNT && (aggs[k].column < 0 || aggs[k].column >= c->n_cols))
+            return set_error(c, RJ_ERR_INVALID_ARGUMENT, "aggregate column out of range");
+        ap.kind[k] = aggs[k].agg;
+        ap.col[k] = aggs[k].agg == RJ_COUNT ? 0 : aggs[k].column;
+    }
+    return label_query_with_cols(c, q, ap, lattice_input(c), c->n_cols, count, values);
 }
 
 rj_status rj_query_interval(rj_ctx *c, const rj_query_desc *q, uint64_t *count, double *value, uint64_t *eps_plus,

@@ -112,6 +112,7 @@ struct Ctx {
     Buf ws[96];                      // slots: see kWs* in rj_internal.cuh
     Buf res_cnt, res_sum, res_val;   // per-polygon partials / values
     Buf res_eps;                     // result intervals: eps+ [n_poly], eps- [n_poly]
+    Buf res_agg;                     // label-pass aggregate partials [n_agg][n_poly] x 8 B
     Buf stats_dev;
     unsigned long long *h_stats = nullptr;   // pinned
     rj_stats last{};
@@ -166,11 +167,32 @@ int choose_level(int W, int H, int target_side);
 // api.cu
 rj_status build_filter(Ctx *c, const rj_query_desc *q, int n_cols, const int *col_dtype, Filter &f);
 
-// stream.cu: the streamed one-shot query (rj_query_stream); partials into
-// d_cnt / d_sum (device), stream-ordered on c->stream.
-rj_status stream_query_impl(Ctx *c, const Filter &f, bool sum, int W, int H, int mode, uint64_t n,
-                            const void *x, const void *y, bool xy_f64, const void *const *cols,
-                            unsigned long long *d_cnt, double *d_sum);
+// label_canvas.cu: the label-canvas point pass -- streamed one-shot queries
+// (rj_query_stream), MIN/MAX and multi-aggregate queries (rj_query_multi).
+constexpr int kMaxAggs = 4;
+struct AggPlan {
+    int n = 0;                    // aggregates besides the per-polygon count
+    int kind[kMaxAggs];           // rj_agg
+    int col[kMaxAggs];            // attribute column (user index)
+};
+// Inputs: lattice == true: the context's loaded (quantised, sorted) columns;
+// else n raw points x/y (f32/f64) + user columns, host or device memory.
+struct LabInput {
+    bool lattice = false;
+    uint64_t n = 0;
+    const void *x = nullptr, *y = nullptr;
+    bool xy_f64 = false;
+    const void *const *cols = nullptr;
+    const int *col_dtype = nullptr;
+};
+// Partials (device, caller-sized): d_cnt[n_poly]; d_agg[k * n_poly ...]:
+// binary64 sums for SUM/AVG, orderable u32 keys (in the low half of the
+// 8-byte slot array) for MIN/MAX.
+rj_status label_query_impl(Ctx *c, const Filter &f, const AggPlan &ap, int W, int H, int mode,
+                           const LabInput &in, unsigned long long *d_cnt, void *d_agg);
+// values[k * n + i] from the partials (NaN for an empty polygon's AVG/MIN/MAX).
+cudaError_t launch_finalize_aggs(Ctx *c, const AggPlan &ap, const int *col_dtype, uint32_t n,
+                                 const unsigned long long *cnt, const void *d_agg, double *values);
 void stream_release(Ctx *c);
 
 

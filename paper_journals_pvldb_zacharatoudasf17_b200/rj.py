@@ -6,7 +6,7 @@ There is no fallback: if librj.so is missing or no sm_100 device is present
 the calls raise.
 
     rj_create, rj_destroy, rj_load_points, rj_load_polygons, rj_query,
-    rj_query_device, rj_query_stream, rj_query_interval, rj_finalize_device, rj_resolve_canvas(_domain),
+    rj_query_device, rj_query_stream, rj_query_interval, rj_query_multi, rj_finalize_device, rj_resolve_canvas(_domain),
     rj_debug_pixel_spans, rj_debug_boundary_mask, rj_debug_point_membership, rj_debug_point_canvas,
     rj_get_stats, rj_set_option  -- same names as the C ABI.
 
@@ -25,7 +25,7 @@ LIB_PATH = os.path.join(_PKG, "librj.so")
 RJ_OK = 0
 STATUS = {0: "RJ_OK", -1: "RJ_ERR_INVALID_ARGUMENT", -2: "RJ_ERR_OUT_OF_DOMAIN", -3: "RJ_ERR_RESOLUTION",
           -4: "RJ_ERR_CAPACITY", -5: "RJ_ERR_OOM", -6: "RJ_ERR_CUDA"}
-AGG = {"count": 0, "sum": 1, "avg": 2}
+AGG = {"count": 0, "sum": 1, "avg": 2, "min": 3, "max": 4}
 MODE = {"bounded": 0, "accurate": 1, "index": 2, "exact": 3}
 OPS = {"<": 0, "<=": 1, ">": 2, ">=": 3, "==": 4}
 DT_I32, DT_F32, DT_F64 = 0, 1, 2
@@ -47,6 +47,10 @@ class rj_query_desc(ctypes.Structure):
     _fields_ = [("agg", ctypes.c_int32), ("agg_column", ctypes.c_int32), ("n_pred", ctypes.c_int32),
                 ("pred", rj_pred * MAX_PRED), ("canvas_w", ctypes.c_int32), ("canvas_h", ctypes.c_int32),
                 ("epsilon", ctypes.c_double), ("mode", ctypes.c_int32)]
+
+
+class rj_agg_spec(ctypes.Structure):
+    _fields_ = [("agg", ctypes.c_int32), ("column", ctypes.c_int32)]
 
 
 class rj_stats(ctypes.Structure):
@@ -84,6 +88,7 @@ def lib():
             "rj_query_device": (i32, [vp, qp, vp, vp]),
             "rj_query_stream": (i32, [vp, qp, u64, vp, vp, i32, i32, vp, vp, vp, vp]),
             "rj_query_interval": (i32, [vp, qp, vp, vp, vp, vp]),
+            "rj_query_multi": (i32, [vp, qp, i32, vp, vp, vp]),
             "rj_debug_point_canvas": (i32, [vp, qp, vp]),
             "rj_finalize_device": (i32, [vp, i32, u32, vp, vp, vp]),
             "rj_resolve_canvas": (i32, [vp, qp, ctypes.POINTER(i32), ctypes.POINTER(i32)]),
@@ -108,7 +113,7 @@ def lib():
 
 
 EXPORTS = ["rj_create", "rj_destroy", "rj_set_allocator", "rj_load_points", "rj_load_polygons", "rj_query",
-           "rj_query_device", "rj_query_stream", "rj_query_interval", "rj_debug_point_canvas", "rj_finalize_device", "rj_resolve_canvas", "rj_resolve_canvas_domain",
+           "rj_query_device", "rj_query_stream", "rj_query_interval", "rj_query_multi", "rj_debug_point_canvas", "rj_finalize_device", "rj_resolve_canvas", "rj_resolve_canvas_domain",
            "rj_debug_pixel_spans", "rj_debug_boundary_mask", "rj_debug_point_membership", "rj_get_stats",
            "rj_set_option", "rj_n_polygons", "rj_n_points", "rj_status_str", "rj_last_error", "rj_version"]
 
@@ -197,6 +202,14 @@ def rj_query_stream(ctx, desc, x, y, cols=(), count=None, value=None):
     dts = (ctypes.c_int32 * max(1, len(cols)))(*[_dtype_code(c) for c in cols])
     _check(lib().rj_query_stream(ctx, ctypes.byref(desc), n, _ptr(x), _ptr(y), _dtype_code(x), len(cols), ptrs, dts,
                                  _ptr(count), _ptr(value)), ctx)
+
+
+def rj_query_multi(ctx, desc, aggs, count=None, values=None):
+    """aggs: [(agg, column)] with agg a name or code; values: float64[len(aggs), n_poly]."""
+    specs = (rj_agg_spec * max(1, len(aggs)))(*[rj_agg_spec(AGG[a] if isinstance(a, str) else int(a), int(c))
+                                                 for a, c in aggs])
+    _check(lib().rj_query_multi(ctx, ctypes.byref(desc), len(aggs), ctypes.addressof(specs), _ptr(count),
+                                _ptr(values)), ctx)
 
 
 def rj_query_interval(ctx, desc, count=None, value=None, eps_plus=None, eps_minus=None):
@@ -305,6 +318,15 @@ class RasterJoin:
         cnt = np.zeros(self.n_poly, dtype=np.uint64)
         val = np.zeros(self.n_poly, dtype=np.float64)
         rj_query_stream(self.ctx, q, x, y, cols, cnt, val)
+        return cnt, val
+
+    def query_multi(self, aggs, **kw):
+        """Several aggregates in one pass: aggs = [("min", col), ("avg", col), ("count", 0), ...].
+        Returns (count uint64[n_poly], values float64[len(aggs), n_poly])."""
+        q = make_desc(**kw)
+        cnt = np.zeros(self.n_poly, dtype=np.uint64)
+        val = np.zeros((len(aggs), self.n_poly), dtype=np.float64)
+        rj_query_multi(self.ctx, q, aggs, cnt, val)
         return cnt, val
 
     def query_interval(self, **kw):

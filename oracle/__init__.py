@@ -53,15 +53,15 @@ def lib():
         L.or_pnpoly.argtypes = [vp, i64, i64, i64]
         L.or_query.restype = u64
         L.or_query.argtypes = [vp, u64, vp, vp, i32, d, d, d, d, i32, vp, vp, i32, i32, vp, vp, vp,
-                               i32, i32, i32, i32, vp, vp]
+                               i32, i32, i32, i32, vp, vp, vp]
         L.or_query_minmax.restype = None
         L.or_query_minmax.argtypes = [vp, u64, vp, vp, i32, d, d, d, d, i32, vp, vp, i32, i32, vp, vp, vp,
-                                      i32, i32, i32, vp, vp]
+                                      i32, i32, i32, vp, vp, vp]
         L.or_avg.restype = None
         L.or_avg.argtypes = [i64, vp, vp, vp]
         L.or_membership.restype = None
         L.or_membership.argtypes = [vp, u64, vp, vp, i32, d, d, d, d, i32, vp, vp, i32, vp, vp, vp,
-                                    i32, i32, i32, vp]
+                                    i32, i32, i32, vp, vp]
         L.or_pixel_membership.restype = None
         L.or_pixel_membership.argtypes = [vp, i32, i32, vp]
         L.or_pixel_spans.restype = i64
@@ -131,6 +131,15 @@ class _Cols:
         return (self.np, self.pc.ctypes.data, self.po.ctypes.data, self.pv.ctypes.data)
 
 
+def _view(view):
+    """O12 window (c0, r0, c1, r1) as an int32 array, or None (whole canvas)."""
+    if view is None:
+        return None, None
+    v = np.ascontiguousarray(view, dtype=np.int32)
+    assert v.shape == (4,)
+    return v, v.ctypes.data
+
+
 def _xy(x, y):
     x = np.ascontiguousarray(x)
     y = np.ascontiguousarray(y)
@@ -138,27 +147,29 @@ def _xy(x, y):
     return x, y, int(x.dtype == np.float64)
 
 
-def query(polys, x, y, cols=(), preds=(), agg_col=-1, W=1024, H=1024, mode="bounded", nthreads=0):
-    """Returns (count u64[n_poly], sum f64[n_poly], n_filtered)."""
+def query(polys, x, y, cols=(), preds=(), agg_col=-1, W=1024, H=1024, mode="bounded", nthreads=0, view=None):
+    """Returns (count u64[n_poly], sum f64[n_poly], n_filtered); view = O12 pixel window."""
     x, y, f64 = _xy(x, y)
     c = _Cols(cols, preds)
+    v, vp = _view(view)
     cnt = np.zeros(polys.n, dtype=np.uint64)
     s = np.zeros(polys.n, dtype=np.float64)
     kept = lib().or_query(polys.h, len(x), x.ctypes.data, y.ctypes.data, f64, *polys.box, *c.args(),
                           int(agg_col), *c.pargs(), int(W), int(H), 0 if mode == "bounded" else 1,
-                          int(nthreads), cnt.ctypes.data, s.ctypes.data)
+                          int(nthreads), cnt.ctypes.data, s.ctypes.data, vp)
     return cnt, s, int(kept)
 
 
-def query_minmax(polys, x, y, cols, agg_col, preds=(), W=1024, H=1024, mode="bounded"):
+def query_minmax(polys, x, y, cols, agg_col, preds=(), W=1024, H=1024, mode="bounded", view=None):
     """O11: (min f64[n_poly], max f64[n_poly]) of column agg_col, NaN for empty polygons."""
     x, y, f64 = _xy(x, y)
     c = _Cols(cols, preds)
+    v, vp = _view(view)
     mn = np.zeros(polys.n, dtype=np.float64)
     mx = np.zeros(polys.n, dtype=np.float64)
     lib().or_query_minmax(polys.h, len(x), x.ctypes.data, y.ctypes.data, f64, *polys.box, *c.args(),
                           int(agg_col), *c.pargs(), int(W), int(H), 0 if mode == "bounded" else 1,
-                          mn.ctypes.data, mx.ctypes.data)
+                          mn.ctypes.data, mx.ctypes.data, vp)
     return mn, mx
 
 
@@ -170,12 +181,13 @@ def avg(cnt, s):
     return out
 
 
-def membership(polys, x, y, cols=(), preds=(), W=1024, H=1024, mode="bounded"):
+def membership(polys, x, y, cols=(), preds=(), W=1024, H=1024, mode="bounded", view=None):
     x, y, f64 = _xy(x, y)
     c = _Cols(cols, preds)
+    v, vp = _view(view)
     bits = np.zeros(len(x), dtype=np.uint64)
     lib().or_membership(polys.h, len(x), x.ctypes.data, y.ctypes.data, f64, *polys.box, *c.args(),
-                        *c.pargs(), int(W), int(H), 0 if mode == "bounded" else 1, bits.ctypes.data)
+                        *c.pargs(), int(W), int(H), 0 if mode == "bounded" else 1, bits.ctypes.data, vp)
     return bits
 
 

@@ -73,12 +73,14 @@ OR_EXPORT int64_t or_qlo(int64_t i, int64_t W) { return or_ceil_div_pos(i * OR_O
 OR_EXPORT int64_t or_qhi(int64_t i, int64_t W) { return or_ceil_div_pos((i + 1) * OR_ONE30, W) - 1; }
 
 /* S0 / reading Z3: epsilon -> resolution, W = ceil(w * sqrt(2) / eps).
- * Returns 0 on success, -1 for a bad epsilon or a resolution outside [1, 32768]. */
+ * Returns 0 on success, -1 for a bad epsilon or a resolution outside
+ * [1, 131072] (reading Z21). */
+#define OR_MAX_CANVAS 131072.0
 OR_EXPORT int or_resolve(double w, double h, double eps, int *W, int *H) {
     if (!(eps > 0.0)) return -1;
     double a = ceil(w * sqrt(2.0) / eps);
     double b = ceil(h * sqrt(2.0) / eps);
-    if (!(a >= 1.0 && a <= 32768.0 && b >= 1.0 && b <= 32768.0)) return -1;
+    if (!(a >= 1.0 && a <= OR_MAX_CANVAS && b >= 1.0 && b <= OR_MAX_CANVAS)) return -1;
     *W = (int)a;
     *H = (int)b;
     return 0;
@@ -239,6 +241,14 @@ static int or_point_q(const void *x, const void *y, int xy_f64, size_t i, double
     return *qx >= 0 && *qx < OR_ONE30 && *qy >= 0 && *qy < OR_ONE30;
 }
 
+/* O12: is the pixel of lattice point (qx, qy) inside the window view =
+ * {c0, r0, c1, r1} (half-open)?  NULL = the whole canvas. */
+static int or_in_view(const int32_t *view, int64_t qx, int64_t qy, int W, int H) {
+    if (!view) return 1;
+    int64_t ix = or_pixel(qx, W), iy = or_pixel(qy, H);
+    return ix >= view[0] && ix < view[2] && iy >= view[1] && iy < view[3];
+}
+
 /* Neumaier-compensated accumulate (O8) */
 static inline void or_nadd(double *s, double *c, double v) {
     double t = *s + v;
@@ -257,7 +267,7 @@ OR_EXPORT uint64_t or_query(const or_polys *p, uint64_t n, const void *x, const 
                             int n_cols, const void *const *cols, const int *dtypes,
                             int agg_col, int n_pred, const int *pcol, const int *pop,
                             const double *pval, int W, int H, int mode, int nthreads,
-                            uint64_t *cnt, double *sum) {
+                            uint64_t *cnt, double *sum, const int32_t *view) {
     or_filter f = {n_cols, cols, dtypes, n_pred, pcol, pop, pval};
     int64_t np = p->n_poly;
     uint64_t kept = 0;
@@ -287,6 +297,7 @@ OR_EXPORT uint64_t or_query(const or_polys *p, uint64_t n, const void *x, const 
             int64_t qx, qy;
             if (!or_point_q(x, y, xy_f64, i, x0, y0, x1, y1, &qx, &qy)) continue;
             if (!or_pass(&f, i)) continue;
+            if (!or_in_view(view, qx, qy, W, H)) continue;
             tkept[tid]++;
             int64_t px = qx, py = qy;
             if (mode == 0) {
@@ -351,7 +362,8 @@ OR_EXPORT void or_query_minmax(const or_polys *p, uint64_t n, const void *x, con
                                double x0, double y0, double x1, double y1,
                                int n_cols, const void *const *cols, const int *dtypes,
                                int agg_col, int n_pred, const int *pcol, const int *pop,
-                               const double *pval, int W, int H, int mode, double *mn, double *mx) {
+                               const double *pval, int W, int H, int mode, double *mn, double *mx,
+                               const int32_t *view) {
     or_filter f = {n_cols, cols, dtypes, n_pred, pcol, pop, pval};
     const int64_t np = p->n_poly;
     const int is_f32 = dtypes[agg_col] == OR_F32;
@@ -362,6 +374,7 @@ OR_EXPORT void or_query_minmax(const or_polys *p, uint64_t n, const void *x, con
         int64_t qx, qy;
         if (!or_point_q(x, y, xy_f64, i, x0, y0, x1, y1, &qx, &qy)) continue;
         if (!or_pass(&f, i)) continue;
+        if (!or_in_view(view, qx, qy, W, H)) continue;
         int64_t px = qx, py = qy;
         if (mode == 0) {
             px = or_centre(or_pixel(qx, W), W);
@@ -399,7 +412,7 @@ OR_EXPORT void or_membership(const or_polys *p, uint64_t n, const void *x, const
                              double x0, double y0, double x1, double y1,
                              int n_cols, const void *const *cols, const int *dtypes,
                              int n_pred, const int *pcol, const int *pop, const double *pval,
-                             int W, int H, int mode, uint64_t *bits) {
+                             int W, int H, int mode, uint64_t *bits, const int32_t *view) {
     or_filter f = {n_cols, cols, dtypes, n_pred, pcol, pop, pval};
     int64_t np = p->n_poly < 64 ? p->n_poly : 64;
     #pragma omp parallel for schedule(dynamic, 1024)
@@ -409,6 +422,7 @@ OR_EXPORT void or_membership(const or_polys *p, uint64_t n, const void *x, const
         bits[i] = 0;
         if (!or_point_q(x, y, xy_f64, i, x0, y0, x1, y1, &qx, &qy)) continue;
         if (!or_pass(&f, i)) continue;
+        if (!or_in_view(view, qx, qy, W, H)) continue;
         int64_t px = qx, py = qy;
         if (mode == 0) {
             px = or_centre(or_pixel(qx, W), W);

@@ -67,7 +67,7 @@ def test_pixel_centre_closed_form_pow2():
         assert L.or_pixel(i * (1 << 20) - 1, 1024) == i - 1
 
 
-@pytest.mark.parametrize("W", [1, 2, 3, 5, 7, 11, 13, 1000, 1024, 4102, 6506, 8191, 32768])
+@pytest.mark.parametrize("W", [1, 2, 3, 5, 7, 11, 13, 1000, 1024, 4102, 6506, 8191, 32768, 81912, 131072])
 def test_pixel_extent_and_centre(W):
     # qlo(i) is the first lattice point of pixel i; the centre lies in the pixel
     L = oracle.lib()
@@ -88,7 +88,10 @@ def test_resolve_epsilon():
     for eps, W in ((80, 1024), (40, 2048), (20, 4096), (10, 8192)):
         assert oracle.resolve(57920.0, 57920.0, eps) == (W, W)
     assert oracle.resolve(4.6e6, 2.9e6, 1000.0) == (6506, 4102)   # C4, eps = 1 km
-    assert oracle.resolve(57920.0, 57920.0, 1.0) is None            # 81912 > 32768
+    # reading Z21: canvases up to 2^17 a side (eps = 1 m on NYC: ceil(57920 sqrt 2) = 81912)
+    assert oracle.resolve(57920.0, 57920.0, 1.0) == (81912, 81912)
+    assert oracle.resolve(131072.0 / math.sqrt(2.0), 1.0, 1.0)[0] in (131072,)  # the cap itself
+    assert oracle.resolve(57920.0, 57920.0, 0.5) is None            # 163824 > 131072
     assert oracle.resolve(1.0, 1.0, 0.0) is None
     assert oracle.resolve(1.0, 1.0, float("nan")) is None
 
@@ -471,3 +474,94 @@ def test_minmax_total_order_special_values():
             else:
                 assert got == exp and np.signbit(got) == np.signbit(exp), vals
         assert np.isnan(mn[1]) and np.isnan(mx[1])          # polygon without points
+
+
+# ---------------------------------------------------------------- O12 viewport
+def _np_pixels(x, y, box, W, H):
+    """O1 + O2 restated in numpy (binary64 division, then an exact shift):
+    the pixel of every point, -1 for points off the domain."""
+    qx = np.floor(((x.astype(np.float64) - box[0]) / (box[2] - box[0])) * 2.0 ** 30)
+    qy = np.floor(((y.astype(np.float64) - box[1]) / (box[3] - box[1])) * 2.0 ** 30)
+    ok = (qx >= 0) & (qx < 2 ** 30) & (qy >= 0) & (qy < 2 ** 30)
+    ix = np.where(ok, (qx.astype(np.int64) * W) >> 30, -1)
+    iy = np.where(ok, (qy.astype(np.int64) * H) >> 30, -1)
+    return ix, iy
+
+
+@pytest.mark.parametrize("mode", ["bounded", "accurate"])
+def test_view_equals_point_subset(mode):
+    # O12: a window query = the full query over the points whose pixel is in
+    # the window (pixels recomputed independently in numpy)
+    polys = C.polygon_set("c1")
+    P = oracle.Polys(PG.flatten(polys), C1)
+    pts = C.c1_points(60_000)
+    x, y = pts["x"], pts["y"]
+    a = (np.arange(len(x)) % 11).astype(np.int32)
+    W, H = 700, 1100
+    view = (123, 201, 650, 977)
+    ix, iy = _np_pixels(x, y, C1, W, H)
+    sel = (ix >= view[0]) & (ix < view[2]) & (iy >= view[1]) & (iy < view[3])
+    cv, sv, kv = oracle.query(P, x, y, cols=[a], agg_col=0, W=W, H=H, mode=mode, view=view)
+    cs, ss, ks = oracle.query(P, x[sel], y[sel], cols=[a[sel]], agg_col=0, W=W, H=H, mode=mode)
+    assert kv == ks == int(sel.sum())
+    assert np.array_equal(cv, cs) and np.array_equal(sv, ss)
+    assert 0 < cv.sum() < oracle.query(P, x, y, W=W, H=H, mode=mode)[0].sum()
+
+
+@pytest.mark.parametrize("mode", ["bounded", "accurate"])
+def test_view_tiles_partition_the_canvas(mode):
+    # multi-canvas rendering (P:625-633): windows tiling the canvas count
+    # every point-polygon pair exactly once
+    polys = C.polygon_set("c1b")
+    P = oracle.Polys(PG.flatten(polys), C1)
+    pts = C.c1_points(40_000)
+    x, y = pts["x"], pts["y"]
+    ax, ay = PG.c1b_points(polys)
+    x, y = np.concatenate([x, ax]), np.concatenate([y, ay])
+    a = (np.arange(len(x)) % 5).astype(np.int32)
+    W, H = 1024, 1024
+    full_c, full_s, full_k = oracle.query(P, x, y, cols=[a], agg_col=0, W=W, H=H, mode=mode)
+    cs, xs = (0, 333, 334, 1024), (0, 512, 1000, 1024)
+    tot_c = np.zeros_like(full_c)
+    tot_s = np.zeros_like(full_s)
+    tot_k = 0
+    for i in range(3):
+        for j in range(3):
+            c, s, k = oracle.query(P, x, y, cols=[a], agg_col=0, W=W, H=H, mode=mode,
+                                   view=(cs[i], xs[j], cs[i + 1], xs[j + 1]))
+            tot_c += c
+            tot_s += s
+            tot_k += k
+    assert tot_k == full_k
+    assert np.array_equal(tot_c, full_c) and np.array_equal(tot_s, full_s)   # integer sums: exact
+
+
+def test_view_lod_zoom_closed_form():
+    # LOD (P:640-650): zooming into a window of a finer canvas.  At W = 8192
+    # on [0,1024)^2 a pixel is 1/8 unit; the window of columns [0, 1200) ends
+    # at x = 150, so the pixel-aligned square P0 = [100,200)^2 counts exactly
+    # the points of [100,150) x [100,200), in both modes.
+    polys = C.polygon_set("c1")
+    P = oracle.Polys(PG.flatten(polys), C1)
+    pts = C.c1_points(100_000)
+    x, y = pts["x"], pts["y"]
+    for mode in ("bounded", "accurate"):
+        c, _, _ = oracle.query(P, x, y, W=8192, H=8192, mode=mode, view=(0, 0, 1200, 8192))
+        assert c[0] == rect_count(x, y, 100, 150, 100, 200)
+        assert c[9] == 0                                   # P9 = [200,300) x [100,200) is clipped
+        c, _, _ = oracle.query(P, x, y, W=8192, H=8192, mode=mode, view=(768, 768, 1792, 1792))
+        assert c[0] == rect_count(x, y, 100, 200, 100, 200)
+
+
+def test_high_resolution_pixel_aligned():
+    # reading Z21: at W = 131072 (2^17) on [0,1024)^2 pixels are 2^-7 units;
+    # P1's vertices (x.5) are on pixel borders, so bounded = accurate =
+    # #[300.5,400.5) x [100.5,200.5) (P1's accurate closed form)
+    polys = C.polygon_set("c1")
+    P = oracle.Polys(PG.flatten(polys), C1)
+    pts = C.c1_points(100_000)
+    x, y = pts["x"], pts["y"]
+    for mode in ("bounded", "accurate"):
+        c, _, _ = oracle.query(P, x, y, W=131072, H=131072, mode=mode)
+        assert c[1] == rect_count(x, y, 300.5, 400.5, 100.5, 200.5)
+        assert c[0] == rect_count(x, y, 100, 200, 100, 200)

@@ -60,7 +60,7 @@ def summarize(rep):
     return "\n".join(lines), result
 
 
-def launches(path):
+def launches(path, steps=0):
     rows = list(csv.reader(open(path)))
     hdr = None
     for i, r in enumerate(rows):
@@ -83,12 +83,23 @@ def launches(path):
     lines = [f"# launch list: {path}", "", "| kernel | launches | total ms | share |", "|---|---|---|---|"]
     for k, v in tot.most_common():
         lines.append(f"| {k} | {cnt[k]} | {v:.3f} | {v / all_ms * 100:.1f} % |")
+    if steps:
+        # kernels launched once (or a fixed number of times) per query step:
+        # launch count a multiple of the number of query steps in the capture
+        q = {k: v for k, v in tot.items() if cnt[k] % steps == 0 and not k.startswith("void at::")
+             and "radix" not in k and "quantize" not in k and "cell_bounds" not in k and "grid_" not in k}
+        q_ms = sum(q.values())
+        lines += ["", f"## per query step ({steps} steps in the capture; load-time kernels excluded)", "",
+                  "| kernel | launches/step | ms/step | share of the step |", "|---|---|---|---|"]
+        for k, v in sorted(q.items(), key=lambda kv: -kv[1]):
+            lines.append(f"| {k} | {cnt[k] // steps} | {v / steps:.4f} | {v / q_ms * 100:.1f} % |")
+        lines.append(f"| (all) | | {q_ms / steps:.4f} | 100 % |")
     return "\n".join(lines)
 
 
 if __name__ == "__main__":
     if sys.argv[1] == "--launches":
-        print(launches(sys.argv[2]))
+        print(launches(sys.argv[2], int(sys.argv[3]) if len(sys.argv) > 3 else 0))
     else:
         text, res = summarize(sys.argv[1])
         print(text)

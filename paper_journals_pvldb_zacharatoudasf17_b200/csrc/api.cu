@@ -91,6 +91,36 @@ static rj_status resolve(double x0, double y0, double x1, double y1, const rj_qu
     return RJ_OK;
 }
 
+// Viewport window (reading Z20): all zero = the whole canvas.
+static rj_status resolve_view(Ctx *c, const rj_query_desc *q, int W, int H, View &v) {
+    v = View{};
+    const int32_t *w = q->view;
+    if (!w[0] && !w[1] && !w[2] && !w[3]) {
+        v.c1 = W;
+        v.r1 = H;
+        return RJ_OK;
+    }
+    if (!(0 <= w[0] && w[0] < w[2] && w[2] <= W && 0 <= w[1] && w[1] < w[3] && w[3] <= H))
+        return set_error(c, RJ_ERR_INVALID_ARGUMENT, "view must be all zero or 0 <= c0 < c1 <= W, 0 <= r0 < r1 <= H");
+    v.c0 = w[0];
+    v.r0 = w[1];
+    v.c1 = w[2];
+    v.r1 = w[3];
+    v.full = v.c0 == 0 && v.r0 == 0 && v.c1 == W && v.r1 == H;
+    return RJ_OK;
+}
+
+// Level-L cell columns [lo, hi] whose pixel extent (cell_pix_lo..hi) meets
+// pixels [p0, p1) of a side of n pixels.
+static void cell_range(int64_t p0, int64_t p1, int64_t n, int L, uint32_t &lo, uint32_t &hi) {
+    const int64_t nc = int64_t(1) << L;
+    int64_t a = 0, b = nc - 1;
+    while (a < nc - 1 && cell_pix_hi(a, n, L) < p0) ++a;
+    while (b > 0 && cell_pix_lo(b, n, L) > p1 - 1) --b;
+    lo = (uint32_t)a;
+    hi = (uint32_t)b;
+}
+
 // Integer predicates become one inclusive int32 range per column:
 // t < c <=> t <= ceil(c)-1,  t <= c <=> t <= floor(c),  t > c <=> t >= floor(c)+1,
 // t >= c <=> t >= ceil(c),   t == c <=> c integral and t == c  (exact for int32 t).
@@ -225,6 +255,7 @@ static int choose_exact(const Ctx *c, int W, int H, float f, uint64_t n_points) 
 
 struct Prepared {
     int W, H, L;
+    View view;
     int mode;                      // executed rj_mode (RJ_EXACT resolved)
     bool sum, acc, index;
     PolyPass pp;
@@ -247,7 +278,8 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     rj_status s = check_ready(c, q);
     if (s != RJ_OK) return s;
     if ((s = resolve(c->x0, c->y0, c->x1, c->y1, q, &P.W, &P.H)) != RJ_OK)
-        return set_error(c, s, "canvas resolution outside [1, 32768] or bad epsilon");
+        return set_error(c, s, "canvas resolution outside [1, 131072] or bad epsilon");
+    if ((s = resolve_view(c, q, P.W, P.H, P.view)) != RJ_OK) return s;
     Filter f;
     if ((s = build_filter(c, q, c->n_cols, c->col_dtype, f)) != RJ_OK) return s;
     P.sum = q->agg != RJ_COUNT;
@@ -279,7 +311,8 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[0], c->stream));
     // the index join needs neither spans nor the boundary mask
     P.pp = PolyPass{};
-    if (need_polygon_pass && !P.index && (s = polygon_pass(c, P.W, P.H, P.L, P.acc || bands, P.pp)) != RJ_OK)
+    if (need_polygon_pass && !P.index &&
+        (s = polygon_pass(c, P.W, P.H, P.L, P.acc || bands, P.pp, P.view)) != RJ_OK)
         return s;
     if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[1], c->stream));
     a.qx = c->qx.as<uint32_t>();
@@ -306,6 +339,37 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     if (dreserve(c, st, 64)) return set_error(c, RJ_ERR_OOM, "workspace allocation failed");
     a.work_counter = st.as<uint32_t>();
     a.stats = reinterpret_cast<unsigned long long *>(st.as<uint32_t>() + 2);
+    a.view[0] = P.view.c0;
+    a.view[1] = P.view.r0;
+    a.view[2] = P.view.c1;
+    a.view[3] = P.view.r1;
+    cell_range(P.view.c0, P.view.c1, P.W, P.L, a.cwin[0], a.cwin[2]);
+    cell_range(P.view.r0, P.view.r1, P.H, P.L, a.cwin[1], a.cwin[3]);
+    return RJ_OK;
+}
+
+// Accurate mode: size the global boundary-point queue (S7).  The capacity
+// follows the previous query's boundary count (grow-only), at least twice
+// the estimated boundary-pixel fraction of the points and >= 2^22; points
+// beyond it are tested inline (always exact).  The index join tests every
+// point inline (no queue).
+static rj_status setup_bqueue(Ctx *c, Prepared &P) {
+    PassArgs &a = P.a;
+    a.bq_cap = 0;
+    a.bq_count = a.work_counter + 8;
+    a.bq_valid = a.work_counter + 9;
+    if (!P.acc || P.index || !c->n_pts) return RJ_OK;
+    const uint64_t est = (uint64_t)(2.0 * c->last.est_boundary_frac * (double)c->n_pts);
+    uint64_t want = std::max<uint64_t>({uint64_t(1) << 22, est, c->h_stats[1] + c->h_stats[1] / 4});
+    want = std::min<uint64_t>(want, c->n_pts);
+    want = std::min<uint64_t>(want, 0xFFFFFFC0ull);
+    Buf &bx = wsbuf(c, kWsBQx), &by = wsbuf(c, kWsBQy), &ba = wsbuf(c, kWsBQa);
+    if (dreserve(c, bx, want * 4) || dreserve(c, by, want * 4) || (P.sum && dreserve(c, ba, want * 4)))
+        return RJ_OK;                                     // no room: inline tests (exact either way)
+    a.bq_x = bx.as<uint32_t>();
+    a.bq_y = by.as<uint32_t>();
+    a.bq_a = P.sum ? ba.as<uint32_t>() : nullptr;
+    a.bq_cap = (uint32_t)want;
     return RJ_OK;
 }
 
@@ -313,11 +377,15 @@ static rj_status run_pass(Ctx *c, Prepared &P, unsigned long long *d_cnt, double
     PassArgs &a = P.a;
     a.A_cnt = d_cnt;
     a.A_sum = d_sum;
+    rj_status s = setup_bqueue(c, P);
+    if (s != RJ_OK) return s;
     RJ_CUDA(c, cudaMemsetAsync(a.work_counter, 0, 64, c->stream));
+    RJ_CUDA(c, cudaMemsetAsync(a.bq_valid, 0xFF, 4, c->stream));
     RJ_CUDA(c, cudaMemsetAsync(d_cnt, 0, (size_t)c->n_poly * 8, c->stream));
     if (P.sum) RJ_CUDA(c, cudaMemsetAsync(d_sum, 0, (size_t)c->n_poly * 8, c->stream));
-    rj_status s = point_pass(c, a, P.sum, P.acc);
+    s = point_pass(c, a, P.sum, P.acc);
     if (s != RJ_OK) return s;
+    if (a.bq_cap && (s = pip_queue_pass(c, a, P.sum)) != RJ_OK) return s;
     if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[2], c->stream));
     RJ_CUDA(c, cudaMemcpyAsync(c->h_stats, a.stats, 2 * sizeof(unsigned long long), cudaMemcpyDeviceToHost, c->stream));
     // statistics of this query
@@ -344,7 +412,9 @@ static rj_status label_query_with_cols(Ctx *c, const rj_query_desc *q, const Agg
     if (cudaSetDevice(c->device) != cudaSuccess) return set_error(c, RJ_ERR_CUDA, "cudaSetDevice failed");
     int W, H;
     rj_status s = resolve(c->x0, c->y0, c->x1, c->y1, q, &W, &H);
-    if (s != RJ_OK) return set_error(c, s, "canvas resolution outside [1, 32768] or bad epsilon");
+    if (s != RJ_OK) return set_error(c, s, "canvas resolution outside [1, 131072] or bad epsilon");
+    View v;
+    if ((s = resolve_view(c, q, W, H, v)) != RJ_OK) return s;
     rj_query_desc qf = *q;
     qf.agg = RJ_COUNT;                        // aggregate columns are read by the plan, not the filter
     Filter f;
@@ -368,7 +438,7 @@ static rj_status label_query_with_cols(Ctx *c, const rj_query_desc *q, const Agg
     if (dreserve(c, c->res_cnt, np * 8) || dreserve(c, c->res_agg, (size_t)std::max(1, kp.n) * np * 8) ||
         dreserve(c, c->res_val, (size_t)nv * np * 8))
         return set_error(c, RJ_ERR_OOM, "result allocation failed");
-    if ((s = label_query_impl(c, f, kp, W, H, mode, in, c->res_cnt.as<unsigned long long>(), c->res_agg.p)) != RJ_OK)
+    if ((s = label_query_impl(c, f, kp, W, H, v, mode, in, c->res_cnt.as<unsigned long long>(), c->res_agg.p)) != RJ_OK)
         return s;
     if (values) {
         for (int k = 0; k < nv; ++k) {
@@ -671,6 +741,8 @@ rj_status rj_query_multi(rj_ctx *c, const rj_query_desc *q, int32_t n_aggs, cons
 rj_status rj_query_interval(rj_ctx *c, const rj_query_desc *q, uint64_t *count, double *value, uint64_t *eps_plus,
                             uint64_t *eps_minus) {
     if (q && q->mode != RJ_BOUNDED) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "result intervals need RJ_BOUNDED");
+    if (q && (q->view[0] || q->view[1] || q->view[2] || q->view[3]))
+        return set_error(c, RJ_ERR_INVALID_ARGUMENT, "result intervals need the whole canvas (view all zero)");
     Prepared P;
     rj_status s = prepare(c, q, P, true, true);
     if (s != RJ_OK) return s;
@@ -699,6 +771,7 @@ rj_status rj_debug_point_canvas(rj_ctx *c, const rj_query_desc *q, uint32_t *cou
     if (!counts || !q) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL counts or query");
     rj_query_desc qq = *q;
     qq.mode = RJ_BOUNDED;
+    qq.view[0] = qq.view[1] = qq.view[2] = qq.view[3] = 0;   // always the whole canvas
     Prepared P;
     rj_status s = prepare(c, &qq, P);
     if (s != RJ_OK) return s;

@@ -41,24 +41,30 @@ constexpr int kLabThreads = 512;
 
 inline unsigned blocks_for(uint64_t n, int t) { return (unsigned)std::max<uint64_t>(1, (n + t - 1) / t); }
 
+// The label canvas covers the viewport window only (reading Z20): pixel
+// (c0 + x, r0 + r) of the W x H canvas is lab[r * vw + x], r < vh, x < vw.
+
 // lab = LAB_BND on boundary pixels (or everywhere: index join), else LAB_NONE.
-__global__ void k_lab_init(uint32_t *__restrict__ lab, int W, const uint32_t *__restrict__ mask, uint32_t wpr,
-                           int all_bnd) {
+__global__ void k_lab_init(uint32_t *__restrict__ lab, uint32_t vw, uint32_t c0, uint32_t r0,
+                           const uint32_t *__restrict__ mask, uint32_t wpr, int all_bnd) {
     const uint64_t r = blockIdx.y;
-    for (uint32_t x = blockIdx.x * blockDim.x + threadIdx.x; x < (uint32_t)W; x += gridDim.x * blockDim.x) {
-        const bool b = all_bnd || (mask && ((mask[r * wpr + (x >> 5)] >> (x & 31)) & 1u));
-        lab[r * W + x] = b ? kLabBnd : kLabNone;
+    for (uint32_t x = blockIdx.x * blockDim.x + threadIdx.x; x < vw; x += gridDim.x * blockDim.x) {
+        const uint32_t px = c0 + x;
+        const bool b = all_bnd || (mask && ((mask[(r0 + r) * wpr + (px >> 5)] >> (px & 31)) & 1u));
+        lab[r * vw + x] = b ? kLabBnd : kLabNone;
     }
 }
 
-// One warp per pixel span (polygon, row, lo, hi): claim its pixels; a pixel
-// claimed twice becomes LAB_MULTI; boundary pixels stay LAB_BND.
-__global__ void k_lab_paint(const uint4 *__restrict__ spans, uint64_t S, uint32_t *__restrict__ lab, int W) {
+// One warp per pixel span (polygon, row, lo, hi) -- clipped to the window by
+// the polygon pass: claim its pixels; a pixel claimed twice becomes
+// LAB_MULTI; boundary pixels stay LAB_BND.
+__global__ void k_lab_paint(const uint4 *__restrict__ spans, uint64_t S, uint32_t *__restrict__ lab, uint32_t vw,
+                            uint32_t c0, uint32_t r0) {
     const uint32_t lane = threadIdx.x & 31;
     const uint64_t nw = ((uint64_t)gridDim.x * blockDim.x) >> 5;
     for (uint64_t s = ((uint64_t)blockIdx.x * blockDim.x + threadIdx.x) >> 5; s < S; s += nw) {
         const uint4 sp = spans[s];
-        uint32_t *row = lab + (uint64_t)sp.y * W;
+        uint32_t *row = lab + (uint64_t)(sp.y - r0) * vw - c0;
         for (uint32_t x = sp.z + lane; x < sp.w; x += 32) {
             const uint32_t o = atomicCAS(&row[x], kLabNone, sp.x);
             if (o != kLabNone && o < kLabBnd) atomicExch(&row[x], kLabMulti);
@@ -66,16 +72,16 @@ __global__ void k_lab_paint(const uint4 *__restrict__ spans, uint64_t S, uint32_
     }
 }
 
-// Row index of the spans (CSR by row), read only for LAB_MULTI pixels.
-__global__ void k_row_count(const uint4 *__restrict__ spans, uint64_t S, uint32_t *__restrict__ cnt) {
+// Row index of the spans (CSR by window row), read only for LAB_MULTI pixels.
+__global__ void k_row_count(const uint4 *__restrict__ spans, uint64_t S, uint32_t r0, uint32_t *__restrict__ cnt) {
     for (uint64_t s = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; s < S; s += (uint64_t)gridDim.x * blockDim.x)
-        atomicAdd(&cnt[spans[s].y], 1u);
+        atomicAdd(&cnt[spans[s].y - r0], 1u);
 }
-__global__ void k_row_fill(const uint4 *__restrict__ spans, uint64_t S, const uint32_t *__restrict__ off,
+__global__ void k_row_fill(const uint4 *__restrict__ spans, uint64_t S, uint32_t r0, const uint32_t *__restrict__ off,
                            uint32_t *__restrict__ cur, uint4 *__restrict__ rs) {
     for (uint64_t s = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; s < S; s += (uint64_t)gridDim.x * blockDim.x) {
         const uint4 sp = spans[s];
-        rs[off[sp.y] + atomicAdd(&cur[sp.y], 1u)] = sp;
+        rs[off[sp.y - r0] + atomicAdd(&cur[sp.y - r0], 1u)] = sp;
     }
 }
 
@@ -84,7 +90,8 @@ struct LabArgs {
     const uint32_t *col[6];          // filter slots
     Filter f;
     double x0, sx, y0, sy;           // lattice transform (S1, reading Z1)
-    uint32_t W, W4, H4;
+    uint32_t W4, H4;
+    uint32_t vc0, vr0, vw, vh;       // viewport window: the label canvas's extent
     const uint32_t *lab;
     const uint32_t *row_off;
     const uint4 *row_spans;
@@ -199,12 +206,13 @@ __global__ void __launch_bounds__(kLabThreads) k_label_pass(const __grid_constan
                     qy = (uint32_t)qyd;
                 }
             }
+            const uint32_t px = __umulhi(qx, s.W4), py = __umulhi(qy, s.H4);   // (q W) >> 30
+            const uint32_t lx = px - s.vc0, ly = py - s.vr0;                     // window-relative
             if (!in) {
                 ++n_ood;                                  // dropped (reading Z11)
-            } else if (lab_filter(s, i)) {
+            } else if (lx < s.vw && ly < s.vh && lab_filter(s, i)) {   // clipped to the window (Z20)
                 ++n_pass;
-                const uint32_t px = __umulhi(qx, s.W4), py = __umulhi(qy, s.H4);   // (q W) >> 30
-                const uint32_t L = __ldg(&s.lab[(uint64_t)py * s.W + px]);
+                const uint32_t L = __ldg(&s.lab[(uint64_t)ly * s.vw + lx]);
                 for (int a = 0; a < na; ++a) {
                     const uint32_t bits = __ldg(&s.agg_col[a][i]);
                     const int kind = s.agg_kind[a];
@@ -216,7 +224,7 @@ __global__ void __launch_bounds__(kLabThreads) k_label_pass(const __grid_constan
                 if (L < kLabBnd) {
                     P = L;
                 } else if (L == kLabMulti) {
-                    for (uint32_t k = __ldg(&s.row_off[py]), e = __ldg(&s.row_off[py + 1]); k < e; ++k) {
+                    for (uint32_t k = __ldg(&s.row_off[ly]), e = __ldg(&s.row_off[ly + 1]); k < e; ++k) {
                         const uint4 sp = __ldg(&s.row_spans[k]);
                         if (sp.z <= px && px < sp.w) emit(sp.x, 1u, v, key);
                     }
@@ -345,7 +353,7 @@ cudaError_t launch_finalize_aggs(Ctx *c, const AggPlan &ap, const int *col_dtype
     return cudaGetLastError();
 }
 
-rj_status label_query_impl(Ctx *c, const Filter &f, const AggPlan &ap, int W, int H, int mode,
+rj_status label_query_impl(Ctx *c, const Filter &f, const AggPlan &ap, int W, int H, const View &v, int mode,
                            const LabInput &in, unsigned long long *d_cnt, void *d_agg) {
     cudaStream_t st = c->stream;
     const bool acc = mode != RJ_BOUNDED, index = mode == RJ_INDEX_JOIN;
@@ -356,32 +364,34 @@ rj_status label_query_impl(Ctx *c, const Filter &f, const AggPlan &ap, int W, in
     // ---- label canvas (S3 spans painted, S5 mask) + row index of the spans
     PolyPass pp;
     rj_status s;
-    if (!index && (s = polygon_pass(c, W, H, -1, acc, pp)) != RJ_OK) return s;
+    if (!index && (s = polygon_pass(c, W, H, -1, acc, pp, v)) != RJ_OK) return s;
     const uint64_t S = pp.n_spans;
+    const uint32_t vc0 = v.full ? 0u : (uint32_t)v.c0, vr0 = v.full ? 0u : (uint32_t)v.r0;
+    const uint32_t vw = v.full ? (uint32_t)W : (uint32_t)(v.c1 - v.c0), vh = v.full ? (uint32_t)H : (uint32_t)(v.r1 - v.r0);
     Buf &lab = wsbuf(c, kWsLab), &rcnt = wsbuf(c, kWsRowCount), &roff = wsbuf(c, kWsRowOff);
     Buf &rcur = wsbuf(c, kWsRowCursor), &rsp = wsbuf(c, kWsRowSpans), &sts = wsbuf(c, kWsStream);
-    if (dreserve(c, lab, (uint64_t)W * H * 4) || dreserve(c, rcnt, (uint64_t)(H + 1) * 4) ||
-        dreserve(c, roff, (uint64_t)(H + 1) * 4) || dreserve(c, rcur, (uint64_t)(H + 1) * 4) ||
+    if (dreserve(c, lab, (uint64_t)vw * vh * 4) || dreserve(c, rcnt, (uint64_t)(vh + 1) * 4) ||
+        dreserve(c, roff, (uint64_t)(vh + 1) * 4) || dreserve(c, rcur, (uint64_t)(vh + 1) * 4) ||
         dreserve(c, rsp, (S + 1) * 16) || dreserve(c, sts, 64))
         return set_error(c, RJ_ERR_OOM, "label-canvas workspace allocation failed");
-    k_lab_init<<<dim3(blocks_for(W, 256), H), 256, 0, st>>>(lab.as<uint32_t>(), W, acc && !index ? pp.mask : nullptr,
-                                                           pp.mask_wpr, index);
+    k_lab_init<<<dim3(blocks_for(vw, 256), vh), 256, 0, st>>>(lab.as<uint32_t>(), vw, vc0, vr0,
+                                                             acc && !index ? pp.mask : nullptr, pp.mask_wpr, index);
     RJ_LAUNCHED(c);
-    RJ_CUDA(c, cudaMemsetAsync(rcnt.p, 0, (uint64_t)(H + 1) * 4, st));
-    RJ_CUDA(c, cudaMemsetAsync(rcur.p, 0, (uint64_t)(H + 1) * 4, st));
+    RJ_CUDA(c, cudaMemsetAsync(rcnt.p, 0, (uint64_t)(vh + 1) * 4, st));
+    RJ_CUDA(c, cudaMemsetAsync(rcur.p, 0, (uint64_t)(vh + 1) * 4, st));
     if (S) {
         const unsigned g = (unsigned)std::min<uint64_t>(blocks_for(S * 32, 256), c->num_sms * 16ull);
-        k_lab_paint<<<g, 256, 0, st>>>(reinterpret_cast<const uint4 *>(pp.spans), S, lab.as<uint32_t>(), W);
+        k_lab_paint<<<g, 256, 0, st>>>(reinterpret_cast<const uint4 *>(pp.spans), S, lab.as<uint32_t>(), vw, vc0, vr0);
         RJ_LAUNCHED(c);
         const unsigned g2 = (unsigned)std::min<uint64_t>(blocks_for(S, 256), c->num_sms * 8ull);
-        k_row_count<<<g2, 256, 0, st>>>(reinterpret_cast<const uint4 *>(pp.spans), S, rcnt.as<uint32_t>());
+        k_row_count<<<g2, 256, 0, st>>>(reinterpret_cast<const uint4 *>(pp.spans), S, vr0, rcnt.as<uint32_t>());
         RJ_LAUNCHED(c);
-        RJ_CUDA(c, scan_u32(c, rcnt.as<uint32_t>(), roff.as<uint32_t>(), (uint64_t)H, kWsScan));
-        k_row_fill<<<g2, 256, 0, st>>>(reinterpret_cast<const uint4 *>(pp.spans), S, roff.as<uint32_t>(),
+        RJ_CUDA(c, scan_u32(c, rcnt.as<uint32_t>(), roff.as<uint32_t>(), (uint64_t)vh, kWsScan));
+        k_row_fill<<<g2, 256, 0, st>>>(reinterpret_cast<const uint4 *>(pp.spans), S, vr0, roff.as<uint32_t>(),
                                        rcur.as<uint32_t>(), rsp.as<uint4>());
         RJ_LAUNCHED(c);
     } else {
-        RJ_CUDA(c, cudaMemsetAsync(roff.p, 0, (uint64_t)(H + 1) * 4, st));
+        RJ_CUDA(c, cudaMemsetAsync(roff.p, 0, (uint64_t)(vh + 1) * 4, st));
     }
     RJ_CUDA(c, cudaGetLastError());
     if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[1], st));
@@ -395,7 +405,10 @@ rj_status label_query_impl(Ctx *c, const Filter &f, const AggPlan &ap, int W, in
     a.sx = c->x1 - c->x0;
     a.y0 = c->y0;
     a.sy = c->y1 - c->y0;
-    a.W = (uint32_t)W;
+    a.vc0 = vc0;
+    a.vr0 = vr0;
+    a.vw = vw;
+    a.vh = vh;
     a.W4 = (uint32_t)W << 2;
     a.H4 = (uint32_t)H << 2;
     a.lab = lab.as<uint32_t>();

@@ -47,8 +47,9 @@ __global__ void k_membership(const PassArgs a, uint64_t n, int accurate, const u
     for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n; i += (uint64_t)gridDim.x * blockDim.x) {
         const uint32_t qx = a.qx[i], qy = a.qy[i];
         unsigned long long m = 0;
-        if (filter_point(a, i)) {
-            const int64_t px = pix(qx, a.W), py = pix(qy, a.H);
+        const int64_t px = pix(qx, a.W), py = pix(qy, a.H);
+        const bool in_view = px >= a.view[0] && px < a.view[2] && py >= a.view[1] && py < a.view[3];
+        if (in_view && filter_point(a, i)) {
             bool bnd = false;
             if (accurate) bnd = a.index_join || ((a.mask[(uint64_t)py * a.mask_wpr + (px >> 5)] >> (px & 31)) & 1u);
             if (bnd) {

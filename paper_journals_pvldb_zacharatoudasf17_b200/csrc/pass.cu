@@ -86,7 +86,7 @@ __device__ __forceinline__ void process(const PassArgs &a, const Shared &sh, con
 #pragma unroll
             for (int j = 0; j < kIPL; ++j) {
                 enqueue<SUM, NS>(a, sh, w, j, (bm >> j) & 1u, qn, n_bnd);   // adds <= 32
-                if (qn >= 32) drain_queue<SUM>(a, sh, qn, false);            // leaves < 32
+                if (qn >= 32) spill_queue<SUM>(a, sh, qn, false);            // leaves < 32
             }
 #pragma unroll
             for (int j = 0; j < kIPL; ++j) ok[j] = ok[j] && !((bm >> j) & 1u);
@@ -208,7 +208,7 @@ __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a)
                 t.tbase = smem_u32(t.cnt) - 4u * t.base;
                 const uint32_t words = t.th * t.stride;
                 if (ACC) {
-                    clear_tile_acc(t.cnt, t.stride, t.th, t.tw, r0, c0, a.mask, a.mask_wpr, a.index_join, kFlag, 0u);
+                    clear_tile_acc(t.cnt, t.stride, t.th, t.tw, r0, c0, a.mask, a.mask_wpr, a.index_join, kFlag, 0u, a.view);
                 } else {
                     for (uint32_t i = threadIdx.x; i < words; i += kThreads) t.cnt[i] = 0u;
                 }
@@ -231,7 +231,6 @@ __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a)
             if (lane == 0) mbar_arrive(smem_u32(&rg.empty[st]));
             if (m.flags & 2u) {
                 // ---- last stage of the cell: reduce the tile over the span pieces (S4)
-                if (ACC && qn) drain_queue<SUM>(a, sh, qn, true);
                 consumers_sync();                          // every point of the cell is in the tile
                 if (a.canvas) dump_canvas(a, t, m.cell, s_lat);
                 for (uint32_t kk = pb + threadIdx.x; kk < pe; kk += kThreads) {
@@ -255,6 +254,7 @@ __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a)
             }
             if (++st == nstage) { st = 0; ph ^= 1u; }
         }
+        if (ACC && qn) spill_queue<SUM>(a, sh, qn, true);   // boundary points are independent of the tiles
         for (int o = 16; o; o >>= 1) {
             n_pass += __shfl_xor_sync(kFull, n_pass, o);
             if (ACC) n_bnd += __shfl_xor_sync(kFull, n_bnd, o);
@@ -274,6 +274,52 @@ __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a)
         atomicAdd(&a.stats[0], (unsigned long long)s_pass);
         if (ACC) atomicAdd(&a.stats[1], (unsigned long long)s_bnd);
     }
+}
+
+// Accurate mode, after the point pass: the exact test (Proc. JoinPoint,
+// P:718-726) of every queued boundary point, one per thread, at full
+// occupancy.  The queue holds the points in the order the consumer warps met
+// them -- batches of 32 from one cell, Morton-ordered -- so neighbouring
+// threads walk the same grid cells (L1 hits) and mostly land in the same
+// polygon (one partial update per distinct polygon of a warp).
+template <bool SUM>
+__global__ void __launch_bounds__(256) k_pip_queue(const __grid_constant__ PassArgs a) {
+    extern __shared__ __align__(16) unsigned char smem_raw[];
+    Shared sh{};
+    sh.pcnt = reinterpret_cast<uint32_t *>(smem_raw);
+    if (a.smem_partials)
+        for (uint32_t k = threadIdx.x; k < a.n_poly; k += blockDim.x) sh.pcnt[k] = 0;
+    __syncthreads();
+    const uint32_t n = min(*a.bq_count, *a.bq_valid);
+    const int lane = threadIdx.x & 31;
+    const uint32_t step = gridDim.x * blockDim.x;
+    for (uint32_t base = blockIdx.x * blockDim.x + (threadIdx.x & ~31u); base < n; base += step) {
+        const uint32_t i = base + lane;
+        uint32_t P = kNoPoly;
+        double v = 0.0;
+        if (i < n) {
+            const uint32_t x = __ldcs(&a.bq_x[i]), y = __ldcs(&a.bq_y[i]);
+            if (SUM) v = attr_val(__ldcs(&a.bq_a[i]), a.f.agg_is_float);
+            P = join_point<SUM>(a, sh, x, y, v);
+        }
+        unsigned active = __ballot_sync(kFull, P != kNoPoly);
+        while (active) {
+            const int leader = __ffs(active) - 1;
+            const uint32_t PL = __shfl_sync(kFull, P, leader);
+            const unsigned m = __ballot_sync(kFull, P == PL);
+            double s = (SUM && P == PL) ? v : 0.0;
+            if (SUM)
+                for (int o = 16; o; o >>= 1) s += __shfl_xor_sync(kFull, s, o);
+            if (lane == leader) emit_poly<SUM>(a, sh, PL, __popc(m), s);
+            active &= ~m;
+        }
+    }
+    __syncthreads();
+    if (a.smem_partials)
+        for (uint32_t k = threadIdx.x; k < a.n_poly; k += blockDim.x) {
+            const uint32_t cc = sh.pcnt[k];
+            if (cc) atomicAdd(&a.A_cnt[k], (unsigned long long)cc);
+        }
 }
 
 template <bool SUM, bool ACC, bool FP>
@@ -357,12 +403,29 @@ size_t point_pass_smem(const Ctx *c, const PassArgs &a, bool sum, bool accurate)
     return use_label(c, a, sum, accurate) ? point_pass_label_smem(a, accurate) : tile_pass_smem(a, sum, accurate);
 }
 
+rj_status pip_queue_pass(Ctx *c, const PassArgs &a_in, bool sum) {
+    PassArgs a = a_in;
+    a.smem_partials = (size_t)a.n_poly * 4 <= 64 * 1024;
+    const size_t smem = a.smem_partials ? (size_t)a.n_poly * 4 : 0;
+    void *k = sum ? (void *)k_pip_queue<true> : (void *)k_pip_queue<false>;
+    RJ_CUDA(c, cudaFuncSetAttribute(k, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem));
+    int per_sm = 0;
+    RJ_CUDA(c, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k, 256, smem));
+    const unsigned grid = (unsigned)std::max(1, per_sm) * (unsigned)c->num_sms;
+    void *args[] = {(void *)&a};
+    RJ_CUDA(c, cudaLaunchKernel(k, dim3(grid), dim3(256), args, smem, c->stream));
+    RJ_LAUNCHED(c);
+    return RJ_OK;
+}
+
 int point_pass_stages(int n_slots) { return (2 + n_slots) <= 4 ? 3 : 2; }
 
 rj_status point_pass(Ctx *c, const PassArgs &a_in, bool sum, bool accurate) {
     if (use_label(c, a_in, sum, accurate)) return point_pass_label(c, a_in, accurate);
     PassArgs a = a_in;
     a.n_stages = (uint32_t)choose_stages(a, tile_pass_smem, sum, accurate, c->force_stages);
+    // a fp64 pixel tile that does not fit (canvases beyond 2^16) -> polygon labels
+    if (!a.n_stages && sum && !a.canvas) return point_pass_label(c, a_in, accurate);
     if (!a.n_stages) return set_error(c, RJ_ERR_RESOLUTION, "point-pass tiles do not fit in shared memory");
     return launch_pass(c, select_kernel(sum, accurate, a.f.n_slots, a.f.n_fpred > 0), a,
                        tile_pass_smem(a, sum, accurate));

@@ -142,6 +142,41 @@ __device__ __noinline__ void drain_queue(const PassArgs &a, const Shared &sh, ui
     }
 }
 
+// Move the warp's queued boundary points to the global queue, 32 at a time
+// (`all`: also a last partial batch), for k_pip_queue to test after the pass:
+// the latency-bound grid walk then runs at full occupancy instead of holding
+// up the stage ring.  A reservation that does not fit the queue records its
+// base in bq_valid and the points are tested inline instead (drain_queue).
+template <bool SUM>
+__device__ __noinline__ void spill_queue(const PassArgs &a, const Shared &sh, uint32_t &qn, bool all) {
+    const int lane = threadIdx.x & 31;
+    while (qn >= 32 || (all && qn > 0)) {
+        __syncwarp();
+        const uint32_t take = qn >= 32 ? 32u : qn;
+        uint32_t base = 0;
+        if (lane == 0) {
+            base = atomicAdd(a.bq_count, take);
+            if (base + take > a.bq_cap) {
+                atomicMin(a.bq_valid, base);
+                base = kDone;
+            }
+        }
+        base = __shfl_sync(kFull, base, 0);
+        if (base == kDone) {
+            drain_queue<SUM>(a, sh, qn, all);
+            return;
+        }
+        if ((uint32_t)lane < take) {
+            const uint32_t pos = qn - take + lane;
+            a.bq_x[base + lane] = sh.qx[pos];
+            a.bq_y[base + lane] = sh.qy[pos];
+            if (SUM) a.bq_a[base + lane] = sh.qa[pos];
+        }
+        __syncwarp();
+        qn -= take;
+    }
+}
+
 template <int NS, bool FP>
 __device__ __forceinline__ bool pass_point(const PassArgs &a, const Consts<NS> &k, const Win<NS> &w, int j) {
     bool ok = true;
@@ -196,20 +231,25 @@ __device__ __forceinline__ void enqueue(const PassArgs &a, const Shared &sh, con
 // the lanes that need them, and the row loop is unrolled so several rows'
 // loads are in flight (the clear sits between two consumer barriers, so its
 // L2 latency is exposed).
+// The index join (`all`) flags only the pixels inside the viewport window
+// view = (c0, r0, c1, r1) (the mask is already clipped to it).
 __device__ __forceinline__ void clear_tile_acc(uint32_t *tile, uint32_t stride, uint32_t th, uint32_t tw,
                                                uint32_t r0, uint32_t c0, const uint32_t *mask, uint32_t wpr,
-                                               bool all, uint32_t flag, uint32_t zero) {
+                                               bool all, uint32_t flag, uint32_t zero, const int32_t *view) {
     const uint32_t lane = threadIdx.x & 31, wid = threadIdx.x >> 5;
     const uint32_t w0 = c0 >> 5;
     const uint32_t nwords = ((c0 + tw - 1) >> 5) - w0 + 1;
+    const uint32_t vc0 = (uint32_t)view[0], vr0 = (uint32_t)view[1], vc1 = (uint32_t)view[2], vr1 = (uint32_t)view[3];
 #pragma unroll 4
     for (uint32_t r = wid; r < th; r += kWarps) {
         uint32_t word = 0xFFFFFFFFu;
         if (!all && lane < nwords) word = __ldg(&mask[(uint64_t)(r0 + r) * wpr + w0 + lane]);
+        const bool row_in = !all || (r0 + r >= vr0 && r0 + r < vr1);
         for (uint32_t x0 = 0; x0 < stride; x0 += 32) {
             const uint32_t x = x0 + lane, px = c0 + x;
             const uint32_t wv = __shfl_sync(kFull, word, ((px >> 5) - w0) & 31u);
-            if (x < stride) tile[r * stride + x] = (x < tw && ((wv >> (px & 31)) & 1u)) ? flag : zero;
+            const bool in = row_in && (!all || (px >= vc0 && px < vc1));
+            if (x < stride) tile[r * stride + x] = (x < tw && in && ((wv >> (px & 31)) & 1u)) ? flag : zero;
         }
     }
 }
@@ -277,6 +317,9 @@ __device__ __forceinline__ void produce(const PassArgs &a, Ring &r, uint32_t *ri
         if (it >= a.n_items) break;
         const int4 I = a.items[it];
         for (uint32_t c = (uint32_t)I.x; c < (uint32_t)I.y; ++c) {
+            // viewport: only the cells meeting the window are streamed
+            const uint32_t ccx = cell_x(c), ccy = cell_y(c);
+            if (ccx < a.cwin[0] || ccx > a.cwin[2] || ccy < a.cwin[1] || ccy > a.cwin[3]) continue;
             const uint32_t b = max((uint32_t)I.z, a.cell_off10[(uint64_t)c << sh2]);
             const uint32_t e = min((uint32_t)I.w, a.cell_off10[(uint64_t)(c + 1) << sh2]);
             if (b >= e) continue;

@@ -79,7 +79,7 @@ __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh,
                             attr_val(agg_bits<NS>(a, w, j), a.f.agg_is_float));
             if (ACC) {
                 enqueue<true, NS>(a, sh, w, j, lab[j] == kBnd, qn, n_bnd);   // adds <= 32
-                if (qn >= 32) drain_queue<true>(a, sh, qn, false);            // leaves < 32
+                if (qn >= 32) spill_queue<true>(a, sh, qn, false);            // leaves < 32
             }
             if (lab[j] >= kBnd) lab[j] = kNone;
         }
@@ -199,7 +199,7 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
                     t.pe = __ldg(&a.piece_off[m.cell + 1]);
                 }
                 if (ACC) {
-                    clear_tile_acc(lt, t.stride, th, tw, t.r0, t.c0, a.mask, a.mask_wpr, a.index_join, kBnd, kNone);
+                    clear_tile_acc(lt, t.stride, th, tw, t.r0, t.c0, a.mask, a.mask_wpr, a.index_join, kBnd, kNone, a.view);
                 } else {
                     for (uint32_t i = threadIdx.x; i < th * t.stride; i += kThreads) lt[i] = kNone;
                 }
@@ -223,12 +223,11 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
                 load_win_smem<NS>(w, ring + (size_t)st * ncol * kStagePts, woff + lane * kIPL);
                 process_lab<ACC, NS, FP>(a, sh, t, k, w, (m.sb - m.cb) - woff, m.se - m.sb, cy, qn, n_pass, n_bnd);
             }
-            if (ACC && (m.flags & 2u) && qn) drain_queue<true>(a, sh, qn, true);
             __syncwarp();
             if (lane == 0) mbar_arrive(smem_u32(&rg.empty[st]));
             if (++st == nstage) { st = 0; ph ^= 1u; }
         }
-        if (ACC && qn) drain_queue<true>(a, sh, qn, true);
+        if (ACC && qn) spill_queue<true>(a, sh, qn, true);
         if (lane == 0) emit_lab_run(a, sh, cy.lab, cy.cnt, cy.sum, true);
         for (int o = 16; o; o >>= 1) {
             n_pass += __shfl_xor_sync(kFull, n_pass, o);

@@ -149,7 +149,16 @@ struct SpanGeo {
     uint32_t n_poly;
     const int4 *mbr;
     const uint32_t *cell_off10; // point cells: skip pieces of empty cells
+    int32_t c0, r0, c1, r1;     // viewport window (reading Z20): spans are clipped to it
 };
+
+// Clip span [lo, hi) of row r to the viewport window; false if nothing is left.
+__device__ __forceinline__ bool clip_span(const SpanGeo &g, int64_t r, int64_t &lo, int64_t &hi) {
+    if (r < g.r0 || r >= g.r1) return false;
+    lo = max(lo, (int64_t)g.c0);
+    hi = min(hi, (int64_t)g.c1);
+    return lo < hi;
+}
 
 __device__ __forceinline__ void polyrow_of(const SpanGeo &g, uint32_t pr, uint32_t &P, int64_t &r) {
     P = upper_bound_u32(g.prow_off, g.n_poly + 1, pr) - 1;
@@ -192,8 +201,8 @@ __global__ void k_prow_count(SpanGeo g, uint32_t n_prow, const uint32_t *__restr
         polyrow_of(g, pr, P, r);
         uint32_t ns = 0;
         for (uint32_t i = b; i + 1 < e; i += 2) {
-            const int64_t lo = tv[i], hi = tv[i + 1];
-            if (lo >= hi) continue;
+            int64_t lo = tv[i], hi = tv[i + 1];
+            if (!clip_span(g, r, lo, hi)) continue;
             ++ns;
             for_each_piece(g, r, lo, hi, [&](uint32_t cell, uint32_t, uint32_t, uint32_t) {
                 atomicAdd(&piece_cnt[cell], 1u);
@@ -214,8 +223,8 @@ __global__ void k_prow_emit(SpanGeo g, uint32_t n_prow, const uint32_t *__restri
         polyrow_of(g, pr, P, r);
         uint32_t k = span_off[pr];
         for (uint32_t i = b; i + 1 < e; i += 2) {
-            const int64_t lo = tv[i], hi = tv[i + 1];
-            if (lo >= hi) continue;
+            int64_t lo = tv[i], hi = tv[i + 1];
+            if (!clip_span(g, r, lo, hi)) continue;
             uint32_t *s = spans + 4 * (uint64_t)k++;
             s[0] = P; s[1] = (uint32_t)r; s[2] = (uint32_t)lo; s[3] = (uint32_t)hi;
             for_each_piece(g, r, lo, hi, [&](uint32_t cell, uint32_t lr, uint32_t a, uint32_t bb) {
@@ -227,15 +236,21 @@ __global__ void k_prow_emit(SpanGeo g, uint32_t n_prow, const uint32_t *__restri
 }
 
 // -------------------------------------------------------------- S5 supercover
+// (marks only inside the viewport window [c0, c1) x [r0, r1))
 __global__ void k_mask_mark(const int4 *__restrict__ edges, const uint32_t *__restrict__ band_off,
-                            uint32_t n_edges, int W, int H, uint32_t wpr, uint32_t *__restrict__ mask) {
+                            uint32_t n_edges, int W, int H, uint32_t wpr, uint32_t *__restrict__ mask,
+                            int4 view) {
     const uint32_t total = band_off[n_edges];
     for (uint32_t j = blockIdx.x * blockDim.x + threadIdx.x; j < total; j += gridDim.x * blockDim.x) {
         const uint32_t e = upper_bound_u32(band_off, n_edges + 1, j) - 1;
         const int4 E = edges[e];
         const int64_t r = pix(min(E.y, E.w), H) + (j - band_off[e]);
+        if (r < view.y || r >= view.w) continue;
         int64_t i0, i1;
         if (!supercover_cols(E.x, E.y, E.z, E.w, r, W, H, i0, i1)) continue;
+        i0 = max(i0, (int64_t)view.x);
+        i1 = min(i1, (int64_t)view.z - 1);
+        if (i0 > i1) continue;
         uint32_t *row = mask + (uint64_t)r * wpr;
         for (int64_t w = i0 >> 5; w <= (i1 >> 5); ++w) {
             const int64_t a = max(i0, w << 5) - (w << 5), b = min(i1, (w << 5) + 31) - (w << 5);
@@ -368,7 +383,7 @@ rj_status load_polygons_impl(Ctx *c, uint32_t n_poly, const uint32_t *pro, const
 }
 
 // ------------------------------------------------------------ per-query pass
-rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp) {
+rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp, const View &v) {
     // L < 0: spans (and mask) only, no pieces (the streamed query)
     const uint64_t ncell = L >= 0 ? 1ull << (2 * L) : 0;
     const uint32_t ne = c->n_edges, np = c->n_poly;
@@ -422,7 +437,8 @@ rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp)
     k_scatter_t<<<gx, 256, 0, st>>>(cpr.as<uint32_t>(), ct.as<uint32_t>(), X, pro.as<uint32_t>(),
                                     prcur.as<uint32_t>(), tv.as<uint32_t>());
     RJ_LAUNCHED(c);
-    SpanGeo g{W, H, L, proff.as<uint32_t>(), np, c->mbr.as<int4>(), c->cell_off.as<uint32_t>()};
+    SpanGeo g{W, H, L, proff.as<uint32_t>(), np, c->mbr.as<int4>(), c->cell_off.as<uint32_t>(),
+              v.full ? 0 : v.c0, v.full ? 0 : v.r0, v.full ? W : v.c1, v.full ? H : v.r1};
     const unsigned gp = (unsigned)std::min<uint64_t>(std::max<uint64_t>(1, blocks_for(NPR, 128)), c->num_sms * 16ull);
     k_prow_count<<<gp, 128, 0, st>>>(g, NPR, pro.as<uint32_t>(), tv.as<uint32_t>(), scnt.as<uint32_t>(),
                                      pcnt.as<uint32_t>());
@@ -459,7 +475,9 @@ rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp)
         if (dreserve(c, mask, (uint64_t)wpr * H * 4)) return set_error(c, RJ_ERR_OOM, "mask allocation failed");
         RJ_CUDA(c, cudaMemsetAsync(mask.p, 0, (uint64_t)wpr * H * 4, st));
         const unsigned gb = (unsigned)std::min<uint64_t>(std::max<uint64_t>(1, blocks_for(B, 256)), c->num_sms * 8ull);
-        k_mask_mark<<<gb, 256, 0, st>>>(c->edges.as<int4>(), boff.as<uint32_t>(), ne, W, H, wpr, mask.as<uint32_t>());
+        const int4 vw = v.full ? make_int4(0, 0, W, H) : make_int4(v.c0, v.r0, v.c1, v.r1);
+        k_mask_mark<<<gb, 256, 0, st>>>(c->edges.as<int4>(), boff.as<uint32_t>(), ne, W, H, wpr, mask.as<uint32_t>(),
+                                        vw);
         RJ_LAUNCHED(c);
         RJ_CUDA(c, cudaGetLastError());
         pp.mask = mask.as<uint32_t>();

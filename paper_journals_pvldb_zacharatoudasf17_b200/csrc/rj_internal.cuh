@@ -38,6 +38,13 @@ struct Filter {
     int32_t agg_is_float = 0;     // its dtype (avoids a dynamically indexed param)
 };
 
+// Viewport window of a query (rj_query_desc.view, reading Z20): pixels
+// [c0, c1) x [r0, r1) of the W x H canvas; full = the whole canvas.
+struct View {
+    int32_t c0 = 0, r0 = 0, c1 = 0, r1 = 0;
+    bool full = true;
+};
+
 // Device-side parameter block of the fused point pass.
 struct PassArgs {
     const uint32_t *qx, *qy;
@@ -69,6 +76,15 @@ struct PassArgs {
     int32_t index_join;           // every pixel is a boundary pixel, no span pieces (RJ_INDEX_JOIN)
     uint32_t *canvas;             // tile kernel: dump per-pixel filtered counts (W x H) when set
     unsigned long long *stats;    // [0] filtered, [1] boundary
+    int32_t view[4];              // viewport pixel window (c0, r0, c1, r1), half-open
+    uint32_t cwin[4];             // level-L cells meeting it: columns [cwin0, cwin2], rows [cwin1, cwin3]
+    // accurate mode: boundary points are appended to this global queue
+    // (SoA, bq_cap entries) and tested by k_pip_queue after the pass;
+    // bq_cap == 0 -> tested inline by the consumer warps
+    uint32_t *bq_x, *bq_y, *bq_a;
+    uint32_t bq_cap;
+    uint32_t *bq_count;           // entries reserved
+    uint32_t *bq_valid;           // first failed reservation (entries below it are written)
 };
 
 struct Ctx {
@@ -140,6 +156,7 @@ enum : int {
     kWsWork, kWsSizes,
     kWsLab, kWsRowCount, kWsRowOff, kWsRowCursor, kWsRowSpans, kWsStream,   // streamed query
     kWsCanvas, kWsBRowCount, kWsBRowOff, kWsBktCount, kWsBktOff, kWsBktCursor, kWsBktRanges,   // intervals
+    kWsBQx, kWsBQy, kWsBQa,                 // accurate mode: global boundary-point queue
     kWsScan = 72,                           // 72..95 recursive scan temporaries
 };
 
@@ -188,7 +205,7 @@ struct LabInput {
 // Partials (device, caller-sized): d_cnt[n_poly]; d_agg[k * n_poly ...]:
 // binary64 sums for SUM/AVG, orderable u32 keys (in the low half of the
 // 8-byte slot array) for MIN/MAX.
-rj_status label_query_impl(Ctx *c, const Filter &f, const AggPlan &ap, int W, int H, int mode,
+rj_status label_query_impl(Ctx *c, const Filter &f, const AggPlan &ap, int W, int H, const View &v, int mode,
                            const LabInput &in, unsigned long long *d_cnt, void *d_agg);
 // values[k * n + i] from the partials (NaN for an empty polygon's AVG/MIN/MAX).
 cudaError_t launch_finalize_aggs(Ctx *c, const AggPlan &ap, const int *col_dtype, uint32_t n,
@@ -207,7 +224,8 @@ struct PolyPass {
     uint32_t *mask = nullptr;        // accurate only
     uint32_t mask_wpr = 0;
 };
-rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp);
+// Spans, pieces and the boundary mask are clipped to the viewport window v.
+rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp, const View &v);
 
 // interval.cu: bounded-mode worst-case result intervals from the
 // per-pixel count canvas, the spans and the S5 bands of the polygon pass.
@@ -216,6 +234,8 @@ rj_status interval_impl(Ctx *c, int W, int H, const PolyPass &pp, const uint32_t
 
 // pass.cu
 rj_status point_pass(Ctx *c, const PassArgs &a, bool sum, bool accurate);
+// accurate mode: exact PIP of the queued boundary points (after point_pass)
+rj_status pip_queue_pass(Ctx *c, const PassArgs &a, bool sum);
 size_t point_pass_smem(const Ctx *c, const PassArgs &a, bool sum, bool accurate);
 int point_pass_stages(int n_slots);
 

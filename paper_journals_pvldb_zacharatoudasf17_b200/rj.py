@@ -46,7 +46,7 @@ class rj_pred(ctypes.Structure):
 class rj_query_desc(ctypes.Structure):
     _fields_ = [("agg", ctypes.c_int32), ("agg_column", ctypes.c_int32), ("n_pred", ctypes.c_int32),
                 ("pred", rj_pred * MAX_PRED), ("canvas_w", ctypes.c_int32), ("canvas_h", ctypes.c_int32),
-                ("epsilon", ctypes.c_double), ("mode", ctypes.c_int32)]
+                ("epsilon", ctypes.c_double), ("mode", ctypes.c_int32), ("view", ctypes.c_int32 * 4)]
 
 
 class rj_agg_spec(ctypes.Structure):
@@ -143,7 +143,8 @@ def _dtype_code(a):
     return {"float32": DT_F32, "float64": DT_F64, "int32": DT_I32}[name]
 
 
-def make_desc(agg="count", agg_column=-1, preds=(), W=0, H=0, epsilon=0.0, mode="bounded"):
+def make_desc(agg="count", agg_column=-1, preds=(), W=0, H=0, epsilon=0.0, mode="bounded", view=None):
+    """view = (c0, r0, c1, r1): viewport pixel window of the W x H canvas (None = whole canvas)."""
     q = rj_query_desc()
     q.agg = AGG[agg] if isinstance(agg, str) else int(agg)
     q.agg_column = int(agg_column)
@@ -157,7 +158,29 @@ def make_desc(agg="count", agg_column=-1, preds=(), W=0, H=0, epsilon=0.0, mode=
     q.canvas_w, q.canvas_h = int(W), int(H if H else W)
     q.epsilon = float(epsilon)
     q.mode = MODE[mode] if isinstance(mode, str) else int(mode)
+    if view is not None:
+        if len(view) != 4:
+            raise ValueError("view = (c0, r0, c1, r1)")
+        for k in range(4):
+            q.view[k] = int(view[k])
     return q
+
+
+def lod_view(box, viewport, W, H=None):
+    """LOD zoom: the canvas resolution and pixel window that
+    render the world rectangle viewport = (vx0, vy0, vx1, vy1) with about
+    W x H pixels -- a window of a finer virtual canvas over the whole domain
+    (rounded outward to whole pixels).  Returns (W_full, H_full, view)."""
+    import math
+    H = H or W
+    bw, bh = box[2] - box[0], box[3] - box[1]
+    Wf = min(131072, max(1, int(round(W * bw / (viewport[2] - viewport[0])))))
+    Hf = min(131072, max(1, int(round(H * bh / (viewport[3] - viewport[1])))))
+    c0 = max(0, int(math.floor((viewport[0] - box[0]) / bw * Wf)))
+    r0 = max(0, int(math.floor((viewport[1] - box[1]) / bh * Hf)))
+    c1 = min(Wf, int(math.ceil((viewport[2] - box[0]) / bw * Wf)))
+    r1 = min(Hf, int(math.ceil((viewport[3] - box[1]) / bh * Hf)))
+    return Wf, Hf, (c0, r0, max(c1, c0 + 1), max(r1, r0 + 1))
 
 
 # ---- C-ABI names ------------------------------------------------------------

@@ -49,8 +49,12 @@ def test_resolve_epsilon_nyc(L, eps, W):
 def test_resolve_us_and_errors(L):
     assert rj.rj_resolve_canvas_domain((0, 0, 4.6e6, 2.9e6), rj.make_desc(epsilon=1000.0)) == (6506, 4102)
     assert rj.rj_resolve_canvas_domain((0, 0, 1, 1), rj.make_desc(W=640, H=480)) == (640, 480)
-    for q in (rj.make_desc(epsilon=0.0), rj.make_desc(epsilon=float("nan")), rj.make_desc(W=32769),
-              rj.make_desc(epsilon=1.0)):    # eps = 1 m on NYC -> 81912 > 32768
+    # reading Z21: up to 2^17 a side; eps = 1 m on NYC -> 81912 (as the oracle)
+    assert rj.rj_resolve_canvas_domain((0, 0, 57920, 57920), rj.make_desc(epsilon=1.0)) == (81912, 81912)
+    assert oracle.resolve(57920, 57920, 1.0) == (81912, 81912)
+    assert rj.rj_resolve_canvas_domain((0, 0, 1, 1), rj.make_desc(W=131072)) == (131072, 131072)
+    for q in (rj.make_desc(epsilon=0.0), rj.make_desc(epsilon=float("nan")), rj.make_desc(W=131073),
+              rj.make_desc(epsilon=0.5)):    # eps = 0.5 m on NYC -> 163824 > 131072
         box = (0, 0, 57920, 57920)
         with pytest.raises(rj.RJError) as e:
             rj.rj_resolve_canvas_domain(box, q)
@@ -80,3 +84,21 @@ def test_product_never_imports_oracle():
             if f.endswith((".py", ".cu", ".cuh", ".h", ".cpp")):
                 s = open(os.path.join(dp, f)).read()
                 assert "import oracle" not in s and "from oracle" not in s and "rj_oracle" not in s, f
+
+
+def test_desc_layout_matches_header(L):
+    # the ctypes mirror of rj_query_desc must match the C layout (view[4] last)
+    import ctypes
+    q = rj.make_desc(W=8, view=(1, 2, 3, 4))
+    assert list(q.view) == [1, 2, 3, 4]
+    # C layout: 3 x int32, 4 B padding, 5 x rj_pred (16 B), 2 x int32, double, mode, view[4], 4 B tail
+    assert rj.rj_query_desc.pred.offset == 16 and rj.rj_query_desc.epsilon.offset == 104
+    assert rj.rj_query_desc.view.offset == 116 and ctypes.sizeof(rj.rj_query_desc) == 136
+
+
+def test_lod_view_helper():
+    # zoom into [100, 150) x [100, 200) of [0,1024)^2 at 1000 px: an 20480-wide
+    # virtual canvas and its window
+    Wf, Hf, v = rj.lod_view((0, 0, 1024, 1024), (100, 100, 150, 200), 1000)
+    assert (Wf, Hf) == (20480, 10240)
+    assert v == (2000, 1000, 3000, 2000)

@@ -218,7 +218,7 @@ def test_errors():
         with pytest.raises((rjmod.RJError, ValueError)):
             R.query(W=64, **kw)
     with pytest.raises(rjmod.RJError) as e:
-        R.query(W=40000)
+        R.query(W=131073)                             # reading Z21: cap 2^17
     assert e.value.status == -3
     bad = PG.flatten([[np.array([(0, 0), (2000, 0), (0, 5)], float)]])
     with pytest.raises(rjmod.RJError) as e:

@@ -155,55 +155,47 @@ rj_status build_filter(Ctx *c, const rj_query_desc *q, int n_cols, const int *co
     }
     if (q->agg != RJ_COUNT && (q->agg_column < 0 || q->agg_column >= n_cols))
         return set_error(c, RJ_ERR_INVALID_ARGUMENT, "agg_column out of range");
-    // slots: int-range columns first, then float-predicate columns, then the agg column
+    // slots: the aggregated column first (slot 0: the kernels read it at a
+    // fixed index), then the other int-predicate columns, then the other
+    // float-predicate columns.  Every slot carries an inclusive int32 range
+    // (the whole int32 range unless int predicates narrow it), so the range
+    // check of any slot -- float columns included -- is exact.
     int slot_of[RJ_MAX_COLS];
     for (int k = 0; k < RJ_MAX_COLS; ++k) slot_of[k] = -1;
-    int64_t lo[RJ_MAX_COLS], hi[RJ_MAX_COLS];
+    int64_t lo[6], hi[6];
+    for (int s = 0; s < 6; ++s) { lo[s] = INT32_MIN; hi[s] = INT32_MAX; }
+    auto slot = [&](int col) {
+        if (slot_of[col] < 0) {
+            slot_of[col] = f.n_slots;
+            f.slot_col[f.n_slots] = col;
+            f.slot_is_float[f.n_slots] = col_dtype[col] == RJ_F32;
+            f.n_slots++;
+        }
+        return slot_of[col];
+    };
+    if (q->agg != RJ_COUNT) {
+        f.agg_slot = slot(q->agg_column);
+        f.agg_is_float = f.slot_is_float[f.agg_slot];
+    }
     for (int k = 0; k < q->n_pred; ++k) {
         const rj_pred &p = q->pred[k];
         if (col_dtype[p.column] != RJ_I32) continue;
-        if (slot_of[p.column] < 0) {
-            slot_of[p.column] = f.n_slots;
-            f.slot_col[f.n_slots] = p.column;
-            f.slot_is_float[f.n_slots] = 0;
-            lo[f.n_slots] = INT32_MIN;
-            hi[f.n_slots] = INT32_MAX;
-            f.n_slots++;
-        }
-        const int s = slot_of[p.column];
+        const int s = slot(p.column);
         int_range(p.op, p.value, lo[s], hi[s], f.never);
-    }
-    f.n_irange = f.n_slots;
-    for (int s = 0; s < f.n_irange; ++s) {
-        if (lo[s] > hi[s]) { f.never = 1; lo[s] = hi[s] = 0; }
-        f.ilo[s] = (int32_t)std::max<int64_t>(lo[s], INT32_MIN);
-        f.ihi[s] = (int32_t)std::min<int64_t>(hi[s], INT32_MAX);
     }
     for (int k = 0; k < q->n_pred; ++k) {
         const rj_pred &p = q->pred[k];
         if (col_dtype[p.column] != RJ_F32) continue;
-        if (slot_of[p.column] < 0) {
-            slot_of[p.column] = f.n_slots;
-            f.slot_col[f.n_slots] = p.column;
-            f.slot_is_float[f.n_slots] = 1;
-            f.n_slots++;
-        }
-        f.f_slot[f.n_fpred] = slot_of[p.column];
+        f.f_slot[f.n_fpred] = slot(p.column);
         f.f_op[f.n_fpred] = p.op;
         f.f_val[f.n_fpred] = (float)p.value;
         f.n_fpred++;
     }
-    // slots without an int range always pass the (unconditional) range check
-    for (int s = f.n_irange; s < 6; ++s) { f.ilo[s] = INT32_MIN; f.ihi[s] = INT32_MAX; }
-    if (q->agg != RJ_COUNT) {
-        if (slot_of[q->agg_column] < 0) {
-            slot_of[q->agg_column] = f.n_slots;
-            f.slot_col[f.n_slots] = q->agg_column;
-            f.slot_is_float[f.n_slots] = col_dtype[q->agg_column] == RJ_F32;
-            f.n_slots++;
-        }
-        f.agg_slot = slot_of[q->agg_column];
-        f.agg_is_float = f.slot_is_float[f.agg_slot];
+    f.n_irange = f.n_slots;
+    for (int s = 0; s < 6; ++s) {
+        if (lo[s] > hi[s]) { f.never = 1; lo[s] = hi[s] = 0; }
+        f.ilo[s] = (int32_t)std::max<int64_t>(lo[s], INT32_MIN);
+        f.ihi[s] = (int32_t)std::min<int64_t>(hi[s], INT32_MAX);
     }
     return RJ_OK;
 }

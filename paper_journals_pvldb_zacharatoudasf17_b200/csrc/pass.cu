@@ -391,12 +391,14 @@ rj_status launch_pass(Ctx *c, void *k, const PassArgs &a, size_t smem) {
 }
 
 // Kernel choice: COUNT always uses the pixel tile (cheapest per cell); SUM/AVG
-// uses polygon labels in bounded mode (no per-pixel fp64 atomics) and the
-// pixel tile in accurate mode (measured faster at C3); RJ_OPT_PASS overrides.
+// use polygon labels (no per-pixel fp64 shared atomics, which are CAS loops
+// on sm_100; measured faster at C3 and C4 in both modes); RJ_OPT_PASS
+// overrides.
 static bool use_label(const Ctx *c, const PassArgs &a, bool sum, bool accurate) {
+    (void)accurate;
     if (!sum || a.canvas) return false;              // the count canvas comes from the pixel tiles
     if (c->pass_variant >= 0) return c->pass_variant == 0;
-    return !accurate;
+    return true;
 }
 
 size_t point_pass_smem(const Ctx *c, const PassArgs &a, bool sum, bool accurate) {

@@ -197,13 +197,10 @@ __device__ __forceinline__ bool pass_point(const PassArgs &a, const Consts<NS> &
     return ok;
 }
 
+// the aggregated attribute is always slot 0 (build_filter)
 template <int NS>
-__device__ __forceinline__ uint32_t agg_bits(const PassArgs &a, const Win<NS> &w, int j) {
-    uint32_t ab = 0;
-#pragma unroll
-    for (int q = 0; q < NS; ++q)
-        if (q == a.f.agg_slot) ab = w.v[q][j];
-    return ab;
+__device__ __forceinline__ uint32_t agg_bits(const PassArgs &, const Win<NS> &w, int j) {
+    return w.v[0][j];
 }
 
 // append the boundary point j of each lane with bnd set to the warp queue

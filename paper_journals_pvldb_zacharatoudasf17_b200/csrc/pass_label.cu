@@ -56,27 +56,74 @@ struct Carry {
     double sum = 0.0;
 };
 
-template <bool ACC, int NS, bool FP>
+// Per-lane partials of the carry's label, filled by windows whose points all
+// carry that label (the common case: Morton order keeps a warp inside one
+// polygon for long stretches), folded into the carry when a window holds
+// another label.
+struct LaneAcc {
+    uint32_t cnt = 0;
+    double sum = 0.0;
+};
+
+// the aggregated attribute as binary64: AF = float32 column, else int32 (exact)
+template <bool AF>
+__device__ __forceinline__ double attr_d(uint32_t bits) {
+    return AF ? (double)__uint_as_float(bits) : (double)(int32_t)bits;
+}
+
+__device__ __forceinline__ void fold(LaneAcc &acc, Carry &cy) {
+    if (__any_sync(kFull, acc.cnt != 0u)) {
+        uint32_t c = acc.cnt;
+        double s = acc.sum;
+#pragma unroll
+        for (int o = 16; o; o >>= 1) {
+            c += __shfl_xor_sync(kFull, c, o);
+            s += __shfl_xor_sync(kFull, s, o);
+        }
+        cy.cnt += c;
+        cy.sum += s;
+        acc.cnt = 0;
+        acc.sum = 0.0;
+    }
+}
+
+template <bool ACC, int NS, bool FP, bool AF>
 __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh, const LabTile &t,
                                             const Consts<NS> &k, const Win<NS> &w, uint32_t first, uint32_t count,
-                                            Carry &cy, uint32_t &qn, uint32_t &n_pass, uint32_t &n_bnd) {
+                                            Carry &cy, LaneAcc &acc, uint32_t &qn, uint32_t &n_pass,
+                                            uint32_t &n_bnd) {
     const int lane = threadIdx.x & 31;
     uint32_t lab[kIPL];
-    bool spec = false;
+    bool spec = false, uni = true;
+    uint32_t okm = 0;
 #pragma unroll
     for (int j = 0; j < kIPL; ++j) {
         const bool ok = ((uint32_t)(lane * kIPL + j) - first) < count && pass_point<NS, FP>(a, k, w, j);
         n_pass += ok ? 1u : 0u;
+        okm |= ok ? 1u << j : 0u;
         const uint32_t px = mulhi(w.x[j], k.W4), py = mulhi(w.y[j], k.H4);
         lab[j] = ok ? lds(t.lab_base + (py * t.stride + px) * 4u) : kNone;
         spec |= lab[j] == kMulti || lab[j] == kBnd;
+        uni &= !ok || lab[j] == cy.lab;
     }
+    // fast path: every point of the window carries the carry's label (never
+    // MULTI / BND: the carry's label is a polygon or NONE)
+    if (__all_sync(kFull, uni)) {
+#pragma unroll
+        for (int j = 0; j < kIPL; ++j)
+            if ((okm >> j) & 1u) {
+                acc.cnt += 1u;
+                acc.sum += attr_d<AF>(agg_bits<NS>(a, w, j));
+            }
+        return;
+    }
+    fold(acc, cy);
     if (__any_sync(kFull, spec)) {                            // rare: overlaps, boundary pixels
 #pragma unroll
         for (int j = 0; j < kIPL; ++j) {
             if (lab[j] == kMulti)
                 multi_point(a, sh, t, mulhi(w.x[j], k.W4), mulhi(w.y[j], k.H4),
-                            attr_val(agg_bits<NS>(a, w, j), a.f.agg_is_float));
+                            attr_d<AF>(agg_bits<NS>(a, w, j)));
             if (ACC) {
                 enqueue<true, NS>(a, sh, w, j, lab[j] == kBnd, qn, n_bnd);   // adds <= 32
                 if (qn >= 32) spill_queue<true>(a, sh, qn, false);            // leaves < 32
@@ -101,7 +148,7 @@ __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh,
     for (int j = 0; j + 1 < kIPL; ++j) {
         const bool c = lab[j] != kNone;
         run += c ? 1u : 0u;
-        if (c) dsum += attr_val(agg_bits<NS>(a, w, j), a.f.agg_is_float);
+        if (c) dsum += attr_d<AF>(agg_bits<NS>(a, w, j));
         const bool tail = lab[j + 1] != lab[j];
         const bool defer = tail && !seen && cin;
         if (defer) { fcnt = run; fsum = dsum; flab = lab[j]; }
@@ -112,7 +159,7 @@ __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh,
     }
     if (lab[kIPL - 1] != kNone) {
         run += 1u;
-        dsum += attr_val(agg_bits<NS>(a, w, kIPL - 1), a.f.agg_is_float);
+        dsum += attr_d<AF>(agg_bits<NS>(a, w, kIPL - 1));
     }
     // lane 0 takes the carry as its incoming partial
     const bool lane0_in = lane == 0 && cin;
@@ -133,7 +180,7 @@ __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh,
     cy.sum = __shfl_sync(kFull, last_sum, 31);
 }
 
-template <bool ACC, int NS, bool FP>
+template <bool ACC, int NS, bool FP, bool AF>
 __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassArgs a) {
     extern __shared__ __align__(128) unsigned char smem_raw[];
     __shared__ __align__(8) Ring rg;
@@ -177,6 +224,7 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
         t.stride = a.tile_stride;
         uint32_t tsel = 0, n_pass = 0, n_bnd = 0, qn = 0;
         Carry cy;
+        LaneAcc acc;
         uint32_t st = 0, ph = 0;
         for (;;) {
             mbar_wait(smem_u32(&rg.full[st]), ph);
@@ -221,13 +269,15 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
             if (woff < ncopy && !never) {
                 Win<NS> w;
                 load_win_smem<NS>(w, ring + (size_t)st * ncol * kStagePts, woff + lane * kIPL);
-                process_lab<ACC, NS, FP>(a, sh, t, k, w, (m.sb - m.cb) - woff, m.se - m.sb, cy, qn, n_pass, n_bnd);
+                process_lab<ACC, NS, FP, AF>(a, sh, t, k, w, (m.sb - m.cb) - woff, m.se - m.sb, cy, acc, qn, n_pass,
+                                             n_bnd);
             }
             __syncwarp();
             if (lane == 0) mbar_arrive(smem_u32(&rg.empty[st]));
             if (++st == nstage) { st = 0; ph ^= 1u; }
         }
         if (ACC && qn) spill_queue<true>(a, sh, qn, true);
+        fold(acc, cy);
         if (lane == 0) emit_lab_run(a, sh, cy.lab, cy.cnt, cy.sum, true);
         for (int o = 16; o; o >>= 1) {
             n_pass += __shfl_xor_sync(kFull, n_pass, o);
@@ -250,18 +300,21 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
     }
 }
 
-template <bool ACC, bool FP>
+// SUM/AVG always stream the aggregated column (slot 0): NS >= 1
+template <bool ACC, bool FP, bool AF>
 void *select_ns(int ns) {
     switch (ns) {
-    case 0: return (void *)k_point_pass_label<ACC, 0, FP>;
-    case 1: return (void *)k_point_pass_label<ACC, 1, FP>;
-    case 2: return (void *)k_point_pass_label<ACC, 2, FP>;
-    case 3: return (void *)k_point_pass_label<ACC, 3, FP>;
-    case 4: return (void *)k_point_pass_label<ACC, 4, FP>;
-    case 5: return (void *)k_point_pass_label<ACC, 5, FP>;
-    default: return (void *)k_point_pass_label<ACC, 6, FP>;
+    case 1: return (void *)k_point_pass_label<ACC, 1, FP, AF>;
+    case 2: return (void *)k_point_pass_label<ACC, 2, FP, AF>;
+    case 3: return (void *)k_point_pass_label<ACC, 3, FP, AF>;
+    case 4: return (void *)k_point_pass_label<ACC, 4, FP, AF>;
+    case 5: return (void *)k_point_pass_label<ACC, 5, FP, AF>;
+    default: return (void *)k_point_pass_label<ACC, 6, FP, AF>;
     }
 }
+
+template <bool ACC, bool FP>
+void *select_af(int ns, bool af) { return af ? select_ns<ACC, FP, true>(ns) : select_ns<ACC, FP, false>(ns); }
 
 size_t label_smem(const PassArgs &a, bool, bool accurate) {
     size_t b = ring_bytes(a.n_stages, a.f.n_slots) + (size_t)a.tile_cap * 2 * 4;
@@ -277,8 +330,9 @@ rj_status point_pass_label(Ctx *c, const PassArgs &a_in, bool accurate) {
     a.n_stages = (uint32_t)choose_stages(a, label_smem, true, accurate, c->force_stages);
     if (!a.n_stages) return set_error(c, RJ_ERR_RESOLUTION, "point-pass tiles do not fit in shared memory");
     const bool fp = a.f.n_fpred > 0;
-    void *k = accurate ? (fp ? select_ns<true, true>(a.f.n_slots) : select_ns<true, false>(a.f.n_slots))
-                       : (fp ? select_ns<false, true>(a.f.n_slots) : select_ns<false, false>(a.f.n_slots));
+    const bool af = a.f.agg_is_float != 0;
+    void *k = accurate ? (fp ? select_af<true, true>(a.f.n_slots, af) : select_af<true, false>(a.f.n_slots, af))
+                       : (fp ? select_af<false, true>(a.f.n_slots, af) : select_af<false, false>(a.f.n_slots, af));
     return launch_pass(c, k, a, label_smem(a, true, accurate));
 }
 

@@ -25,8 +25,9 @@ struct Filter {
     int32_t n_slots = 0;          // columns streamed by the point pass (<= 6)
     int32_t slot_col[6];          // slot -> attribute column
     int32_t slot_is_float[6];
-    // integer-range predicates: slot s in [0, n_irange) has all its int32
-    // predicates merged into one inclusive range [ilo, ihi]
+    // integer-range predicates: every slot s has its int32 predicates merged
+    // into one inclusive range [ilo, ihi] (the whole int32 range when it has
+    // none); n_irange == n_slots
     int32_t n_irange = 0;
     int32_t ilo[6], ihi[6];
     // float32 predicates (slot, op, value)
@@ -34,7 +35,7 @@ struct Filter {
     int32_t f_slot[5], f_op[5];
     float f_val[5];
     int32_t never = 0;            // an int predicate can never hold
-    int32_t agg_slot = -1;        // slot of the summed attribute (SUM/AVG)
+    int32_t agg_slot = -1;        // slot of the summed attribute (SUM/AVG): always 0
     int32_t agg_is_float = 0;     // its dtype (avoids a dynamically indexed param)
 };
 

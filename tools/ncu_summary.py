@@ -31,6 +31,30 @@ def ncu_csv(args):
     return list(csv.reader(io.StringIO(out)))
 
 
+def _stalls(rep, kname):
+    """Warp stall shares from the SASS source page of one kernel of the report."""
+    src = ncu_csv(["-i", rep, "-k", "regex:" + kname, "-c", "1", "--page", "source", "--csv", "--print-source=sass"])
+    hdr = None
+    data = []
+    for r in src:
+        if "Warp Stall Sampling (All Samples)" in r:
+            hdr = {k: i for i, k in enumerate(r)}
+            continue
+        if hdr and len(r) == len(hdr):
+            data.append(r)
+    if not hdr or not data:
+        return []
+    stalls = [k for k in hdr if k.startswith("stall_") and "Not Issued" not in k]
+    f = lambda r, k: float(r[hdr[k]] or 0)
+    tot = sum(f(r, "Warp Stall Sampling (All Samples)") for r in data) or 1.0
+    st = {k: sum(f(r, k) for r in data) for k in stalls}
+    lines = ["", "### warp stall reasons (share of samples)"]
+    for k, v in sorted(st.items(), key=lambda x: -x[1])[:10]:
+        lines.append(f"- {k[6:]}: {v / tot * 100:.1f} %")
+    lines.append(f"- warp instructions executed: {sum(f(r, 'Instructions Executed') for r in data):.4g}")
+    return lines
+
+
 def summarize(rep):
     rows = ncu_csv(["-i", rep, "--page", "raw", "--csv"])
     h, units = rows[0], rows[1]
@@ -39,24 +63,16 @@ def summarize(rep):
     for r in rows[2:]:
         name = r[h.index("Kernel Name")] if "Kernel Name" in h else "?"
         lines.append(f"## {name}")
+        res = {}
         for m in METRICS:
             if m in h:
                 i = h.index(m)
                 lines.append(f"- {m} = {r[i]} {units[i]}")
-                result[m] = r[i]
-    src = ncu_csv(["-i", rep, "--page", "source", "--csv", "--print-source=sass"])
-    if len(src) > 2:
-        sh, data = src[1], src[2:]
-        ix = {k: i for i, k in enumerate(sh)}
-        stalls = [k for k in sh if k.startswith("stall_") and "Not Issued" not in k]
-        tot = sum(float(r[ix["Warp Stall Sampling (All Samples)"]] or 0) for r in data) or 1.0
-        st = {k: sum(float(r[ix[k]] or 0) for r in data) for k in stalls}
+                res[m] = r[i]
+        short = name.split("(")[0].split("::")[-1].split("<")[0]
+        lines += _stalls(rep, short)
         lines.append("")
-        lines.append("### warp stall reasons (share of samples)")
-        for k, v in sorted(st.items(), key=lambda x: -x[1])[:10]:
-            lines.append(f"- {k[6:]}: {v / tot * 100:.1f} %")
-        inst = sum(float(r[ix["Instructions Executed"]] or 0) for r in data)
-        lines.append(f"- warp instructions executed: {inst:.4g}")
+        result[short] = res
     return "\n".join(lines), result
 
 

@@ -320,6 +320,8 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     a.pieces = P.pp.pieces;
     a.mask = P.acc ? P.pp.mask : nullptr;
     a.mask_wpr = P.pp.mask_wpr;
+    a.bpiece_off = P.pp.bpiece_off;
+    a.bpieces = P.pp.bpieces;
     a.index_join = P.index;
     a.grid_off = c->grid_off.as<uint32_t>();
     a.grid_ent = c->grid_ent.as<uint32_t>();
@@ -362,6 +364,9 @@ static rj_status setup_bqueue(Ctx *c, Prepared &P) {
     a.bq_y = by.as<uint32_t>();
     a.bq_a = P.sum ? ba.as<uint32_t>() : nullptr;
     a.bq_cap = (uint32_t)want;
+    // chunks: a few per consumer warp of a full grid (2 CTAs x 8 warps per SM), 32..512 entries
+    const uint64_t warps = (uint64_t)c->num_sms * 16;
+    a.bq_chunk = (uint32_t)std::min<uint64_t>(512, std::max<uint64_t>(32, (want / (4 * warps)) & ~uint64_t(31)));
     return RJ_OK;
 }
 
@@ -606,6 +611,8 @@ rj_status rj_set_option(rj_ctx *c, int32_t option, int64_t value) {
     }
     return set_error(c, RJ_ERR_INVALID_ARGUMENT, "unknown option");
 }
+
+void *rj_get_stream(const rj_ctx *c) { return c ? (void *)c->stream : nullptr; }
 
 uint32_t rj_n_polygons(const rj_ctx *c) { return c ? c->n_poly : 0; }
 uint64_t rj_n_points(const rj_ctx *c) { return c ? c->n_pts : 0; }

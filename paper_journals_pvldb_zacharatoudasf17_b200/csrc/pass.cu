@@ -66,7 +66,7 @@ __device__ __forceinline__ void emit_pixel_run(const Tile &t, uint32_t key, uint
 // their points skip the tile and go to the warp queue.
 template <bool SUM, bool ACC, int NS, bool FP>
 __device__ __forceinline__ void process(const PassArgs &a, const Shared &sh, const Tile &t, const Consts<NS> &k,
-                                        const Win<NS> &w, uint32_t first, uint32_t count, uint32_t &qn,
+                                        const Win<NS> &w, uint32_t first, uint32_t count, BQ &bq,
                                         uint32_t &n_pass, uint32_t &n_bnd) {
     const int lane = threadIdx.x & 31;
     bool ok[kIPL];
@@ -85,8 +85,7 @@ __device__ __forceinline__ void process(const PassArgs &a, const Shared &sh, con
         if (__any_sync(kFull, bm != 0u)) {
 #pragma unroll
             for (int j = 0; j < kIPL; ++j) {
-                enqueue<SUM, NS>(a, sh, w, j, (bm >> j) & 1u, qn, n_bnd);   // adds <= 32
-                if (qn >= 32) spill_queue<SUM>(a, sh, qn, false);            // leaves < 32
+                enqueue<SUM, NS>(a, sh, w, j, (bm >> j) & 1u, bq, n_bnd);
             }
 #pragma unroll
             for (int j = 0; j < kIPL; ++j) ok[j] = ok[j] && !((bm >> j) & 1u);
@@ -182,7 +181,8 @@ __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a)
         Tile t;
         t.stride = a.tile_stride;
         uint32_t tsel = 0, pb = 0, pe = 0;
-        uint32_t n_pass = 0, n_bnd = 0, qn = 0;
+        uint32_t n_pass = 0, n_bnd = 0;
+        BQ bq = bq_init(a);
         uint32_t st = 0, ph = 0;
         for (;;) {
             mbar_wait(smem_u32(&rg.full[st]), ph);
@@ -208,13 +208,21 @@ __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a)
                 t.tbase = smem_u32(t.cnt) - 4u * t.base;
                 const uint32_t words = t.th * t.stride;
                 if (ACC) {
-                    clear_tile_acc(t.cnt, t.stride, t.th, t.tw, r0, c0, a.mask, a.mask_wpr, a.index_join, kFlag, 0u, a.view);
+                    clear_tile_acc(t.cnt, t.stride, t.th, t.tw, r0, c0, a.index_join, kFlag, 0u, a.view);
                 } else {
                     for (uint32_t i = threadIdx.x; i < words; i += kThreads) t.cnt[i] = 0u;
                 }
                 if (SUM)
                     for (uint32_t i = threadIdx.x; i < words; i += kThreads) t.sum[i] = 0.0;
                 consumers_sync();
+                if (ACC && !a.index_join) {
+                    // flag the cell's boundary pixels (cell-uniform branch: the barrier is safe)
+                    const uint32_t bb = __ldg(&a.bpiece_off[m.cell]), be = __ldg(&a.bpiece_off[m.cell + 1]);
+                    if (bb < be) {
+                        paint_bnd(t.cnt, t.stride, a.bpieces, bb, be, kFlag);
+                        consumers_sync();
+                    }
+                }
             }
             uint2 pc0 = make_uint2(0u, 0u);
             if ((m.flags & 2u) && pb + threadIdx.x < pe) pc0 = __ldg(&a.pieces[pb + threadIdx.x]);  // in flight
@@ -225,7 +233,7 @@ __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a)
                 Win<NS> w;
                 load_win_smem<NS>(w, ring + (size_t)st * ncol * kStagePts, woff + lane * kIPL);
                 const uint32_t first = (m.sb - m.cb) - woff;    // may wrap: unsigned range test
-                process<SUM, ACC, NS, FP>(a, sh, t, k, w, first, m.se - m.sb, qn, n_pass, n_bnd);
+                process<SUM, ACC, NS, FP>(a, sh, t, k, w, first, m.se - m.sb, bq, n_pass, n_bnd);
             }
             __syncwarp();
             if (lane == 0) mbar_arrive(smem_u32(&rg.empty[st]));
@@ -254,7 +262,7 @@ __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a)
             }
             if (++st == nstage) { st = 0; ph ^= 1u; }
         }
-        if (ACC && qn) spill_queue<SUM>(a, sh, qn, true);   // boundary points are independent of the tiles
+        if (ACC) bq_finish<SUM>(a, sh, bq);                 // boundary points are independent of the tiles
         for (int o = 16; o; o >>= 1) {
             n_pass += __shfl_xor_sync(kFull, n_pass, o);
             if (ACC) n_bnd += __shfl_xor_sync(kFull, n_bnd, o);
@@ -297,8 +305,9 @@ __global__ void __launch_bounds__(256) k_pip_queue(const __grid_constant__ PassA
         const uint32_t i = base + lane;
         uint32_t P = kNoPoly;
         double v = 0.0;
-        if (i < n) {
-            const uint32_t x = __ldcs(&a.bq_x[i]), y = __ldcs(&a.bq_y[i]);
+        const uint32_t x = i < n ? __ldcs(&a.bq_x[i]) : kDone;
+        if (x != kDone) {                                   // kDone: padding of a chunk
+            const uint32_t y = __ldcs(&a.bq_y[i]);
             if (SUM) v = attr_val(__ldcs(&a.bq_a[i]), a.f.agg_is_float);
             P = join_point<SUM>(a, sh, x, y, v);
         }

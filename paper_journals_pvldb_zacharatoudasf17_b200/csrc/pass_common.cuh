@@ -142,41 +142,6 @@ __device__ __noinline__ void drain_queue(const PassArgs &a, const Shared &sh, ui
     }
 }
 
-// Move the warp's queued boundary points to the global queue, 32 at a time
-// (`all`: also a last partial batch), for k_pip_queue to test after the pass:
-// the latency-bound grid walk then runs at full occupancy instead of holding
-// up the stage ring.  A reservation that does not fit the queue records its
-// base in bq_valid and the points are tested inline instead (drain_queue).
-template <bool SUM>
-__device__ __noinline__ void spill_queue(const PassArgs &a, const Shared &sh, uint32_t &qn, bool all) {
-    const int lane = threadIdx.x & 31;
-    while (qn >= 32 || (all && qn > 0)) {
-        __syncwarp();
-        const uint32_t take = qn >= 32 ? 32u : qn;
-        uint32_t base = 0;
-        if (lane == 0) {
-            base = atomicAdd(a.bq_count, take);
-            if (base + take > a.bq_cap) {
-                atomicMin(a.bq_valid, base);
-                base = kDone;
-            }
-        }
-        base = __shfl_sync(kFull, base, 0);
-        if (base == kDone) {
-            drain_queue<SUM>(a, sh, qn, all);
-            return;
-        }
-        if ((uint32_t)lane < take) {
-            const uint32_t pos = qn - take + lane;
-            a.bq_x[base + lane] = sh.qx[pos];
-            a.bq_y[base + lane] = sh.qy[pos];
-            if (SUM) a.bq_a[base + lane] = sh.qa[pos];
-        }
-        __syncwarp();
-        qn -= take;
-    }
-}
-
 template <int NS, bool FP>
 __device__ __forceinline__ bool pass_point(const PassArgs &a, const Consts<NS> &k, const Win<NS> &w, int j) {
     bool ok = true;
@@ -203,51 +168,117 @@ __device__ __forceinline__ uint32_t agg_bits(const PassArgs &, const Win<NS> &w,
     return w.v[0][j];
 }
 
-// append the boundary point j of each lane with bnd set to the warp queue
-template <bool SUM, int NS>
-__device__ __forceinline__ void enqueue(const PassArgs &a, const Shared &sh, const Win<NS> &w, int j, bool bnd,
-                                        uint32_t &qn, uint32_t &n_bnd) {
-    const unsigned bb = __ballot_sync(kFull, bnd);
-    if (bb) {
-        const int lane = threadIdx.x & 31;
-        if (bnd) {
-            const uint32_t pos = qn + __popc(bb & ((1u << lane) - 1u));
-            sh.qx[pos] = w.x[j];
-            sh.qy[pos] = w.y[j];
-            sh.qa[pos] = SUM ? agg_bits<NS>(a, w, j) : 0u;
-            ++n_bnd;
+// Boundary points of a warp (accurate mode).  Normally they go straight to
+// the global queue: the warp reserves chunks of bq_chunk entries with one
+// atomic each and fills them in order (boundary points are tested by
+// k_pip_queue after the pass, at full occupancy, instead of holding up the
+// stage ring with latency-bound grid walks).  A chunk is closed by padding its
+// unused entries with x = kDone.  When the queue is full the warp falls back
+// to its shared-memory queue, tested inline 32 at a time (drain_queue).
+struct BQ {
+    uint32_t pos = 0, end = 0;   // current chunk [pos, end) of the global queue (warp-uniform)
+    uint32_t qn = 0;             // fallback: entries in the warp's shared queue
+    bool global = false;         // chunks may still be reserved
+};
+
+__device__ __forceinline__ BQ bq_init(const PassArgs &a) {
+    BQ q;
+    q.global = a.bq_cap != 0;
+    return q;
+}
+
+// pad the rest of the current chunk with sentinels (x = kDone)
+__device__ __forceinline__ void bq_pad(const PassArgs &a, BQ &q) {
+    const uint32_t lane = threadIdx.x & 31;
+    for (uint32_t i = q.pos + lane; i < q.end; i += 32) a.bq_x[i] = kDone;
+    q.pos = q.end;
+}
+
+// close the current chunk and reserve the next (warp-collective)
+static __device__ __noinline__ void bq_next_chunk(const PassArgs &a, BQ &q) {
+    bq_pad(a, q);
+    uint32_t base = 0;
+    if ((threadIdx.x & 31) == 0) {
+        base = atomicAdd(a.bq_count, a.bq_chunk);
+        if (base + a.bq_chunk > a.bq_cap) {
+            atomicMin(a.bq_valid, base);
+            base = kDone;
         }
-        qn += __popc(bb);
+    }
+    base = __shfl_sync(kFull, base, 0);
+    if (base == kDone) {
+        q.global = false;
+        q.pos = q.end = 0;
+    } else {
+        q.pos = base;
+        q.end = base + a.bq_chunk;
     }
 }
 
-// Accurate-mode tile clear: word (r, x) of a th x stride tile becomes `flag`
-// when x < tw and pixel (c0 + x, r0 + r) is a boundary pixel (every pixel
-// when `all`, the index join), else `zero`.  Warp w clears rows w, w + 8, ...;
-// each row's <= 5 mask words are loaded once (one lane each) and shuffled to
-// the lanes that need them, and the row loop is unrolled so several rows'
-// loads are in flight (the clear sits between two consumer barriers, so its
-// L2 latency is exposed).
-// The index join (`all`) flags only the pixels inside the viewport window
-// view = (c0, r0, c1, r1) (the mask is already clipped to it).
-__device__ __forceinline__ void clear_tile_acc(uint32_t *tile, uint32_t stride, uint32_t th, uint32_t tw,
-                                               uint32_t r0, uint32_t c0, const uint32_t *mask, uint32_t wpr,
-                                               bool all, uint32_t flag, uint32_t zero, const int32_t *view) {
-    const uint32_t lane = threadIdx.x & 31, wid = threadIdx.x >> 5;
-    const uint32_t w0 = c0 >> 5;
-    const uint32_t nwords = ((c0 + tw - 1) >> 5) - w0 + 1;
-    const uint32_t vc0 = (uint32_t)view[0], vr0 = (uint32_t)view[1], vc1 = (uint32_t)view[2], vr1 = (uint32_t)view[3];
-#pragma unroll 4
-    for (uint32_t r = wid; r < th; r += kWarps) {
-        uint32_t word = 0xFFFFFFFFu;
-        if (!all && lane < nwords) word = __ldg(&mask[(uint64_t)(r0 + r) * wpr + w0 + lane]);
-        const bool row_in = !all || (r0 + r >= vr0 && r0 + r < vr1);
-        for (uint32_t x0 = 0; x0 < stride; x0 += 32) {
-            const uint32_t x = x0 + lane, px = c0 + x;
-            const uint32_t wv = __shfl_sync(kFull, word, ((px >> 5) - w0) & 31u);
-            const bool in = row_in && (!all || (px >= vc0 && px < vc1));
-            if (x < stride) tile[r * stride + x] = (x < tw && in && ((wv >> (px & 31)) & 1u)) ? flag : zero;
+// append point j of the lanes with bnd set
+template <bool SUM, int NS>
+__device__ __forceinline__ void enqueue(const PassArgs &a, const Shared &sh, const Win<NS> &w, int j, bool bnd,
+                                        BQ &q, uint32_t &n_bnd) {
+    const unsigned bb = __ballot_sync(kFull, bnd);
+    if (!bb) return;
+    const int lane = threadIdx.x & 31;
+    const uint32_t n = __popc(bb), rank = __popc(bb & ((1u << lane) - 1u));
+    n_bnd += bnd ? 1u : 0u;
+    if (q.global && q.pos + n > q.end) bq_next_chunk(a, q);
+    if (q.pos + n <= q.end) {
+        if (bnd) {
+            a.bq_x[q.pos + rank] = w.x[j];
+            a.bq_y[q.pos + rank] = w.y[j];
+            if (SUM) a.bq_a[q.pos + rank] = agg_bits<NS>(a, w, j);
         }
+        q.pos += n;
+        return;
+    }
+    if (bnd) {
+        const uint32_t pos = q.qn + rank;
+        sh.qx[pos] = w.x[j];
+        sh.qy[pos] = w.y[j];
+        sh.qa[pos] = SUM ? agg_bits<NS>(a, w, j) : 0u;
+    }
+    q.qn += n;
+    if (q.qn >= 32) drain_queue<SUM>(a, sh, q.qn, false);       // leaves < 32
+}
+
+// end of the pass: close the chunk, test what is left in the shared queue
+template <bool SUM>
+__device__ __forceinline__ void bq_finish(const PassArgs &a, const Shared &sh, BQ &q) {
+    bq_pad(a, q);
+    if (q.qn) drain_queue<SUM>(a, sh, q.qn, true);
+}
+
+// Accurate-mode tile setup, phase 1: word (r, x) of a th x stride tile
+// becomes `flag` for the pixels (c0 + x, r0 + r), x < tw, inside the viewport
+// window view = (c0, r0, c1, r1) when `all` (the index join: every pixel is a
+// boundary pixel), else `zero`.  Phase 2 (paint_bnd, after a barrier) flags
+// the cell's boundary pixels from its boundary pieces.
+__device__ __forceinline__ void clear_tile_acc(uint32_t *tile, uint32_t stride, uint32_t th, uint32_t tw,
+                                               uint32_t r0, uint32_t c0, bool all, uint32_t flag, uint32_t zero,
+                                               const int32_t *view) {
+    if (!all) {
+        for (uint32_t i = threadIdx.x; i < th * stride; i += kThreads) tile[i] = zero;
+        return;
+    }
+    const uint32_t vc0 = (uint32_t)view[0], vr0 = (uint32_t)view[1], vc1 = (uint32_t)view[2], vr1 = (uint32_t)view[3];
+    for (uint32_t i = threadIdx.x; i < th * stride; i += kThreads) {
+        const uint32_t r = i / stride, x = i - r * stride;
+        const bool in = x < tw && c0 + x >= vc0 && c0 + x < vc1 && r0 + r >= vr0 && r0 + r < vr1;
+        tile[i] = in ? flag : zero;
+    }
+}
+
+// Accurate-mode tile setup, phase 2: the boundary pixels of the cell (S5
+// supercover as pieces [bb, be), polygons.cu k_bnd_pieces) become `flag`.
+__device__ __forceinline__ void paint_bnd(uint32_t *tile, uint32_t stride, const uint32_t *bp, uint32_t bb,
+                                          uint32_t be, uint32_t flag) {
+    for (uint32_t kk = bb + threadIdx.x; kk < be; kk += kThreads) {
+        const uint32_t v = __ldg(&bp[kk]);
+        uint32_t *row = tile + (v & 255u) * stride;
+        for (uint32_t x = (v >> 8) & 255u, hi = v >> 16; x < hi; ++x) row[x] = flag;
     }
 }
 

@@ -90,7 +90,7 @@ __device__ __forceinline__ void fold(LaneAcc &acc, Carry &cy) {
 template <bool ACC, int NS, bool FP, bool AF>
 __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh, const LabTile &t,
                                             const Consts<NS> &k, const Win<NS> &w, uint32_t first, uint32_t count,
-                                            Carry &cy, LaneAcc &acc, uint32_t &qn, uint32_t &n_pass,
+                                            Carry &cy, LaneAcc &acc, BQ &bq, uint32_t &n_pass,
                                             uint32_t &n_bnd) {
     const int lane = threadIdx.x & 31;
     uint32_t lab[kIPL];
@@ -125,8 +125,7 @@ __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh,
                 multi_point(a, sh, t, mulhi(w.x[j], k.W4), mulhi(w.y[j], k.H4),
                             attr_d<AF>(agg_bits<NS>(a, w, j)));
             if (ACC) {
-                enqueue<true, NS>(a, sh, w, j, lab[j] == kBnd, qn, n_bnd);   // adds <= 32
-                if (qn >= 32) spill_queue<true>(a, sh, qn, false);            // leaves < 32
+                enqueue<true, NS>(a, sh, w, j, lab[j] == kBnd, bq, n_bnd);
             }
             if (lab[j] >= kBnd) lab[j] = kNone;
         }
@@ -222,7 +221,8 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
         const bool never = a.f.never != 0;
         LabTile t;
         t.stride = a.tile_stride;
-        uint32_t tsel = 0, n_pass = 0, n_bnd = 0, qn = 0;
+        uint32_t tsel = 0, n_pass = 0, n_bnd = 0;
+        BQ bq = bq_init(a);
         Carry cy;
         LaneAcc acc;
         uint32_t st = 0, ph = 0;
@@ -247,19 +247,36 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
                     t.pe = __ldg(&a.piece_off[m.cell + 1]);
                 }
                 if (ACC) {
-                    clear_tile_acc(lt, t.stride, th, tw, t.r0, t.c0, a.mask, a.mask_wpr, a.index_join, kBnd, kNone, a.view);
+                    clear_tile_acc(lt, t.stride, th, tw, t.r0, t.c0, a.index_join, kBnd, kNone, a.view);
                 } else {
                     for (uint32_t i = threadIdx.x; i < th * t.stride; i += kThreads) lt[i] = kNone;
                 }
                 consumers_sync();
-                // one thread per span piece; shared CAS turns overlaps into MULTI
+                // one thread per piece.  Labels only move up the order
+                // polygon < MULTI < BND: a polygon claims NONE, a second
+                // polygon turns a polygon into MULTI (CAS, so a concurrent
+                // BND is never overwritten), boundary pixels become BND.
                 for (uint32_t kk = t.pb + threadIdx.x; kk < t.pe; kk += kThreads) {
                     const uint2 pc = __ldg(&a.pieces[kk]);
                     uint32_t *row = lt + (pc.y & 255u) * t.stride;
                     const uint32_t lo = (pc.y >> 8) & 255u, hi = pc.y >> 16;
                     for (uint32_t x = lo; x < hi; ++x) {
-                        const uint32_t o = atomicCAS(&row[x], kNone, pc.x);
-                        if (o != kNone && o < kBnd) atomicExch(&row[x], kMulti);   // BND / MULTI stay
+                        uint32_t o = atomicCAS(&row[x], kNone, pc.x);
+                        while (o < kBnd) {
+                            const uint32_t o2 = atomicCAS(&row[x], o, kMulti);
+                            if (o2 == o) break;
+                            o = o2;
+                        }
+                    }
+                }
+                if (ACC && !a.index_join) {
+                    const uint32_t bb = __ldg(&a.bpiece_off[m.cell]), be = __ldg(&a.bpiece_off[m.cell + 1]);
+                    for (uint32_t kk = bb + threadIdx.x; kk < be; kk += kThreads) {
+                        const uint32_t v = __ldg(&a.bpieces[kk]);
+                        uint32_t *row = lt + (v & 255u) * t.stride;
+                        // plain stores: a polygon's CAS never overwrites BND, and BND
+                        // landing after a CAS wins either way
+                        for (uint32_t x = (v >> 8) & 255u, hi = v >> 16; x < hi; ++x) row[x] = kBnd;
                     }
                 }
                 consumers_sync();
@@ -269,14 +286,14 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
             if (woff < ncopy && !never) {
                 Win<NS> w;
                 load_win_smem<NS>(w, ring + (size_t)st * ncol * kStagePts, woff + lane * kIPL);
-                process_lab<ACC, NS, FP, AF>(a, sh, t, k, w, (m.sb - m.cb) - woff, m.se - m.sb, cy, acc, qn, n_pass,
+                process_lab<ACC, NS, FP, AF>(a, sh, t, k, w, (m.sb - m.cb) - woff, m.se - m.sb, cy, acc, bq, n_pass,
                                              n_bnd);
             }
             __syncwarp();
             if (lane == 0) mbar_arrive(smem_u32(&rg.empty[st]));
             if (++st == nstage) { st = 0; ph ^= 1u; }
         }
-        if (ACC && qn) spill_queue<true>(a, sh, qn, true);
+        if (ACC) bq_finish<true>(a, sh, bq);
         fold(acc, cy);
         if (lane == 0) emit_lab_run(a, sh, cy.lab, cy.cnt, cy.sum, true);
         for (int o = 16; o; o >>= 1) {

@@ -260,6 +260,32 @@ __global__ void k_mask_mark(const int4 *__restrict__ edges, const uint32_t *__re
     }
 }
 
+// S5 as pieces (accurate mode): the supercover column range of every (edge,
+// row band) -- the pixels the boundary mask marks -- clipped to the window and
+// cut at the level-L point cells, binned per cell as (local row, lo, hi).
+// The point-pass kernels paint them into their tiles from this list instead
+// of reading the mask rows per cell (a dependent global load between two
+// CTA barriers).  A pixel touched by several edges appears several times.
+template <bool EMIT>
+__global__ void k_bnd_pieces(SpanGeo g, const int4 *__restrict__ edges, const uint32_t *__restrict__ band_off,
+                             uint32_t n_edges, uint32_t *__restrict__ cnt, const uint32_t *__restrict__ off,
+                             uint32_t *__restrict__ cur, uint32_t *__restrict__ out) {
+    const uint32_t total = band_off[n_edges];
+    for (uint32_t j = blockIdx.x * blockDim.x + threadIdx.x; j < total; j += gridDim.x * blockDim.x) {
+        const uint32_t e = upper_bound_u32(band_off, n_edges + 1, j) - 1;
+        const int4 E = edges[e];
+        const int64_t r = pix(min(E.y, E.w), g.H) + (j - band_off[e]);
+        int64_t i0, i1;
+        if (!supercover_cols(E.x, E.y, E.z, E.w, r, g.W, g.H, i0, i1)) continue;
+        int64_t lo = i0, hi = i1 + 1;
+        if (!clip_span(g, r, lo, hi)) continue;
+        for_each_piece(g, r, lo, hi, [&](uint32_t cell, uint32_t lr, uint32_t a, uint32_t b) {
+            if (EMIT) out[off[cell] + atomicAdd(&cur[cell], 1u)] = lr | (a << 8) | (b << 16);
+            else atomicAdd(&cnt[cell], 1u);
+        });
+    }
+}
+
 }  // namespace
 
 // ------------------------------------------------------------------- loading
@@ -446,12 +472,30 @@ rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp,
     RJ_CUDA(c, cudaGetLastError());
     RJ_CUDA(c, scan_u32(c, scnt.as<uint32_t>(), soff.as<uint32_t>(), NPR, kWsScan));
     if (ncell) RJ_CUDA(c, scan_u32(c, pcnt.as<uint32_t>(), poff.as<uint32_t>(), ncell, kWsScan));
+    // accurate mode with point cells: boundary pieces (count pass)
+    const bool bnd_pieces = accurate && ncell;
+    const uint32_t B = accurate ? hs[2] : 0;
+    Buf &bpc = wsbuf(c, kWsBPCount), &bpo = wsbuf(c, kWsBPOff), &bpu = wsbuf(c, kWsBPCursor);
+    const unsigned gb = (unsigned)std::min<uint64_t>(std::max<uint64_t>(1, blocks_for(B, 256)), c->num_sms * 8ull);
+    if (bnd_pieces) {
+        if (dreserve(c, bpc, (ncell + 1) * 4) || dreserve(c, bpo, (ncell + 1) * 4) || dreserve(c, bpu, (ncell + 1) * 4))
+            return set_error(c, RJ_ERR_OOM, "workspace allocation failed");
+        RJ_CUDA(c, cudaMemsetAsync(bpc.p, 0, (ncell + 1) * 4, st));
+        RJ_CUDA(c, cudaMemsetAsync(bpu.p, 0, (ncell + 1) * 4, st));
+        k_bnd_pieces<false><<<gb, 256, 0, st>>>(g, c->edges.as<int4>(), boff.as<uint32_t>(), ne, bpc.as<uint32_t>(),
+                                                nullptr, nullptr, nullptr);
+        RJ_LAUNCHED(c);
+        RJ_CUDA(c, cudaGetLastError());
+        RJ_CUDA(c, scan_u32(c, bpc.as<uint32_t>(), bpo.as<uint32_t>(), ncell, kWsScan));
+    }
     // sync 2: span / piece totals
     hs[4] = 0;
+    hs[5] = 0;
     RJ_CUDA(c, cudaMemcpyAsync(hs + 3, soff.as<uint32_t>() + NPR, 4, cudaMemcpyDeviceToHost, st));
     if (ncell) RJ_CUDA(c, cudaMemcpyAsync(hs + 4, poff.as<uint32_t>() + ncell, 4, cudaMemcpyDeviceToHost, st));
+    if (bnd_pieces) RJ_CUDA(c, cudaMemcpyAsync(hs + 5, bpo.as<uint32_t>() + ncell, 4, cudaMemcpyDeviceToHost, st));
     RJ_CUDA(c, cudaStreamSynchronize(st));
-    const uint32_t S = hs[3], NP = hs[4];
+    const uint32_t S = hs[3], NP = hs[4], NB = hs[5];
     Buf &spans = wsbuf(c, kWsSpans), &pieces = wsbuf(c, kWsPieces);
     if (dreserve(c, spans, (uint64_t)(S + 1) * 16) || dreserve(c, pieces, (uint64_t)(NP + 1) * 8))
         return set_error(c, RJ_ERR_OOM, "workspace allocation failed");
@@ -461,6 +505,18 @@ rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp,
     RJ_LAUNCHED(c);
     RJ_CUDA(c, cudaGetLastError());
 
+    if (bnd_pieces) {
+        Buf &bp = wsbuf(c, kWsBPieces);
+        if (dreserve(c, bp, (uint64_t)(NB + 1) * 4)) return set_error(c, RJ_ERR_OOM, "workspace allocation failed");
+        k_bnd_pieces<true><<<gb, 256, 0, st>>>(g, c->edges.as<int4>(), boff.as<uint32_t>(), ne, nullptr,
+                                               bpo.as<uint32_t>(), bpu.as<uint32_t>(), bp.as<uint32_t>());
+        RJ_LAUNCHED(c);
+        RJ_CUDA(c, cudaGetLastError());
+        pp.bpiece_off = bpo.as<uint32_t>();
+        pp.bpieces = bp.as<uint32_t>();
+        pp.n_bpieces = NB;
+    }
+
     pp.n_cross = X;
     pp.n_spans = S;
     pp.n_pieces = NP;
@@ -468,13 +524,11 @@ rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp,
     pp.piece_off = poff.as<uint32_t>();
     pp.pieces = pieces.as<uint2>();
     if (accurate) {
-        const uint32_t B = hs[2];
         pp.n_bands = B;
         const uint32_t wpr = (uint32_t)((W + 31) / 32);
         Buf &mask = wsbuf(c, kWsMask);
         if (dreserve(c, mask, (uint64_t)wpr * H * 4)) return set_error(c, RJ_ERR_OOM, "mask allocation failed");
         RJ_CUDA(c, cudaMemsetAsync(mask.p, 0, (uint64_t)wpr * H * 4, st));
-        const unsigned gb = (unsigned)std::min<uint64_t>(std::max<uint64_t>(1, blocks_for(B, 256)), c->num_sms * 8ull);
         const int4 vw = v.full ? make_int4(0, 0, W, H) : make_int4(v.c0, v.r0, v.c1, v.r1);
         k_mask_mark<<<gb, 256, 0, st>>>(c->edges.as<int4>(), boff.as<uint32_t>(), ne, W, H, wpr, mask.as<uint32_t>(),
                                         vw);

@@ -60,8 +60,10 @@ struct PassArgs {
     uint32_t tile_stride;         // row stride of a warp's tile (odd: conflict-free row prefix)
     const uint32_t *piece_off;    // [4^L + 1]
     const uint2 *pieces;
-    const uint32_t *mask;         // accurate: boundary bitmask
+    const uint32_t *mask;         // accurate: boundary bitmask (diagnostics; the kernels use bpieces)
     uint32_t mask_wpr;
+    const uint32_t *bpiece_off;   // accurate: boundary pieces per point cell [4^L + 1]
+    const uint32_t *bpieces;      // (local row | lo << 8 | hi << 16)
     const uint32_t *grid_off;     // accurate: edge grid CSR
     const uint32_t *grid_ent;
     const int4 *grid_edge;        // per entry: (xa, ya, xb, yb)
@@ -84,6 +86,7 @@ struct PassArgs {
     // bq_cap == 0 -> tested inline by the consumer warps
     uint32_t *bq_x, *bq_y, *bq_a;
     uint32_t bq_cap;
+    uint32_t bq_chunk;            // entries a warp reserves at a time
     uint32_t *bq_count;           // entries reserved
     uint32_t *bq_valid;           // first failed reservation (entries below it are written)
 };
@@ -158,6 +161,7 @@ enum : int {
     kWsLab, kWsRowCount, kWsRowOff, kWsRowCursor, kWsRowSpans, kWsStream,   // streamed query
     kWsCanvas, kWsBRowCount, kWsBRowOff, kWsBktCount, kWsBktOff, kWsBktCursor, kWsBktRanges,   // intervals
     kWsBQx, kWsBQy, kWsBQa,                 // accurate mode: global boundary-point queue
+    kWsBPCount, kWsBPOff, kWsBPCursor, kWsBPieces,   // accurate mode: boundary pieces per point cell
     kWsScan = 72,                           // 72..95 recursive scan temporaries
 };
 
@@ -224,6 +228,9 @@ struct PolyPass {
     uint2 *pieces = nullptr;
     uint32_t *mask = nullptr;        // accurate only
     uint32_t mask_wpr = 0;
+    uint32_t *bpiece_off = nullptr;  // accurate with point cells: [4^L + 1]
+    uint32_t *bpieces = nullptr;     // (local row | lo << 8 | hi << 16) of boundary pixels
+    uint64_t n_bpieces = 0;
 };
 // Spans, pieces and the boundary mask are clipped to the viewport window v.
 rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp, const View &v);

@@ -43,12 +43,18 @@ def query_sharded(R: "rj.RasterJoin", desc, d_count: torch.Tensor, d_sum: torch.
                   group=None):
     """Partials on this rank's shard -> all-reduce -> finalise (all on device).
 
-    R's stream must be torch's current stream (create R with
-    stream=torch.cuda.current_stream().cuda_stream) so NCCL orders after it."""
+    The query and the finalisation run on the context's stream (rj_get_stream),
+    the collective on torch's current stream; each waits for the other, so any
+    stream choice at rj_create is safe."""
     rj.rj_query_device(R.ctx, desc, d_count, d_sum)
+    ctx_stream = torch.cuda.ExternalStream(rj.rj_get_stream(R.ctx))
+    cur = torch.cuda.current_stream()
+    cur.wait_stream(ctx_stream)
     if dist.get_backend(group) == "gloo":
         # gloo stages device tensors through the host outside the stream order
-        torch.cuda.current_stream().synchronize()
+        cur.synchronize()
     allreduce_partials(d_count, d_sum if desc.agg != 0 else None, group)
+    ctx_stream.wait_stream(cur)
     rj.rj_finalize_device(R.ctx, desc.agg, d_count, d_sum, d_value)
+    cur.wait_stream(ctx_stream)
     return d_value

@@ -98,6 +98,7 @@ def lib():
             "rj_debug_point_membership": (i32, [vp, qp, vp]),
             "rj_get_stats": (i32, [vp, ctypes.POINTER(rj_stats)]),
             "rj_set_option": (i32, [vp, i32, ctypes.c_int64]),
+            "rj_get_stream": (vp, [vp]),
             "rj_n_polygons": (u32, [vp]),
             "rj_n_points": (u64, [vp]),
             "rj_status_str": (ctypes.c_char_p, [i32]),
@@ -115,7 +116,7 @@ def lib():
 EXPORTS = ["rj_create", "rj_destroy", "rj_set_allocator", "rj_load_points", "rj_load_polygons", "rj_query",
            "rj_query_device", "rj_query_stream", "rj_query_interval", "rj_query_multi", "rj_debug_point_canvas", "rj_finalize_device", "rj_resolve_canvas", "rj_resolve_canvas_domain",
            "rj_debug_pixel_spans", "rj_debug_boundary_mask", "rj_debug_point_membership", "rj_get_stats",
-           "rj_set_option", "rj_n_polygons", "rj_n_points", "rj_status_str", "rj_last_error", "rj_version"]
+           "rj_set_option", "rj_get_stream", "rj_n_polygons", "rj_n_points", "rj_status_str", "rj_last_error", "rj_version"]
 
 
 def _check(status, ctx=None):
@@ -266,6 +267,11 @@ def rj_resolve_canvas(ctx, desc):
     W, H = ctypes.c_int32(), ctypes.c_int32()
     _check(lib().rj_resolve_canvas(ctx, ctypes.byref(desc), ctypes.byref(W), ctypes.byref(H)), ctx)
     return W.value, H.value
+
+
+def rj_get_stream(ctx):
+    """cudaStream_t (as an int) the context issues its work on."""
+    return lib().rj_get_stream(ctx) or 0
 
 
 def rj_get_stats(ctx):

@@ -75,6 +75,12 @@ def lib():
                                       i32, i32, vp]
         L.or_error_interval.restype = None
         L.or_error_interval.argtypes = [vp, i32, i32, vp, vp, vp]
+        L.or_ring_sigma.restype = i32
+        L.or_ring_sigma.argtypes = [vp, i64, i64]
+        L.or_area_fraction.restype = d
+        L.or_area_fraction.argtypes = [vp, i64, i64, i64, i32, i32]
+        L.or_expected_interval.restype = None
+        L.or_expected_interval.argtypes = [vp, i32, i32, vp, vp, vp]
         _lib = L
     return _lib
 
@@ -232,4 +238,23 @@ def error_interval(polys, W, H, counts):
     ep = np.zeros(polys.n, dtype=np.uint64)
     em = np.zeros(polys.n, dtype=np.uint64)
     lib().or_error_interval(polys.h, int(W), int(H), counts.ctypes.data, ep.ctypes.data, em.ctypes.data)
+    return ep, em
+
+
+def ring_sigma(polys, P, r):
+    """O13: orientation(ring r) * (-1)^depth -- the ring's even-odd weight."""
+    return int(lib().or_ring_sigma(polys.h, int(P), int(r)))
+
+
+def area_fraction(polys, P, i, r, W, H):
+    """O13: fraction of pixel (i, r)'s lattice rectangle inside polygon P."""
+    return float(lib().or_area_fraction(polys.h, int(P), int(i), int(r), int(W), int(H)))
+
+
+def expected_interval(polys, W, H, counts):
+    """O13: (E+, E-) per polygon, binary64."""
+    counts = np.ascontiguousarray(counts, np.uint32)
+    ep = np.zeros(polys.n, dtype=np.float64)
+    em = np.zeros(polys.n, dtype=np.float64)
+    lib().or_expected_interval(polys.h, int(W), int(H), counts.ctypes.data, ep.ctypes.data, em.ctypes.data)
     return ep, em

@@ -39,6 +39,8 @@
  *       IEEE 754 totalOrder for float32 (-NaN < -inf < ... < -0 < +0 < ...
  *       < +inf < +NaN, NaNs further ordered by payload; reading Z16), plain
  *       order for int32; NaN result for a polygon without points.
+ *   O13 expected interval [A - E+, A + E-] with the pixel-polygon area
+ *       fraction f (reading Z22).
  */
 #include <math.h>
 #include <stdint.h>
@@ -562,6 +564,126 @@ OR_EXPORT void or_error_interval(const or_polys *p, int W, int H, const uint32_t
                 }
         eplus[P] = ep;
         eminus[P] = em;
+    }
+    free(bits);
+}
+
+/* --------------------------------------------------------------------- O13
+ * Expected result interval: under a uniform distribution of the
+ * points inside each pixel, a boundary pixel (x,y) of polygon i holds
+ * f_i(x,y) x Fpt(x,y) points that are really inside i, where f_i(x,y) is
+ * "the fraction area of the pixel that intersects polygon i".
+ * Reading Z22: the garbled formula writes f_i for both sums; the
+ * expected number of false positives in a P+ pixel (centre inside, whole
+ * pixel counted) is (1 - f) Fpt and of false negatives in a P- pixel is
+ * f Fpt, so
+ *     E+_i = sum over P+_i of (1 - f_i) Fpt,  E-_i = sum over P-_i of f_i Fpt,
+ * and the expected interval is [A - E+, A + E-].
+ *
+ * The pixel's region is the half-open lattice rectangle
+ * [qlo(i), qlo(i+1)) x [qlo(r), qlo(r+1)) (O2: a lattice point Q stands for
+ * [Q, Q+1), and the pixel of Q changes exactly at qlo).  Even-odd area of
+ * polygon i inside it: every ring is clipped to the rectangle
+ * (Sutherland-Hodgman; the clip of a closed ring against a convex window
+ * keeps its signed area) and its signed shoelace area is added with weight
+ * sigma_r = orientation(ring) * (-1)^depth(ring), depth = number of the
+ * polygon's other rings containing the ring's first vertex (O3).  This is
+ * the even-odd area whenever the rings of a polygon neither cross
+ * themselves nor each other; for other rings it is the winding-weighted
+ * area (reading Z22).  f is clamped to [0, 1]. */
+static int or_ring_contains(const or_polys *p, int64_t r, int64_t px, int64_t py) {
+    int inside = 0;
+    int64_t v0 = p->vert_off[r], v1 = p->vert_off[r + 1];
+    for (int64_t a = v0; a < v1; ++a) {
+        int64_t b = (a + 1 < v1) ? a + 1 : v0;
+        int64_t xa = p->qx[a], ya = p->qy[a], xb = p->qx[b], yb = p->qy[b];
+        if ((ya > py) != (yb > py)) {
+            int64_t lhs = (px - xa) * (yb - ya);
+            int64_t rhs = (xb - xa) * (py - ya);
+            if (yb > ya ? lhs < rhs : lhs > rhs) inside = !inside;
+        }
+    }
+    return inside;
+}
+
+OR_EXPORT int or_ring_sigma(const or_polys *p, int64_t P, int64_t r) {
+    __int128 s = 0;                                    /* twice the signed area, exact */
+    int64_t v0 = p->vert_off[r], v1 = p->vert_off[r + 1];
+    for (int64_t a = v0; a < v1; ++a) {
+        int64_t b = (a + 1 < v1) ? a + 1 : v0;
+        s += (__int128)p->qx[a] * p->qy[b] - (__int128)p->qx[b] * p->qy[a];
+    }
+    int orient = (s > 0) - (s < 0);
+    int depth = 0;
+    for (int64_t o = p->ring_off[P]; o < p->ring_off[P + 1]; ++o)
+        if (o != r && or_ring_contains(p, o, p->qx[v0], p->qy[v0])) ++depth;
+    return (depth & 1) ? -orient : orient;
+}
+
+/* keep the part of polygon (xs, ys)[n] with s * (coord - c) >= 0 on axis ax */
+static int64_t or_clip_half(const double *xs, const double *ys, int64_t n, int ax, double c, double s,
+                            double *ox, double *oy) {
+    int64_t m = 0;
+    for (int64_t k = 0; k < n; ++k) {
+        int64_t l = (k + 1 < n) ? k + 1 : 0;
+        double ak = s * ((ax ? ys[k] : xs[k]) - c), al = s * ((ax ? ys[l] : xs[l]) - c);
+        if (ak >= 0) { ox[m] = xs[k]; oy[m] = ys[k]; ++m; }
+        if ((ak >= 0) != (al >= 0)) {                 /* the edge crosses the line */
+            double t = ak / (ak - al);
+            if (ax) { ox[m] = xs[k] + t * (xs[l] - xs[k]); oy[m] = c; }
+            else { ox[m] = c; oy[m] = ys[k] + t * (ys[l] - ys[k]); }
+            ++m;
+        }
+    }
+    return m;
+}
+
+OR_EXPORT double or_area_fraction(const or_polys *p, int64_t P, int64_t i, int64_t r, int W, int H) {
+    int64_t X0 = or_qlo(i, W), X1 = or_qlo(i + 1, W), Y0 = or_qlo(r, H), Y1 = or_qlo(r + 1, H);
+    double w = (double)(X1 - X0), h = (double)(Y1 - Y0), area = 0.0;
+    for (int64_t rg = p->ring_off[P]; rg < p->ring_off[P + 1]; ++rg) {
+        int64_t v0 = p->vert_off[rg], n = p->vert_off[rg + 1] - v0, cap = 16 * n + 64;
+        double *buf = (double *)malloc(sizeof(double) * 4 * (size_t)cap);
+        double *ax = buf, *ay = buf + cap, *bx = buf + 2 * cap, *by = buf + 3 * cap;
+        for (int64_t k = 0; k < n; ++k) {              /* pixel-local coordinates (exact) */
+            ax[k] = (double)(p->qx[v0 + k] - X0);
+            ay[k] = (double)(p->qy[v0 + k] - Y0);
+        }
+        int64_t m = or_clip_half(ax, ay, n, 0, 0.0, 1.0, bx, by);      /* x >= 0 */
+        m = or_clip_half(bx, by, m, 0, w, -1.0, ax, ay);               /* x <= w */
+        m = or_clip_half(ax, ay, m, 1, 0.0, 1.0, bx, by);              /* y >= 0 */
+        m = or_clip_half(bx, by, m, 1, h, -1.0, ax, ay);               /* y <= h */
+        double s = 0.0;
+        for (int64_t k = 0; k < m; ++k) {
+            int64_t l = (k + 1 < m) ? k + 1 : 0;
+            s += ax[k] * ay[l] - ax[l] * ay[k];
+        }
+        area += or_ring_sigma(p, P, rg) * 0.5 * s;
+        free(buf);
+    }
+    double f = area / (w * h);
+    return f < 0.0 ? 0.0 : (f > 1.0 ? 1.0 : f);
+}
+
+/* O13: expected interval sums over the same boundary pixels as O10. */
+OR_EXPORT void or_expected_interval(const or_polys *p, int W, int H, const uint32_t *pixel_counts,
+                                    double *eplus, double *eminus) {
+    int64_t wpr = (W + 31) / 32;
+    uint32_t *bits = (uint32_t *)malloc(sizeof(uint32_t) * (size_t)wpr * H);
+    for (int64_t P = 0; P < p->n_poly; ++P) {
+        or_boundary_mask(p, P, P + 1, W, H, bits);
+        double ep = 0.0, em = 0.0, cp = 0.0, cm = 0.0;
+        for (int64_t r = 0; r < H; ++r)
+            for (int64_t i = 0; i < W; ++i)
+                if (bits[r * wpr + i / 32] >> (i % 32) & 1) {
+                    uint32_t c = pixel_counts[r * W + i];
+                    if (!c) continue;
+                    double f = or_area_fraction(p, P, i, r, W, H);
+                    if (or_contains(p, P, or_centre(i, W), or_centre(r, H))) or_nadd(&ep, &cp, (1.0 - f) * c);
+                    else or_nadd(&em, &cm, f * c);
+                }
+        eplus[P] = ep + cp;
+        eminus[P] = em + cm;
     }
     free(bits);
 }

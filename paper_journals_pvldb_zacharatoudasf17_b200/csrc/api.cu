@@ -737,8 +737,8 @@ rj_status rj_query_multi(rj_ctx *c, const rj_query_desc *q, int32_t n_aggs, cons
     return label_query_with_cols(c, q, ap, lattice_input(c), c->n_cols, count, values);
 }
 
-rj_status rj_query_interval(rj_ctx *c, const rj_query_desc *q, uint64_t *count, double *value, uint64_t *eps_plus,
-                            uint64_t *eps_minus) {
+static rj_status query_interval(rj_ctx *c, const rj_query_desc *q, uint64_t *count, double *value,
+                                uint64_t *eps_plus, uint64_t *eps_minus, double *exp_plus, double *exp_minus) {
     if (q && q->mode != RJ_BOUNDED) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "result intervals need RJ_BOUNDED");
     if (q && (q->view[0] || q->view[1] || q->view[2] || q->view[3]))
         return set_error(c, RJ_ERR_INVALID_ARGUMENT, "result intervals need the whole canvas (view all zero)");
@@ -748,22 +748,36 @@ rj_status rj_query_interval(rj_ctx *c, const rj_query_desc *q, uint64_t *count, 
     const size_t n = c->n_poly;
     Buf &cv = wsbuf(c, kWsCanvas);
     if (dreserve(c, c->res_cnt, n * 8) || dreserve(c, c->res_sum, n * 8) || dreserve(c, c->res_val, n * 8) ||
-        dreserve(c, c->res_eps, n * 16) || dreserve(c, cv, (uint64_t)P.W * P.H * 4))
+        dreserve(c, c->res_eps, n * 32) || dreserve(c, cv, (uint64_t)P.W * P.H * 4))
         return set_error(c, RJ_ERR_OOM, "result allocation failed");
     RJ_CUDA(c, cudaMemsetAsync(cv.p, 0, (uint64_t)P.W * P.H * 4, c->stream));
     P.a.canvas = cv.as<uint32_t>();
     if ((s = run_pass(c, P, c->res_cnt.as<unsigned long long>(), c->res_sum.as<double>())) != RJ_OK) return s;
     unsigned long long *ep = c->res_eps.as<unsigned long long>(), *em = ep + n;
-    if ((s = interval_impl(c, P.W, P.H, P.pp, cv.as<uint32_t>(), ep, em)) != RJ_OK) return s;
+    const bool expected = exp_plus || exp_minus;
+    double *xp = expected ? reinterpret_cast<double *>(em + n) : nullptr, *xm = expected ? xp + n : nullptr;
+    if ((s = interval_impl(c, P.W, P.H, P.pp, cv.as<uint32_t>(), ep, em, xp, xm)) != RJ_OK) return s;
     if (value) RJ_CUDA(c, launch_finalize(c, q->agg, (uint32_t)n, c->res_cnt.as<unsigned long long>(),
                                           c->res_sum.as<double>(), c->res_val.as<double>()));
     if (count) RJ_CUDA(c, cudaMemcpyAsync(count, c->res_cnt.p, n * 8, cudaMemcpyDeviceToHost, c->stream));
     if (value) RJ_CUDA(c, cudaMemcpyAsync(value, c->res_val.p, n * 8, cudaMemcpyDeviceToHost, c->stream));
     if (eps_plus) RJ_CUDA(c, cudaMemcpyAsync(eps_plus, ep, n * 8, cudaMemcpyDeviceToHost, c->stream));
     if (eps_minus) RJ_CUDA(c, cudaMemcpyAsync(eps_minus, em, n * 8, cudaMemcpyDeviceToHost, c->stream));
+    if (exp_plus) RJ_CUDA(c, cudaMemcpyAsync(exp_plus, xp, n * 8, cudaMemcpyDeviceToHost, c->stream));
+    if (exp_minus) RJ_CUDA(c, cudaMemcpyAsync(exp_minus, xm, n * 8, cudaMemcpyDeviceToHost, c->stream));
     if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[3], c->stream));
     RJ_CUDA(c, cudaStreamSynchronize(c->stream));
     return RJ_OK;
+}
+
+rj_status rj_query_interval(rj_ctx *c, const rj_query_desc *q, uint64_t *count, double *value, uint64_t *eps_plus,
+                            uint64_t *eps_minus) {
+    return query_interval(c, q, count, value, eps_plus, eps_minus, nullptr, nullptr);
+}
+
+rj_status rj_query_interval_ex(rj_ctx *c, const rj_query_desc *q, uint64_t *count, double *value,
+                               uint64_t *eps_plus, uint64_t *eps_minus, double *exp_plus, double *exp_minus) {
+    return query_interval(c, q, count, value, eps_plus, eps_minus, exp_plus, exp_minus);
 }
 
 rj_status rj_debug_point_canvas(rj_ctx *c, const rj_query_desc *q, uint32_t *counts) {

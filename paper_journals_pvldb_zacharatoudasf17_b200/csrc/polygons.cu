@@ -349,11 +349,18 @@ rj_status load_polygons_impl(Ctx *c, uint32_t n_poly, const uint32_t *pro, const
     }
 
     dfree(c, c->edges); dfree(c, c->edge_poly); dfree(c, c->poly_edge_off); dfree(c, c->mbr);
+    dfree(c, c->poly_ring_off); dfree(c, c->ring_edge_off); dfree(c, c->edge_sigma);
     dfree(c, c->grid_off); dfree(c, c->grid_ent);
     c->n_poly = 0;
     if (dalloc(c, c->edges, ne * sizeof(int4)) || dalloc(c, c->edge_poly, ne * 4) ||
-        dalloc(c, c->poly_edge_off, (n_poly + 1) * 4) || dalloc(c, c->mbr, n_poly * sizeof(int4)))
+        dalloc(c, c->poly_edge_off, (n_poly + 1) * 4) || dalloc(c, c->mbr, n_poly * sizeof(int4)) ||
+        dalloc(c, c->poly_ring_off, (n_poly + 1) * 4) || dalloc(c, c->ring_edge_off, (n_ring + 1) * 4) ||
+        dalloc(c, c->edge_sigma, ne))
         return set_error(c, RJ_ERR_OOM, "polygon allocation failed");
+    // one edge per vertex, in vertex order: ring r's edges are [rvo[r], rvo[r+1])
+    RJ_CUDA(c, cudaMemcpyAsync(c->poly_ring_off.p, pro, (n_poly + 1) * 4, cudaMemcpyHostToDevice, c->stream));
+    RJ_CUDA(c, cudaMemcpyAsync(c->ring_edge_off.p, rvo, (n_ring + 1) * 4, cudaMemcpyHostToDevice, c->stream));
+    c->n_ring = n_ring;
     RJ_CUDA(c, cudaMemcpyAsync(c->edges.p, edges.data(), ne * sizeof(int4), cudaMemcpyHostToDevice, c->stream));
     RJ_CUDA(c, cudaMemcpyAsync(c->edge_poly.p, epoly.data(), ne * 4, cudaMemcpyHostToDevice, c->stream));
     RJ_CUDA(c, cudaMemcpyAsync(c->poly_edge_off.p, peoff.data(), (n_poly + 1) * 4, cudaMemcpyHostToDevice, c->stream));
@@ -396,6 +403,10 @@ rj_status load_polygons_impl(Ctx *c, uint32_t n_poly, const uint32_t *pro, const
             c->grid_edge.as<int4>(), c->grid_poly.as<uint32_t>());
         RJ_LAUNCHED(c);
         RJ_CUDA(c, cudaGetLastError());
+    }
+    {
+        rj_status rs = ring_sigma_impl(c, n_poly, n_ring);
+        if (rs != RJ_OK) return rs;
     }
     RJ_CUDA(c, cudaStreamSynchronize(c->stream));
     dfree(c, cnt);

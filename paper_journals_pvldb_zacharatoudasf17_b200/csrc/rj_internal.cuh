@@ -124,6 +124,9 @@ struct Ctx {
     uint32_t n_edges = 0;
     double edge_len_x = 0.0, edge_len_y = 0.0;   // sum of |dx|, |dy| over edges (lattice units)
     Buf edges, edge_poly, poly_edge_off, mbr;   // int4 edges/mbr
+    Buf poly_ring_off, ring_edge_off;          // rings: [n_poly + 1] first ring, [n_ring + 1] first edge
+    Buf edge_sigma;                            // int8 per edge: ring weight orientation * (-1)^depth (Z22)
+    uint32_t n_ring = 0;
     Buf grid_off, grid_ent;
     Buf grid_edge, grid_poly;                  // entries inlined: edge endpoints + polygon
     uint64_t n_grid_ent = 0;
@@ -237,8 +240,13 @@ rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp,
 
 // interval.cu: bounded-mode worst-case result intervals from the
 // per-pixel count canvas, the spans and the S5 bands of the polygon pass.
+// With d_exp_plus / d_exp_minus (binary64, may be NULL) also the expected
+// interval sums of P:811-827 (reading Z22).
 rj_status interval_impl(Ctx *c, int W, int H, const PolyPass &pp, const uint32_t *canvas,
-                        unsigned long long *d_eps_plus, unsigned long long *d_eps_minus);
+                        unsigned long long *d_eps_plus, unsigned long long *d_eps_minus,
+                        double *d_exp_plus = nullptr, double *d_exp_minus = nullptr);
+// interval.cu: per-edge ring weights (load time)
+rj_status ring_sigma_impl(Ctx *c, uint32_t n_poly, uint32_t n_ring);
 
 // pass.cu
 rj_status point_pass(Ctx *c, const PassArgs &a, bool sum, bool accurate);

@@ -6,7 +6,7 @@ There is no fallback: if librj.so is missing or no sm_100 device is present
 the calls raise.
 
     rj_create, rj_destroy, rj_load_points, rj_load_polygons, rj_query,
-    rj_query_device, rj_query_stream, rj_query_interval, rj_query_multi, rj_finalize_device, rj_resolve_canvas(_domain),
+    rj_query_device, rj_query_stream, rj_query_interval, rj_query_interval_ex, rj_query_multi, rj_finalize_device, rj_resolve_canvas(_domain),
     rj_debug_pixel_spans, rj_debug_boundary_mask, rj_debug_point_membership, rj_debug_point_canvas,
     rj_get_stats, rj_set_option  -- same names as the C ABI.
 
@@ -88,6 +88,7 @@ def lib():
             "rj_query_device": (i32, [vp, qp, vp, vp]),
             "rj_query_stream": (i32, [vp, qp, u64, vp, vp, i32, i32, vp, vp, vp, vp]),
             "rj_query_interval": (i32, [vp, qp, vp, vp, vp, vp]),
+            "rj_query_interval_ex": (i32, [vp, qp, vp, vp, vp, vp, vp, vp]),
             "rj_query_multi": (i32, [vp, qp, i32, vp, vp, vp]),
             "rj_debug_point_canvas": (i32, [vp, qp, vp]),
             "rj_finalize_device": (i32, [vp, i32, u32, vp, vp, vp]),
@@ -114,7 +115,7 @@ def lib():
 
 
 EXPORTS = ["rj_create", "rj_destroy", "rj_set_allocator", "rj_load_points", "rj_load_polygons", "rj_query",
-           "rj_query_device", "rj_query_stream", "rj_query_interval", "rj_query_multi", "rj_debug_point_canvas", "rj_finalize_device", "rj_resolve_canvas", "rj_resolve_canvas_domain",
+           "rj_query_device", "rj_query_stream", "rj_query_interval", "rj_query_interval_ex", "rj_query_multi", "rj_debug_point_canvas", "rj_finalize_device", "rj_resolve_canvas", "rj_resolve_canvas_domain",
            "rj_debug_pixel_spans", "rj_debug_boundary_mask", "rj_debug_point_membership", "rj_get_stats",
            "rj_set_option", "rj_get_stream", "rj_n_polygons", "rj_n_points", "rj_status_str", "rj_last_error", "rj_version"]
 
@@ -241,6 +242,12 @@ def rj_query_interval(ctx, desc, count=None, value=None, eps_plus=None, eps_minu
                                    _ptr(eps_minus)), ctx)
 
 
+def rj_query_interval_ex(ctx, desc, count=None, value=None, eps_plus=None, eps_minus=None, exp_plus=None,
+                         exp_minus=None):
+    _check(lib().rj_query_interval_ex(ctx, ctypes.byref(desc), _ptr(count), _ptr(value), _ptr(eps_plus),
+                                      _ptr(eps_minus), _ptr(exp_plus), _ptr(exp_minus)), ctx)
+
+
 def rj_debug_point_canvas(ctx, desc):
     W, H = rj_resolve_canvas(ctx, desc)
     out = np.zeros((H, W), dtype=np.uint32)
@@ -363,6 +370,15 @@ class RasterJoin:
         q = make_desc(**kw)
         out = [np.zeros(self.n_poly, dtype=t) for t in (np.uint64, np.float64, np.uint64, np.uint64)]
         rj_query_interval(self.ctx, q, *out)
+        return tuple(out)
+
+    def query_interval_ex(self, **kw):
+        """Bounded query with worst-case and expected intervals:
+        (count, value, eps_plus, eps_minus, exp_plus, exp_minus)."""
+        q = make_desc(**kw)
+        out = [np.zeros(self.n_poly, dtype=t)
+               for t in (np.uint64, np.float64, np.uint64, np.uint64, np.float64, np.float64)]
+        rj_query_interval_ex(self.ctx, q, *out)
         return tuple(out)
 
     def point_canvas(self, **kw):

@@ -100,3 +100,47 @@ def test_interval_rejects_other_modes(c1):
     R = c1[0]
     with pytest.raises(rjmod.RJError):
         R.query_interval(W=64, mode="accurate")
+
+
+def _close(g, o, scale):
+    """binary64 sums of f * Fpt by two different area computations (Green
+    edge integrals vs ring clipping): within 1e-9 of the worst-case mass."""
+    return np.all(np.abs(g - o) <= 1e-9 * (scale + 1.0))
+
+
+@pytest.mark.parametrize("W,H", [(16, 16), (64, 64), (200, 200), (777, 555), (1024, 1024)])
+def test_expected_interval_parity(c1, W, H):
+    # P:811-827, reading Z22 / oracle O13
+    R, P, x, y, cols = c1
+    preds = [(0, "<", 25)]
+    cnt, _, ep, em, xp, xm = R.query_interval_ex(W=W, H=H, preds=preds)
+    counts = oracle.pixel_counts(x, y, C.C1_BOX, cols=cols, preds=preds, W=W, H=H)
+    oep, oem = oracle.error_interval(P, W, H, counts)
+    oxp, oxm = oracle.expected_interval(P, W, H, counts)
+    assert np.array_equal(ep, oep) and np.array_equal(em, oem)
+    assert _close(xp, oxp, oep.astype(np.float64)), (xp, oxp)
+    assert _close(xm, oxm, oem.astype(np.float64)), (xm, oxm)
+    assert np.all(xp <= ep + 1e-9) and np.all(xm <= em + 1e-9)
+    # the plain call gives the same worst case
+    c2, _, ep2, em2 = R.query_interval(W=W, H=H, preds=preds)
+    assert np.array_equal(c2, cnt) and np.array_equal(ep2, ep) and np.array_equal(em2, em)
+
+
+def test_expected_interval_taxi_neighbourhoods():
+    """Tiling with shared vertices, 1M taxi-shaped points, 256^2 (parity)
+    and the estimate's quality at 2048^2 against the accurate count."""
+    flat = C.array_polys("neighborhoods")
+    pts = C.taxi(1_000_000)
+    R = rjmod.RasterJoin(C.NYC_BOX)
+    R.load_points(pts["x"], pts["y"])
+    R.load_polygons(flat)
+    P = oracle.Polys(flat, C.NYC_BOX)
+    _, _, ep, em, xp, xm = R.query_interval_ex(W=256, H=256)
+    counts = oracle.pixel_counts(pts["x"], pts["y"], C.NYC_BOX, W=256, H=256)
+    oxp, oxm = oracle.expected_interval(P, 256, 256, counts)
+    assert _close(xp, oxp, ep.astype(np.float64)) and _close(xm, oxm, em.astype(np.float64))
+    cnt, _, ep, em, xp, xm = R.query_interval_ex(W=2048, H=2048)
+    acc, _ = R.query(W=2048, H=2048, mode="accurate")
+    b, a = cnt.astype(np.float64), acc.astype(np.float64)
+    est = b - xp + xm
+    assert np.abs(a - est).sum() < 0.5 * np.abs(a - b).sum()

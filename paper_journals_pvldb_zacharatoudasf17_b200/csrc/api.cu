@@ -25,6 +25,7 @@ rj_status cuda_error(Ctx *c, cudaError_t e, const char *where) {
 }
 
 cudaError_t dalloc(Ctx *c, Buf &b, size_t bytes) {
+    ++c->alloc_gen;
     b.p = nullptr;
     b.bytes = 0;
     if (bytes == 0) bytes = 16;
@@ -44,6 +45,7 @@ cudaError_t dalloc(Ctx *c, Buf &b, size_t bytes) {
 }
 
 void dfree(Ctx *c, Buf &b) {
+    ++c->alloc_gen;
     if (b.p) {
         if (c->free_fn) c->free_fn(b.p, c->alloc_user);
         else cudaFree(b.p);
@@ -54,6 +56,7 @@ void dfree(Ctx *c, Buf &b) {
 
 cudaError_t dreserve(Ctx *c, Buf &b, size_t bytes) {
     if (b.p && b.bytes >= bytes) return cudaSuccess;
+    if (c->capturing) return cudaErrorNotPermitted;          // never grow inside a graph capture
     if (b.p) {
         cudaError_t e = cudaStreamSynchronize(c->stream);    // grow: no kernel may still use it
         if (e != cudaSuccess) return e;
@@ -64,6 +67,7 @@ cudaError_t dreserve(Ctx *c, Buf &b, size_t bytes) {
 
 cudaError_t dreserve_exact(Ctx *c, Buf &b, size_t bytes) {
     if (b.p && b.bytes >= bytes) return cudaSuccess;
+    if (c->capturing) return cudaErrorNotPermitted;
     if (b.p) {
         cudaError_t e = cudaStreamSynchronize(c->stream);
         if (e != cudaSuccess) return e;
@@ -264,6 +268,11 @@ static rj_status check_ready(Ctx *c, const rj_query_desc *q) {
     return RJ_OK;
 }
 
+// Timing events; inside a graph capture they become event-record nodes.
+static cudaError_t record_ev(Ctx *c, int i) {
+    return cudaEventRecordWithFlags(c->ev[i], c->stream, c->capturing ? cudaEventRecordExternal : cudaEventRecordDefault);
+}
+
 // Everything up to (not including) the point-pass launch.
 static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_polygon_pass = true,
                          bool bands = false) {
@@ -300,13 +309,13 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     a.n_stages = (uint32_t)point_pass_stages(f.n_slots);
     if ((s = items_for_level(c, P.L)) != RJ_OK) return s;
     c->launches = 0;
-    if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[0], c->stream));
+    if (c->timing) RJ_CUDA(c, record_ev(c, 0));
     // the index join needs neither spans nor the boundary mask
     P.pp = PolyPass{};
     if (need_polygon_pass && !P.index &&
         (s = polygon_pass(c, P.W, P.H, P.L, P.acc || bands, P.pp, P.view)) != RJ_OK)
         return s;
-    if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[1], c->stream));
+    if (c->timing) RJ_CUDA(c, record_ev(c, 1));
     a.qx = c->qx.as<uint32_t>();
     a.qy = c->qy.as<uint32_t>();
     for (int k = 0; k < f.n_slots; ++k) a.col[k] = c->col[f.slot_col[k]].as<uint32_t>();
@@ -383,7 +392,7 @@ static rj_status run_pass(Ctx *c, Prepared &P, unsigned long long *d_cnt, double
     s = point_pass(c, a, P.sum, P.acc);
     if (s != RJ_OK) return s;
     if (a.bq_cap && (s = pip_queue_pass(c, a, P.sum)) != RJ_OK) return s;
-    if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[2], c->stream));
+    if (c->timing) RJ_CUDA(c, record_ev(c, 2));
     RJ_CUDA(c, cudaMemcpyAsync(c->h_stats, a.stats, 2 * sizeof(unsigned long long), cudaMemcpyDeviceToHost, c->stream));
     // statistics of this query
     c->stream_stats_pending = 0;
@@ -451,7 +460,7 @@ static rj_status label_query_with_cols(Ctx *c, const rj_query_desc *q, const Agg
         RJ_CUDA(c, cudaMemcpyAsync(values, c->res_val.p, (size_t)nv * np * 8, cudaMemcpyDeviceToHost, c->stream));
     }
     if (count) RJ_CUDA(c, cudaMemcpyAsync(count, c->res_cnt.p, np * 8, cudaMemcpyDeviceToHost, c->stream));
-    if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[3], c->stream));
+    if (c->timing) RJ_CUDA(c, record_ev(c, 3));
     RJ_CUDA(c, cudaStreamSynchronize(c->stream));
     return RJ_OK;
 }
@@ -474,6 +483,92 @@ static AggPlan single_plan(const rj_query_desc *q) {
         ap.col[0] = q->agg_column;
     }
     return ap;
+}
+
+// ---- CUDA-graph replay of repeated queries ---------------------------------
+// A query's device work is ~40 launches (the polygon pass's small kernels,
+// scans and memsets, the point pass, finalise); at 1/8 of the points per GPU
+// the polygon pass becomes launch-bound.  The second consecutive call with
+// the same key (descriptor, output pointers, options, loaded data and every
+// device allocation) is captured into a CUDA graph, and later calls with
+// that key replay it with one cudaGraphLaunch.  Every kernel still runs on
+// every query: only the host-side launch sequence is reused.  The capture
+// needs a host-sync-free sequence, which the polygon pass's size cache
+// (same key => same sizes) provides; if anything would allocate or sync
+// during the capture, it is abandoned and the query runs eagerly.
+static void key_desc(std::vector<int64_t> &k, const rj_query_desc *q) {
+    auto bits = [](double v) { int64_t b; memcpy(&b, &v, 8); return b; };
+    k.insert(k.end(), {q->agg, q->agg_column, q->n_pred});
+    for (int i = 0; i < q->n_pred && i < RJ_MAX_PRED; ++i)
+        k.insert(k.end(), {q->pred[i].column, q->pred[i].op, bits(q->pred[i].value)});
+    k.insert(k.end(), {q->canvas_w, q->canvas_h, bits(q->epsilon), q->mode, q->view[0], q->view[1], q->view[2],
+                       q->view[3]});
+}
+
+static std::vector<int64_t> query_key(Ctx *c, const rj_query_desc *q, int entry, const void *p0, const void *p1) {
+    std::vector<int64_t> k = {entry, (int64_t)(uintptr_t)p0, (int64_t)(uintptr_t)p1, (int64_t)c->data_gen,
+                              (int64_t)c->alloc_gen, c->timing, c->chunk, c->tile_side, c->force_stages,
+                              c->pass_variant, (int64_t)(uintptr_t)c->stream};
+    key_desc(k, q);
+    return k;
+}
+
+static void drop_graph(Ctx *c) {
+    if (c->graph_exec) cudaGraphExecDestroy(c->graph_exec);
+    c->graph_exec = nullptr;
+    c->graph_key.clear();
+}
+
+template <class F>
+static rj_status run_graphed(Ctx *c, std::vector<int64_t> key, F body) {
+    if (c->use_graphs && c->graph_exec && key == c->graph_key) {
+        RJ_CUDA(c, cudaGraphLaunch(c->graph_exec, c->stream));
+        c->last = c->graph_last;
+        c->launches = c->graph_launches;
+        c->last_stages = c->graph_stages;
+        c->last_ctas_per_sm = c->graph_ctas;
+        c->stream_stats_pending = 0;
+        return RJ_OK;
+    }
+    if (!c->use_graphs || key != c->pending_key) {
+        rj_status s = body();
+        c->pending_key.clear();
+        if (s == RJ_OK) {
+            key[4] = (int64_t)c->alloc_gen;      // allocations made by this call are part of the state
+            c->pending_key = key;
+        }
+        return s;
+    }
+    drop_graph(c);
+    c->pending_key.clear();
+    if (cudaStreamBeginCapture(c->stream, cudaStreamCaptureModeRelaxed) != cudaSuccess) {
+        cudaGetLastError();
+        return body();
+    }
+    c->capturing = true;
+    rj_status s = body();
+    c->capturing = false;
+    cudaGraph_t g = nullptr;
+    cudaError_t e = cudaStreamEndCapture(c->stream, &g);
+    cudaGraphExec_t ex = nullptr;
+    if (s == RJ_OK && e == cudaSuccess && g) e = cudaGraphInstantiate(&ex, g, 0);
+    if (g) cudaGraphDestroy(g);
+    if (s != RJ_OK || e != cudaSuccess || !ex) {
+        // nothing of the capture ran: clear its error and run eagerly
+        cudaGetLastError();
+        c->poisoned = false;
+        c->err.clear();
+        return body();
+    }
+    c->graph_exec = ex;
+    key[4] = (int64_t)c->alloc_gen;
+    c->graph_key = key;
+    c->graph_last = c->last;
+    c->graph_launches = c->launches;
+    c->graph_stages = c->last_stages;
+    c->graph_ctas = c->last_ctas_per_sm;
+    RJ_CUDA(c, cudaGraphLaunch(ex, c->stream));
+    return RJ_OK;
 }
 
 }  // namespace rj
@@ -551,11 +646,13 @@ rj_status rj_destroy(rj_ctx *c) {
     if (!c) return RJ_ERR_INVALID_ARGUMENT;
     cudaSetDevice(c->device);
     cudaStreamSynchronize(c->stream);
+    drop_graph(c);
     dfree(c, c->qx); dfree(c, c->qy); dfree(c, c->idx);
     for (auto &b : c->col) dfree(c, b);
     free_load_scratch(c);
     dfree(c, c->cell_off); drop_items(c);
     dfree(c, c->edges); dfree(c, c->edge_poly); dfree(c, c->poly_edge_off); dfree(c, c->mbr);
+    dfree(c, c->poly_ring_off); dfree(c, c->ring_edge_off); dfree(c, c->edge_sigma);
     dfree(c, c->grid_off); dfree(c, c->grid_ent); dfree(c, c->grid_edge); dfree(c, c->grid_poly);
     for (auto &b : c->ws) dfree(c, b);
     dfree(c, c->res_cnt); dfree(c, c->res_sum); dfree(c, c->res_val); dfree(c, c->res_eps); dfree(c, c->res_agg);
@@ -579,6 +676,11 @@ rj_status rj_set_allocator(rj_ctx *c, void *(*alloc_fn)(size_t, void *), void (*
 rj_status rj_set_option(rj_ctx *c, int32_t option, int64_t value) {
     if (!c) return RJ_ERR_INVALID_ARGUMENT;
     if (option == RJ_OPT_TIMING) { c->timing = value ? 1 : 0; return RJ_OK; }
+    if (option == RJ_OPT_GRAPHS) {
+        c->use_graphs = value ? 1 : 0;
+        if (!value) { drop_graph(c); c->pending_key.clear(); }
+        return RJ_OK;
+    }
     if (option == RJ_OPT_PASS) {
         if (value < -1 || value > 1) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "RJ_OPT_PASS must be -1, 0 or 1");
         c->pass_variant = (int)value;
@@ -646,14 +748,17 @@ rj_status rj_load_polygons(rj_ctx *c, uint32_t n_poly, const uint32_t *pro, cons
 
 rj_status rj_query_device(rj_ctx *c, const rj_query_desc *q, uint64_t *d_count, double *d_sum) {
     if (!d_count) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL d_count");
-    if (q && q->agg > RJ_AVG) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "rj_query_device: COUNT/SUM/AVG partials only");
-    Prepared P;
-    rj_status s = prepare(c, q, P);
+    if (!q) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL query descriptor");
+    if (q->agg > RJ_AVG) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "rj_query_device: COUNT/SUM/AVG partials only");
+    if (q->agg != RJ_COUNT && !d_sum) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL d_sum for SUM/AVG");
+    rj_status s = check_ready(c, q);
     if (s != RJ_OK) return s;
-    Buf &scratch = wsbuf(c, kWsSizes);
-    if (P.sum && !d_sum) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL d_sum for SUM/AVG");
-    (void)scratch;
-    return run_pass(c, P, reinterpret_cast<unsigned long long *>(d_count), d_sum);
+    return run_graphed(c, query_key(c, q, 1, d_count, d_sum), [&]() -> rj_status {
+        Prepared P;
+        rj_status s2 = prepare(c, q, P);
+        if (s2 != RJ_OK) return s2;
+        return run_pass(c, P, reinterpret_cast<unsigned long long *>(d_count), d_sum);
+    });
 }
 
 rj_status rj_finalize_device(rj_ctx *c, int32_t agg, uint32_t n, const uint64_t *d_count, const double *d_sum,
@@ -673,18 +778,24 @@ rj_status rj_query(rj_ctx *c, const rj_query_desc *q, uint64_t *count, double *v
             return set_error(c, RJ_ERR_INVALID_ARGUMENT, "agg_column out of range");
         return label_query_with_cols(c, q, single_plan(q), lattice_input(c), c->n_cols, count, value);
     }
-    Prepared P;
-    rj_status s = prepare(c, q, P);
+    rj_status s = check_ready(c, q);
     if (s != RJ_OK) return s;
     const size_t n = c->n_poly;
     if (dreserve(c, c->res_cnt, n * 8) || dreserve(c, c->res_sum, n * 8) || dreserve(c, c->res_val, n * 8))
         return set_error(c, RJ_ERR_OOM, "result allocation failed");
-    if ((s = run_pass(c, P, c->res_cnt.as<unsigned long long>(), c->res_sum.as<double>())) != RJ_OK) return s;
-    if (value) RJ_CUDA(c, launch_finalize(c, q->agg, (uint32_t)n, c->res_cnt.as<unsigned long long>(),
-                                          c->res_sum.as<double>(), c->res_val.as<double>()));
+    s = run_graphed(c, query_key(c, q, 2, nullptr, value ? c->res_val.p : nullptr), [&]() -> rj_status {
+        Prepared P;
+        rj_status s2 = prepare(c, q, P);
+        if (s2 != RJ_OK) return s2;
+        if ((s2 = run_pass(c, P, c->res_cnt.as<unsigned long long>(), c->res_sum.as<double>())) != RJ_OK) return s2;
+        if (value) RJ_CUDA(c, launch_finalize(c, q->agg, (uint32_t)n, c->res_cnt.as<unsigned long long>(),
+                                              c->res_sum.as<double>(), c->res_val.as<double>()));
+        return RJ_OK;
+    });
+    if (s != RJ_OK) return s;
     if (count) RJ_CUDA(c, cudaMemcpyAsync(count, c->res_cnt.p, n * 8, cudaMemcpyDeviceToHost, c->stream));
     if (value) RJ_CUDA(c, cudaMemcpyAsync(value, c->res_val.p, n * 8, cudaMemcpyDeviceToHost, c->stream));
-    if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[3], c->stream));
+    if (c->timing) RJ_CUDA(c, record_ev(c, 3));
     RJ_CUDA(c, cudaStreamSynchronize(c->stream));
     return RJ_OK;
 }
@@ -765,7 +876,7 @@ static rj_status query_interval(rj_ctx *c, const rj_query_desc *q, uint64_t *cou
     if (eps_minus) RJ_CUDA(c, cudaMemcpyAsync(eps_minus, em, n * 8, cudaMemcpyDeviceToHost, c->stream));
     if (exp_plus) RJ_CUDA(c, cudaMemcpyAsync(exp_plus, xp, n * 8, cudaMemcpyDeviceToHost, c->stream));
     if (exp_minus) RJ_CUDA(c, cudaMemcpyAsync(exp_minus, xm, n * 8, cudaMemcpyDeviceToHost, c->stream));
-    if (c->timing) RJ_CUDA(c, cudaEventRecord(c->ev[3], c->stream));
+    if (c->timing) RJ_CUDA(c, record_ev(c, 3));
     RJ_CUDA(c, cudaStreamSynchronize(c->stream));
     return RJ_OK;
 }

@@ -218,6 +218,7 @@ rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int
     dfree(c, c->cell_off);
     drop_items(c);
     c->n_in = c->n_pts = 0; c->n_cols = 0;
+    ++c->data_gen;
 
     const size_t esz = xy_f64 ? 8 : 4;
     const void *dx = nullptr, *dy = nullptr, *dcol[RJ_MAX_COLS] = {};
@@ -300,6 +301,7 @@ rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int
     RJ_CUDA(c, cudaMemcpyAsync(&n_valid, c->cell_off.as<uint32_t>() + kCells10, 4, cudaMemcpyDeviceToHost, c->stream));
     RJ_CUDA(c, cudaStreamSynchronize(c->stream));
     c->n_pts = n_valid;
+    ++c->data_gen;
     if (n_ood) *n_ood = n - n_valid;
     if (!c->keep_load_scratch) free_load_scratch(c);
     return RJ_OK;

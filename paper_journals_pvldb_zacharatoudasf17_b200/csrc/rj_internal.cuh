@@ -127,6 +127,27 @@ struct Ctx {
     Buf poly_ring_off, ring_edge_off;          // rings: [n_poly + 1] first ring, [n_ring + 1] first edge
     Buf edge_sigma;                            // int8 per edge: ring weight orientation * (-1)^depth (Z22)
     uint32_t n_ring = 0;
+
+    // polygon-pass sizes of the last query (host metadata only: every
+    // kernel still runs per query).  They are a pure function of the key
+    // (canvas, level, mode, window, loaded data), so a repeated key skips the
+    // two device->host size reads and the whole query is enqueued without a
+    // host round trip.
+    uint64_t data_gen = 0;                     // bumped by every load
+    int64_t pp_key[9] = {};
+    bool pp_key_valid = false;
+    uint32_t pp_sizes[6] = {};                 // X, NPR, B, S, NP, NB
+
+    // CUDA-graph replay of a repeated query (api.cu run_graphed): the key
+    // covers the descriptor, outputs, options and every allocation
+    uint64_t alloc_gen = 0;                    // bumped by every device (re)allocation / free
+    bool capturing = false;
+    int use_graphs = 1;                        // RJ_OPT_GRAPHS
+    std::vector<int64_t> graph_key, pending_key;
+    cudaGraphExec_t graph_exec = nullptr;
+    rj_stats graph_last{};
+    uint32_t graph_launches = 0;
+    int graph_stages = 0, graph_ctas = 0;
     Buf grid_off, grid_ent;
     Buf grid_edge, grid_poly;                  // entries inlined: edge endpoints + polygon
     uint64_t n_grid_ent = 0;

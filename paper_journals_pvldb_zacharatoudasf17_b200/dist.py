@@ -58,3 +58,83 @@ def query_sharded(R: "rj.RasterJoin", desc, d_count: torch.Tensor, d_sum: torch.
     rj.rj_finalize_device(R.ctx, desc.agg, d_count, d_sum, d_value)
     cur.wait_stream(ctx_stream)
     return d_value
+
+
+# ---- spatially compact shards (second milestone) -----------
+#
+# Index-range shards of time-ordered input are spatially random: every rank
+# then rasterises every polygon over the whole canvas, a fixed per-rank cost
+# that caps strong scaling.  Exchanging the points once at load time into x
+# strips of equal point count (splitters = x-quantiles of an all-gathered
+# sample, one all_to_all per column over NVLink) lets each rank query only
+# the pixel window of its strip (a viewport): its spans and pieces
+# shrink by the world size.  Pixels on a strip border are seen by two ranks
+# with disjoint points, and the per-polygon partials still just add
+# (distributivity), so no pixel ownership is needed.
+
+def strip_splitters(x: torch.Tensor, world: int, group=None, sample: int = 1 << 16) -> torch.Tensor:
+    """world-1 increasing x splitters (float64, on x's device) giving strips
+    of about equal point count over all ranks' points."""
+    n = x.numel()
+    if n:
+        idx = torch.linspace(0, n - 1, sample, device=x.device).round().long()
+        s = x[idx].to(torch.float64)
+    else:
+        s = torch.full((sample,), float("nan"), dtype=torch.float64, device=x.device)
+    parts = [torch.empty_like(s) for _ in range(world)]
+    dist.all_gather(parts, s, group=group)
+    return splitters_from_sample(torch.cat(parts), world)
+
+
+def splitters_from_sample(allv: torch.Tensor, world: int) -> torch.Tensor:
+    """The k/world quantiles (k = 1..world-1) of a sample of x (NaN ignored)."""
+    allv = torch.sort(allv[~torch.isnan(allv)].to(torch.float64)).values
+    if allv.numel() == 0:
+        return torch.zeros(world - 1, dtype=torch.float64, device=allv.device)
+    k = torch.arange(1, world, device=allv.device) * allv.numel() // world
+    return allv[k]
+
+
+def strip_of(x: torch.Tensor, splitters: torch.Tensor) -> torch.Tensor:
+    """Destination rank of every point: the number of splitters <= x (NaN
+    coordinates go to the last rank and are dropped at load)."""
+    d = torch.bucketize(x.to(torch.float64), splitters, right=True)
+    return torch.where(torch.isnan(x), torch.full_like(d, splitters.numel()), d)
+
+
+def exchange(columns, dest: torch.Tensor, world: int, group=None):
+    """Send every point (all its columns) to rank dest[i]; returns this
+    rank's received columns (grouped by source rank, input order kept)."""
+    order = torch.argsort(dest, stable=True)
+    send = torch.bincount(dest, minlength=world).to(torch.int64)
+    recv = torch.empty_like(send)
+    dist.all_to_all_single(recv, send, group=group)
+    s_l, r_l = send.tolist(), recv.tolist()
+    out = []
+    for c in columns:
+        o = torch.empty(sum(r_l), dtype=c.dtype, device=c.device)
+        dist.all_to_all_single(o, c[order].contiguous(), r_l, s_l, group=group)
+        out.append(o)
+    return out
+
+
+def strip_window(box, splitters, rank: int, world: int, W: int, H: int):
+    """Pixel window (c0, 0, c1, H) of the W x H canvas holding every point of
+    rank's strip [split[rank-1], split[rank]) -- padded by one column each
+    side against rounding, so it is a superset (extra columns hold no point
+    of this rank and cost nothing but their spans)."""
+    import math
+    sp = [float(v) for v in splitters.tolist()] if hasattr(splitters, "tolist") else list(splitters)
+    bw = box[2] - box[0]
+    c0 = 0 if rank == 0 else max(0, int(math.floor((sp[rank - 1] - box[0]) / bw * W)) - 1)
+    c1 = W if rank == world - 1 else min(W, int(math.ceil((sp[rank] - box[0]) / bw * W)) + 1)
+    return (c0, 0, max(c1, c0 + 1), H)
+
+
+def spatial_shard(x, y, cols, world: int, group=None):
+    """Load-time exchange: (x, y, cols) of this rank's index range ->
+    (x, y, cols, splitters) of its x strip."""
+    sp = strip_splitters(x, world, group)
+    dest = strip_of(x, sp)
+    got = exchange([x, y, *cols], dest, world, group)
+    return got[0], got[1], got[2:], sp

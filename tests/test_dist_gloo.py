@@ -67,3 +67,83 @@ def test_shards_allreduce_to_unsharded():
     cnt, s, _ = oracle.query(P, pts["x"], pts["y"], cols=[pts["fare"]], agg_col=0, W=2048, H=2048, mode="accurate")
     assert np.array_equal(got[0], cnt.astype(np.int64))
     assert np.allclose(got[1], s, rtol=1e-12, atol=0)
+
+
+def _spatial_worker(rank, world, port, q):
+    os.environ["MASTER_ADDR"] = "127.0.0.1"
+    os.environ["MASTER_PORT"] = str(port)
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        import oracle
+        from datagen import configs as C
+        from paper_journals_pvldb_zacharatoudasf17_b200 import dist as rjdist
+
+        n = 90_001
+        pts = C.taxi(n, fare=True)
+        lo, hi = rjdist.shard_range(n, rank, world)
+        cols = [torch.from_numpy(pts["t"][lo:hi].copy()), torch.from_numpy(pts["fare"][lo:hi].copy())]
+        x, y, cols, sp = rjdist.spatial_shard(torch.from_numpy(pts["x"][lo:hi].copy()),
+                                              torch.from_numpy(pts["y"][lo:hi].copy()), cols, world)
+        xs = x.numpy()
+        # every point lands in its strip
+        lo_x = -np.inf if rank == 0 else float(sp[rank - 1])
+        hi_x = np.inf if rank == world - 1 else float(sp[rank])
+        assert np.all((xs >= lo_x) & (xs < hi_x))
+        W = 4096
+        view = rjdist.strip_window(C.NYC_BOX, sp, rank, world, W, W)
+        P = oracle.Polys(C.array_polys("neighborhoods"), C.NYC_BOX)
+        preds = [(0, ">=", C.T_2012[0]), (0, "<", C.T_2012[1])]
+        out = []
+        for mode in ("bounded", "accurate"):
+            # the window must hold every point of the strip: the windowed query
+            # equals the unwindowed one on this rank's points
+            c_w, s_w, _ = oracle.query(P, xs, y.numpy(), cols=[c.numpy() for c in cols], preds=preds,
+                                       agg_col=1, W=W, H=W, mode=mode, view=view)
+            c_a, _, _ = oracle.query(P, xs, y.numpy(), cols=[c.numpy() for c in cols], preds=preds,
+                                     agg_col=1, W=W, H=W, mode=mode)
+            assert np.array_equal(c_w, c_a)
+            tc = torch.from_numpy(c_w.astype(np.int64))
+            ts = torch.from_numpy(s_w.copy())
+            rjdist.allreduce_partials(tc, ts)
+            out.append((tc.numpy().copy(), ts.numpy().copy()))
+        if rank == 0:
+            q.put((out, len(xs), view))
+        else:
+            q.put((None, len(xs), view))
+    finally:
+        dist.destroy_process_group()
+
+
+@pytest.mark.parametrize("world", [2, 3])
+def test_spatial_shards_allreduce_to_unsharded(world):
+    """x-strip shards by all_to_all + per-rank pixel windows
+    give the unsharded result (COUNT exact, SUM to 1e-12) in both modes, with
+    balanced strips."""
+    import oracle
+    from datagen import configs as C
+
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = _free_port()
+    procs = [ctx.Process(target=_spatial_worker, args=(r, world, port, q)) for r in range(world)]
+    for p in procs:
+        p.start()
+    res = [q.get(timeout=300) for _ in range(world)]
+    for p in procs:
+        p.join(timeout=120)
+        assert p.exitcode == 0
+    out = next(r[0] for r in res if r[0] is not None)
+    sizes = [r[1] for r in res]
+    n = 90_001
+    assert sum(sizes) == n
+    assert max(sizes) - min(sizes) <= 0.05 * n / world        # x-quantile strips balance the points
+    widths = sorted(r[2][2] - r[2][0] for r in res)
+    assert widths[-1] < 4096                                   # windows are strips, not the canvas
+    pts = C.taxi(n, fare=True)
+    P = oracle.Polys(C.array_polys("neighborhoods"), C.NYC_BOX)
+    preds = [(0, ">=", C.T_2012[0]), (0, "<", C.T_2012[1])]
+    for (gc, gs), mode in zip(out, ("bounded", "accurate")):
+        cnt, s, _ = oracle.query(P, pts["x"], pts["y"], cols=[pts["t"], pts["fare"]], preds=preds, agg_col=1,
+                                 W=4096, H=4096, mode=mode)
+        assert np.array_equal(gc, cnt.astype(np.int64)), mode
+        assert np.allclose(gs, s, rtol=1e-12, atol=0), mode

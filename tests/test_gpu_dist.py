@@ -27,16 +27,16 @@ def _port():
 N = 300_001
 
 
-def _worker(rank, world, port, q):
+def _worker(rank, world, port, q, spatial=False):
     try:
-        _run(rank, world, port, q)
+        _run(rank, world, port, q, spatial)
     except BaseException as e:          # report, do not hang the parent
         import traceback
         q.put(("error", rank, traceback.format_exc()))
         raise
 
 
-def _run(rank, world, port, q):
+def _run(rank, world, port, q, spatial=False):
     os.environ["MASTER_ADDR"] = "127.0.0.1"
     os.environ["MASTER_PORT"] = str(port)
     dist.init_process_group("gloo", rank=rank, world_size=world)
@@ -50,11 +50,20 @@ def _run(rank, world, port, q):
         lo, hi = rjdist.shard_range(N, rank, world)
         stream = torch.cuda.current_stream()
         R = rj.RasterJoin(C.NYC_BOX, device=0, stream=stream.cuda_stream)
-        R.load_points(pts["x"][lo:hi], pts["y"][lo:hi], [pts["t"][lo:hi], pts["fare"][lo:hi]])
+        x, y, cols = pts["x"][lo:hi], pts["y"][lo:hi], [pts["t"][lo:hi], pts["fare"][lo:hi]]
+        view = None
+        if spatial:
+            # x strips by all_to_all, each rank queries its window
+            tx, ty, tc, sp = rjdist.spatial_shard(torch.from_numpy(x.copy()), torch.from_numpy(y.copy()),
+                                                  [torch.from_numpy(c.copy()) for c in cols], world)
+            x, y, cols = tx.numpy(), ty.numpy(), [c.numpy() for c in tc]
+            view = rjdist.strip_window(C.NYC_BOX, sp, rank, world, 4096, 4096)
+        R.load_points(x, y, cols)
         R.load_polygons(C.array_polys("neighborhoods"))
         out = {}
         for mode in ("bounded", "accurate"):
-            desc = rj.make_desc(agg="avg", agg_column=1, preds=[(0, ">=", C.T_2012[0])], W=4096, H=4096, mode=mode)
+            desc = rj.make_desc(agg="avg", agg_column=1, preds=[(0, ">=", C.T_2012[0])], W=4096, H=4096, mode=mode,
+                                view=view)
             n = R.n_poly
             d_cnt = torch.zeros(n, dtype=torch.int64, device="cuda")
             d_sum = torch.zeros(n, dtype=torch.float64, device="cuda")
@@ -69,7 +78,8 @@ def _run(rank, world, port, q):
         dist.destroy_process_group()
 
 
-def test_sharded_query_allreduce_on_one_gpu():
+@pytest.mark.parametrize("spatial", [False, True])
+def test_sharded_query_allreduce_on_one_gpu(spatial):
     if not torch.cuda.is_available():
         pytest.skip("needs a CUDA device")
     import oracle
@@ -78,7 +88,7 @@ def test_sharded_query_allreduce_on_one_gpu():
     ctx = mp.get_context("spawn")
     q = ctx.Queue()
     port = _port()
-    procs = [ctx.Process(target=_worker, args=(r, 2, port, q)) for r in range(2)]
+    procs = [ctx.Process(target=_worker, args=(r, 2, port, q, spatial)) for r in range(2)]
     for p in procs:
         p.start()
     status, rank, got = q.get(timeout=600)

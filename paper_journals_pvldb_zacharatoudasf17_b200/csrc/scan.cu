@@ -1,7 +1,6 @@
 // scan.cu -- device exclusive prefix sum (u32) used by every CSR build of
 // the path (radix-sort digit offsets, crossings, spans, pieces, edge grid).
-// Three-phase: per-block scan of 4096 elements with block totals, recursive
-// scan of the totals, add-back.  256 threads x 16 elements per block.
+// Single pass with decoupled look-back, 256 threads x 16 elements per block.
 // out[n] receives the total; in == out (in place) is allowed.
 #include "rj_internal.cuh"
 
@@ -41,40 +40,74 @@ __device__ __forceinline__ uint32_t block_excl_scan(uint32_t v, uint32_t &total)
     return warp_tot[w] + inc - v;
 }
 
-__global__ void __launch_bounds__(kScanThreads) k_scan_tiles(const uint32_t *in,
-                                                             uint32_t *out, uint64_t n,
-                                                             uint32_t *__restrict__ tile_sums) {
-    const uint64_t base = (uint64_t)blockIdx.x * kScanTile + (uint64_t)threadIdx.x * kScanItems;
+// Single-pass scan with decoupled look-back: every block takes a ticket (so
+// all its predecessors are already resident), scans its 4096-element tile,
+// publishes the tile aggregate, then warp 0 walks back over the predecessors'
+// status words 32 at a time until it meets an inclusive prefix, and
+// publishes its own.  One memset + one launch per scan instead of a
+// recursive three-phase scan (the polygon pass runs six of them per query).
+constexpr unsigned long long kFlagAgg = 1ull << 32, kFlagInc = 2ull << 32;
+
+__device__ __forceinline__ unsigned long long ld_volatile(const unsigned long long *p) {
+    return *reinterpret_cast<const volatile unsigned long long *>(p);
+}
+
+__global__ void __launch_bounds__(kScanThreads) k_scan_lb(const uint32_t *in, uint32_t *out, uint64_t n,
+                                                          unsigned long long *__restrict__ ws) {
+    __shared__ uint32_t s_tile, s_excl;
+    unsigned long long *status = ws + 1;                  // ws[0]: ticket
+    if (threadIdx.x == 0) s_tile = (uint32_t)atomicAdd(ws, 1ull);
+    __syncthreads();
+    const uint32_t tile = s_tile;
+    const uint64_t base = (uint64_t)tile * kScanTile + (uint64_t)threadIdx.x * kScanItems;
     uint32_t v[kScanItems];
-    uint32_t s = 0;
+    uint32_t sum = 0;
 #pragma unroll
     for (int k = 0; k < kScanItems; ++k) {
-        uint64_t i = base + k;
+        const uint64_t i = base + k;
         v[k] = i < n ? in[i] : 0u;
-        s += v[k];
+        sum += v[k];
     }
     uint32_t total;
-    uint32_t pre = block_excl_scan(s, total);
+    uint32_t pre = block_excl_scan(sum, total);
+    if (tile == 0) {
+        if (threadIdx.x == 0) {
+            atomicExch(&status[0], kFlagInc | total);
+            s_excl = 0;
+        }
+    } else if (threadIdx.x < 32) {
+        const int lane = threadIdx.x;
+        if (lane == 0) atomicExch(&status[tile], kFlagAgg | total);
+        uint32_t excl = 0;
+        int64_t j = (int64_t)tile - 1;
+        for (;;) {
+            const int64_t k = j - lane;
+            unsigned long long st = k >= 0 ? ld_volatile(&status[k]) : kFlagInc;
+            while (__any_sync(0xffffffffu, (st >> 32) == 0))
+                if ((st >> 32) == 0) st = ld_volatile(&status[k]);
+            const unsigned inc = __ballot_sync(0xffffffffu, (st >> 32) == 2);
+            const int first = inc ? __ffs(inc) - 1 : 32;
+            uint32_t c = lane <= first ? (uint32_t)st : 0u;
+#pragma unroll
+            for (int o = 16; o; o >>= 1) c += __shfl_xor_sync(0xffffffffu, c, o);
+            excl += c;
+            if (inc) break;
+            j -= 32;
+        }
+        if (lane == 0) {
+            atomicExch(&status[tile], kFlagInc | (excl + total));
+            s_excl = excl;
+        }
+    }
+    __syncthreads();
+    pre += s_excl;
 #pragma unroll
     for (int k = 0; k < kScanItems; ++k) {
-        uint64_t i = base + k;
+        const uint64_t i = base + k;
         if (i < n) out[i] = pre;
         pre += v[k];
         if (i + 1 == n) out[n] = pre;
     }
-    if (threadIdx.x == 0) tile_sums[blockIdx.x] = total;
-}
-
-__global__ void __launch_bounds__(kScanThreads) k_scan_add(uint32_t *out, uint64_t n,
-                                                           const uint32_t *__restrict__ tile_pre) {
-    const uint32_t add = tile_pre[blockIdx.x];
-    if (add == 0) return;
-    const uint64_t base = (uint64_t)blockIdx.x * kScanTile;
-    for (int k = threadIdx.x; k < kScanTile; k += kScanThreads) {
-        uint64_t i = base + k;
-        if (i < n) out[i] += add;
-    }
-    if (blockIdx.x == gridDim.x - 1 && threadIdx.x == 0) out[n] += add;
 }
 
 __global__ void k_scan_zero(uint32_t *out) { out[0] = 0u; }
@@ -87,20 +120,13 @@ cudaError_t scan_u32(Ctx *c, const uint32_t *in, uint32_t *out, uint64_t n, int 
         return cudaGetLastError();
     }
     const uint64_t tiles = (n + kScanTile - 1) / kScanTile;
-    Buf &sums = wsbuf(c, ws_base);
-    cudaError_t e = dreserve(c, sums, (tiles + 1) * sizeof(uint32_t));
+    Buf &ws = wsbuf(c, ws_base);
+    cudaError_t e = dreserve(c, ws, (tiles + 1) * sizeof(unsigned long long));
     if (e != cudaSuccess) return e;
-    k_scan_tiles<<<(unsigned)tiles, kScanThreads, 0, c->stream>>>(in, out, n, sums.as<uint32_t>());
+    e = cudaMemsetAsync(ws.p, 0, (tiles + 1) * sizeof(unsigned long long), c->stream);
+    if (e != cudaSuccess) return e;
+    k_scan_lb<<<(unsigned)tiles, kScanThreads, 0, c->stream>>>(in, out, n, ws.as<unsigned long long>());
     RJ_LAUNCHED(c);
-    if (tiles > 1) {
-        Buf &pre = wsbuf(c, ws_base + 1);
-        e = dreserve(c, pre, (tiles + 1) * sizeof(uint32_t));
-        if (e != cudaSuccess) return e;
-        e = scan_u32(c, sums.as<uint32_t>(), pre.as<uint32_t>(), tiles, ws_base + 2);
-        if (e != cudaSuccess) return e;
-        k_scan_add<<<(unsigned)tiles, kScanThreads, 0, c->stream>>>(out, n, pre.as<uint32_t>());
-        RJ_LAUNCHED(c);
-    }
     return cudaGetLastError();
 }
 

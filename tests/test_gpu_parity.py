@@ -168,6 +168,33 @@ def test_sum_avg_filters(c1, mode, variant):
             assert ok, (cs, bad)
 
 
+@pytest.mark.parametrize("mode", ["bounded", "accurate"])
+def test_label_widths_many_polygons(mode):
+    """Polygon ids beyond 16 bits through the label kernel (SUM/AVG): a grid
+    of 257^2 = 66049 squares (non-dyadic side), and its first 1000 squares;
+    SUM of an integer attribute is bit-exact in both."""
+    m = 257
+    s = 1024.0 / m
+    ii, jj = np.meshgrid(np.arange(m), np.arange(m), indexing="xy")
+    x0, y0 = (ii.ravel() * s), (jj.ravel() * s)
+    x1, y1 = np.minimum(1024.0, x0 + s), np.minimum(1024.0, y0 + s)
+    n = m * m
+    vx = np.stack([x0, x1, x1, x0], 1).ravel()
+    vy = np.stack([y0, y0, y1, y1], 1).ravel()
+    pts = C.c1_points(20000)
+    rng = np.random.default_rng(5)
+    fav = rng.integers(0, 9, 20000).astype(np.int32)
+    for k in (1000, n):
+        flat = (np.arange(k + 1, dtype=np.uint32), np.arange(k + 1, dtype=np.uint32) * 4, vx[:4 * k], vy[:4 * k])
+        R = gpu_ctx(C.C1_BOX, flat, pts["x"], pts["y"], [fav])
+        P = oracle.Polys(flat, C.C1_BOX)
+        cnt, val = R.query(W=700, H=700, mode=mode, agg="sum", agg_column=0)
+        ocnt, osum, _ = oracle.query(P, pts["x"], pts["y"], cols=[fav], agg_col=0, W=700, H=700, mode=mode)
+        assert np.array_equal(cnt, ocnt), k
+        assert np.array_equal(val, osum), k
+        R.close()
+
+
 # ------------------------------------------------------------- edge cases
 def test_empty_and_degenerate_point_sets():
     flat = PG.flatten(C.polygon_set("c1"))

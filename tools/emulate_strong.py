@@ -58,6 +58,7 @@ def main():
     ap.add_argument("--points", type=float, default=1e9)
     ap.add_argument("--ranks", default="2,4,8")
     ap.add_argument("--steps", type=int, default=10)
+    ap.add_argument("--only-rank", type=int, default=-1, help="profile: run only this rank's spatial shard")
     args = ap.parse_args()
     n = int(args.points)
     box, polys_name, recipe, q, desc_s = bench.workload(args.config)
@@ -79,9 +80,9 @@ def main():
         for a in range(0, n, 1 << 26):              # chunked: int64 ranks for 1e9 points would be 8 GB
             dest[a:a + (1 << 26)] = rjdist.strip_of(torch.from_numpy(x[a:a + (1 << 26)]), sp).numpy()
         res = {}
-        for kind in ("range", "spatial"):
+        for kind in (("spatial",) if args.only_rank >= 0 else ("range", "spatial")):
             per, tot = [], np.zeros_like(c1)
-            for r in range(P):
+            for r in (range(P) if args.only_rank < 0 else [args.only_rank]):
                 if kind == "range":
                     lo, hi = rjdist.shard_range(n, r, P)
                     sel = slice(lo, hi)
@@ -97,7 +98,8 @@ def main():
                             "point_pass_ms": st["ms_point_pass"]})
             worst = max(p["ms"] for p in per)
             res[kind] = {"max_rank_ms": worst, "projected_efficiency": t1 / (P * worst),
-                         "sum_equals_1gpu": bool(np.array_equal(tot, c1)), "per_rank": per}
+                         "sum_equals_1gpu": bool(np.array_equal(tot, c1)) if args.only_rank < 0 else None,
+                         "per_rank": per}
         out["ranks"][P] = res
         print(json.dumps({"P": P, **{k: {kk: vv for kk, vv in v.items() if kk != "per_rank"}
                                        for k, v in res.items()}}), flush=True)

@@ -310,8 +310,14 @@ def main():
     R.set_option(rj.OPT_TIMING, 1)
     pp_ms, poly_ms = [], []
 
+    step_ev = []
+
     def timed_step():
+        e_a, e_b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        e_a.record(stream)
         step()
+        e_b.record(stream)
+        step_ev.append((e_a, e_b))
         s_ = R.stats()
         pp_ms.append(s_["ms_point_pass"])
         poly_ms.append(s_["ms_polygon"])
@@ -336,6 +342,7 @@ def main():
         ms = float(t.item())
         dist.barrier()
     ms_step = ms / args.steps
+    lat = [a.elapsed_time(b) for a, b in step_ev]        # per-step latency (this rank)
     value = n_total / (ms_step / 1e3)
 
     # sanity: exact tiling -> every filtered point lands in exactly one polygon
@@ -418,6 +425,7 @@ def main():
                        "one NCCL allreduce of per-polygon partials" if world > 1 else "1 GPU",
                        "rank0_view": view, "l2": "inputs (>= 12 GB) larger than L2, no flush needed"},
             "latency_ms": ms_step,
+            "latency_ms_p50": float(np.percentile(lat, 50)), "latency_ms_p90": float(np.percentile(lat, 90)),
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                          "frac": achieved / peak, "traffic": ncu_traffic(args.config),
                          "kernel": "k_point_pass (fused filter+project+tile scatter+span reduce)",

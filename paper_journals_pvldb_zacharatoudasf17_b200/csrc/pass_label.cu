@@ -345,6 +345,16 @@ size_t point_pass_label_smem(const PassArgs &a, bool accurate) { return label_sm
 rj_status point_pass_label(Ctx *c, const PassArgs &a_in, bool accurate) {
     PassArgs a = a_in;
     a.n_stages = (uint32_t)choose_stages(a, label_smem, true, accurate, c->force_stages);
+    if (a.smem_partials && a.n_stages < 3 && !c->force_stages) {
+        // A deeper ring beats shared-memory count partials: the sums already
+        // reduce in global memory, and Morton-ordered label runs make the
+        // count reductions rare.  Two stages of 2048 points leave too few
+        // bytes in flight per SM to cover HBM latency.
+        PassArgs b = a;
+        b.smem_partials = 0;
+        b.n_stages = (uint32_t)choose_stages(b, label_smem, true, accurate, 0);
+        if (b.n_stages >= 3) a = b;
+    }
     if (!a.n_stages) return set_error(c, RJ_ERR_RESOLUTION, "point-pass tiles do not fit in shared memory");
     const bool fp = a.f.n_fpred > 0;
     const bool af = a.f.agg_is_float != 0;

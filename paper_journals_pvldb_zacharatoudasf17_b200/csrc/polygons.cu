@@ -165,7 +165,7 @@ struct SpanGeo {
     const uint32_t *prow_off;   // [n_poly + 1]
     uint32_t n_poly;
     const int4 *mbr;
-    const uint32_t *cell_off10; // point cells: skip pieces of empty cells
+    const uint32_t *cell_bits;  // level-L point cells holding points (pieces of empty cells are skipped)
     int32_t c0, r0, c1, r1;     // viewport window (reading Z20): spans are clipped to it
 };
 
@@ -186,19 +186,39 @@ __device__ __forceinline__ void polyrow_of(const SpanGeo &g, uint32_t pr, uint32
 template <class F>
 __device__ __forceinline__ void for_each_piece(const SpanGeo &g, int64_t r, int64_t lo, int64_t hi, F f) {
     if (g.L < 0) return;                                   // spans only
-    const int s = kLatticeBits - g.L, sh = 2 * (kMaxLevel - g.L);
+    const int s = kLatticeBits - g.L;
     const int64_t cr0 = qlo(r, g.H) >> s, cr1 = qhi(r, g.H) >> s;
     const int64_t cc0 = qlo(lo, g.W) >> s, cc1 = qhi(hi - 1, g.W) >> s;
     for (int64_t cr = cr0; cr <= cr1; ++cr) {
         const int64_t r0 = cell_pix_lo(cr, g.H, g.L);
         for (int64_t cc = cc0; cc <= cc1; ++cc) {
             const uint32_t cell = spread16((uint32_t)cc) | (spread16((uint32_t)cr) << 1);
-            if (g.cell_off10[(uint64_t)(cell + 1) << sh] == g.cell_off10[(uint64_t)cell << sh]) continue;  // no points
+            if (!((__ldg(&g.cell_bits[cell >> 5]) >> (cell & 31)) & 1u)) continue;  // no points
             const int64_t c0 = cell_pix_lo(cc, g.W, g.L), c1 = cell_pix_hi(cc, g.W, g.L);
             const int64_t a = max(lo, c0) - c0, b = min(hi, c1 + 1) - c0;
             f(cell, (uint32_t)(r - r0), (uint32_t)a, (uint32_t)b);
         }
     }
+}
+
+// Sort m <= N values in place through registers (compare-exchange insertion
+// network, fully unrolled; padding with UINT32_MAX keeps it in place).
+template <int N>
+__device__ __forceinline__ void sort_small(uint32_t *p, uint32_t m) {
+    uint32_t r[N];
+#pragma unroll
+    for (int i = 0; i < N; ++i) r[i] = (uint32_t)i < m ? p[i] : 0xFFFFFFFFu;
+#pragma unroll
+    for (int i = 1; i < N; ++i)
+#pragma unroll
+        for (int j = i; j > 0; --j) {
+            const uint32_t lo = min(r[j - 1], r[j]), hi = max(r[j - 1], r[j]);
+            r[j - 1] = lo;
+            r[j] = hi;
+        }
+#pragma unroll
+    for (int i = 0; i < N; ++i)
+        if ((uint32_t)i < m) p[i] = r[i];
 }
 
 // Sort each (polygon,row) threshold list, count its spans and their pieces.
@@ -207,11 +227,23 @@ __global__ void k_prow_count(SpanGeo g, uint32_t n_prow, const uint32_t *__restr
                              uint32_t *__restrict__ piece_cnt) {
     for (uint32_t pr = blockIdx.x * blockDim.x + threadIdx.x; pr < n_prow; pr += gridDim.x * blockDim.x) {
         const uint32_t b = pr_off[pr], e = pr_off[pr + 1];
-        for (uint32_t i = b + 1; i < e; ++i) {
-            const uint32_t v = tv[i];
-            uint32_t j = i;
-            while (j > b && tv[j - 1] > v) { tv[j] = tv[j - 1]; --j; }
-            tv[j] = v;
+        const uint32_t m = e - b;                            // the usual case: sort in registers
+        if (m <= 2) {
+            if (m == 2) {
+                const uint32_t u = tv[b], v = tv[b + 1];
+                if (u > v) { tv[b] = v; tv[b + 1] = u; }
+            }
+        } else if (m <= 4) {
+            sort_small<4>(tv + b, m);
+        } else if (m <= 16) {
+            sort_small<16>(tv + b, m);
+        } else {
+            for (uint32_t i = b + 1; i < e; ++i) {
+                const uint32_t v = tv[i];
+                uint32_t j = i;
+                while (j > b && tv[j - 1] > v) { tv[j] = tv[j - 1]; --j; }
+                tv[j] = v;
+            }
         }
         uint32_t P;
         int64_t r;
@@ -244,10 +276,28 @@ __global__ void k_prow_emit(SpanGeo g, uint32_t n_prow, const uint32_t *__restri
             if (!clip_span(g, r, lo, hi)) continue;
             uint32_t *s = spans + 4 * (uint64_t)k++;
             s[0] = P; s[1] = (uint32_t)r; s[2] = (uint32_t)lo; s[3] = (uint32_t)hi;
+            // batches of 8 pieces: the slot atomics of a batch are all in
+            // flight together instead of one L2 round trip per piece
+            constexpr int kB = 8;
+            uint32_t bc[kB], bv[kB];
+            int nb = 0;
+            auto flush = [&]() {
+                uint32_t slot[kB];
+#pragma unroll
+                for (int q = 0; q < kB; ++q)
+                    if (q < nb) slot[q] = atomicAdd(&piece_cur[bc[q]], 1u);
+#pragma unroll
+                for (int q = 0; q < kB; ++q)
+                    if (q < nb) pieces[piece_off[bc[q]] + slot[q]] = make_uint2(P, bv[q]);
+                nb = 0;
+            };
             for_each_piece(g, r, lo, hi, [&](uint32_t cell, uint32_t lr, uint32_t a, uint32_t bb) {
-                const uint32_t slot = piece_off[cell] + atomicAdd(&piece_cur[cell], 1u);
-                pieces[slot] = make_uint2(P, lr | (a << 8) | (bb << 16));
+#pragma unroll
+                for (int q = 0; q < kB; ++q)
+                    if (q == nb) { bc[q] = cell; bv[q] = lr | (a << 8) | (bb << 16); }
+                if (++nb == kB) flush();
             });
+            if (nb) flush();
         }
     }
 }
@@ -502,7 +552,7 @@ rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp,
     k_scatter_t<<<gx, 256, 0, st>>>(cpr.as<uint32_t>(), ct.as<uint32_t>(), X, pro.as<uint32_t>(),
                                     prcur.as<uint32_t>(), tv.as<uint32_t>());
     RJ_LAUNCHED(c);
-    SpanGeo g{W, H, L, proff.as<uint32_t>(), np, c->mbr.as<int4>(), c->cell_off.as<uint32_t>(),
+    SpanGeo g{W, H, L, proff.as<uint32_t>(), np, c->mbr.as<int4>(), L >= 0 ? c->cell_bits[L].as<uint32_t>() : nullptr,
               v.full ? 0 : v.c0, v.full ? 0 : v.r0, v.full ? W : v.c1, v.full ? H : v.r1};
     const unsigned gp = (unsigned)std::min<uint64_t>(std::max<uint64_t>(1, blocks_for(NPR, 128)), c->num_sms * 16ull);
     k_prow_count<<<gp, 128, 0, st>>>(g, NPR, pro.as<uint32_t>(), tv.as<uint32_t>(), scnt.as<uint32_t>(),

@@ -116,6 +116,7 @@ struct Ctx {
     Buf cell_off;                 // [kCells10 + 1]
     std::vector<uint32_t> h_cell_off;          // host copy (work-item planning)
     Buf items[kMaxLevel + 1];                  // per level L: int4 work items
+    Buf cell_bits[kMaxLevel + 1];              // per level L: bit per point cell, set when it holds points
     uint32_t n_items[kMaxLevel + 1] = {};
     int64_t items_chunk[kMaxLevel + 1] = {};
 

@@ -23,6 +23,7 @@ int choose_level(int W, int H, int target) {
 void drop_items(Ctx *c) {
     for (int L = 0; L <= kMaxLevel; ++L) {
         dfree(c, c->items[L]);
+        dfree(c, c->cell_bits[L]);
         c->n_items[L] = 0;
         c->items_chunk[L] = 0;
     }
@@ -70,6 +71,14 @@ rj_status items_for_level(Ctx *c, int L) {
         gcells += 1;
     }
     flush();
+    // non-empty point cells of the level as a bitmask (the polygon pass skips
+    // span pieces of empty cells with one L1-friendly word load)
+    std::vector<uint32_t> bits((ncell + 31) / 32, 0u);
+    for (uint64_t cc = 0; cc < ncell; ++cc)
+        if (off[(cc + 1) << sh] != off[cc << sh]) bits[cc >> 5] |= 1u << (cc & 31);
+    dfree(c, c->cell_bits[L]);
+    if (dalloc(c, c->cell_bits[L], bits.size() * 4)) return set_error(c, RJ_ERR_OOM, "cell mask allocation failed");
+    RJ_CUDA(c, cudaMemcpyAsync(c->cell_bits[L].p, bits.data(), bits.size() * 4, cudaMemcpyHostToDevice, c->stream));
     dfree(c, c->items[L]);
     if (dalloc(c, c->items[L], std::max<size_t>(1, items.size()) * sizeof(int4)))
         return set_error(c, RJ_ERR_OOM, "work item allocation failed");

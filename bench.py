@@ -248,9 +248,16 @@ def main():
         # every point to the rank owning its x strip; each rank then queries
         # only its strip's pixel window.  Load-time, outside the timed region.
         t0 = time.perf_counter()
-        dx, dy, dcols, splitters = rjdist.spatial_shard(
-            torch.from_numpy(x).cuda(), torch.from_numpy(y).cuda(), [torch.from_numpy(c).cuda() for c in cols],
-            world)
+        gx, gy, gcols = torch.from_numpy(x).cuda(), torch.from_numpy(y).cuda(), [torch.from_numpy(c).cuda() for c in cols]
+        # release the generated pinned host columns before pinning the received
+        # ones (8 ranks x 2 x 12 GB of pinned memory would not fit a host)
+        del x, y, cols
+        import gc
+        gc.collect()
+        if hasattr(torch._C, "_host_emptyCache"):
+            torch._C._host_emptyCache()
+        dx, dy, dcols, splitters = rjdist.spatial_shard(gx, gy, gcols, world)
+        del gx, gy, gcols
         def pin(t):
             h = torch.empty(t.numel(), dtype=t.dtype, pin_memory=True)
             h.copy_(t)

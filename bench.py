@@ -206,6 +206,7 @@ def main():
     ap.add_argument("--pass-variant", type=int, default=-1, help="SUM/AVG kernel: 0 label, 1 pixel tile")
     ap.add_argument("--stages", type=int, default=0, help="point-pass ring depth (0 = library default)")
     ap.add_argument("--mode", default="", help="override the config's mode: bounded|accurate|index|exact")
+    ap.add_argument("--no-graphs", action="store_true", help="launch every query eagerly (no CUDA-graph replay)")
     ap.add_argument("--shard", default="spatial", choices=("spatial", "range"),
                     help="N > 1: x-strip shards via all_to_all + per-rank pixel windows, or plain index ranges")
     args = ap.parse_args()
@@ -277,6 +278,8 @@ def main():
         R.set_option(rj.OPT_STAGES, args.stages)
     if args.pass_variant >= 0:
         R.set_option(rj.OPT_PASS, args.pass_variant)
+    if args.no_graphs:
+        R.set_option(rj.OPT_GRAPHS, 0)
     flat = C.array_polys(polys_name)
     t0 = time.perf_counter()
     n_ood = R.load_points(x, y, cols)

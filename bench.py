@@ -257,7 +257,7 @@ def main():
         gc.collect()
         if hasattr(torch._C, "_host_emptyCache"):
             torch._C._host_emptyCache()
-        dx, dy, dcols, splitters = rjdist.spatial_shard(gx, gy, gcols, world)
+        dx, dy, dcols, splitters = rjdist.spatial_shard(gx, gy, gcols, world, box=box, poly_weight=0.1)
         del gx, gy, gcols
         def pin(t):
             h = torch.empty(t.numel(), dtype=t.dtype, pin_memory=True)

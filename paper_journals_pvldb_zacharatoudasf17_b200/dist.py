@@ -72,9 +72,10 @@ def query_sharded(R: "rj.RasterJoin", desc, d_count: torch.Tensor, d_sum: torch.
 # with disjoint points, and the per-polygon partials still just add
 # (distributivity), so no pixel ownership is needed.
 
-def strip_splitters(x: torch.Tensor, world: int, group=None, sample: int = 1 << 16) -> torch.Tensor:
+def strip_splitters(x: torch.Tensor, world: int, group=None, sample: int = 1 << 16, box=None,
+                    poly_weight: float = 0.0) -> torch.Tensor:
     """world-1 increasing x splitters (float64, on x's device) giving strips
-    of about equal point count over all ranks' points."""
+    of about equal cost over all ranks' points (see splitters_from_sample)."""
     n = x.numel()
     if n:
         idx = torch.linspace(0, n - 1, sample, device=x.device).round().long()
@@ -83,15 +84,29 @@ def strip_splitters(x: torch.Tensor, world: int, group=None, sample: int = 1 << 
         s = torch.full((sample,), float("nan"), dtype=torch.float64, device=x.device)
     parts = [torch.empty_like(s) for _ in range(world)]
     dist.all_gather(parts, s, group=group)
-    return splitters_from_sample(torch.cat(parts), world)
+    return splitters_from_sample(torch.cat(parts), world, box, poly_weight)
 
 
-def splitters_from_sample(allv: torch.Tensor, world: int) -> torch.Tensor:
-    """The k/world quantiles (k = 1..world-1) of a sample of x (NaN ignored)."""
+def splitters_from_sample(allv: torch.Tensor, world: int, box=None, poly_weight: float = 0.0) -> torch.Tensor:
+    """Splitters at the k/world quantiles (k = 1..world-1) of the strip cost
+    (1 - w) * (share of the points) + w * (share of the domain width) over a
+    sample of x (NaN ignored).  w = poly_weight = 0 balances points only; a
+    rank's polygon pass grows with its strip's width (it rasterises the
+    polygons of its window), so w ~ the polygon pass's share of a one-GPU
+    query balances the two."""
     allv = torch.sort(allv[~torch.isnan(allv)].to(torch.float64)).values
-    if allv.numel() == 0:
+    n = allv.numel()
+    if n == 0:
         return torch.zeros(world - 1, dtype=torch.float64, device=allv.device)
-    k = torch.arange(1, world, device=allv.device) * allv.numel() // world
+    if poly_weight <= 0.0 or box is None:
+        k = torch.arange(1, world, device=allv.device) * n // world
+        return allv[k]
+    w = float(poly_weight)
+    cost = (1.0 - w) * torch.arange(1, n + 1, device=allv.device, dtype=torch.float64) / n + \
+        w * ((allv - box[0]) / (box[2] - box[0])).clamp(0.0, 1.0)
+    cost, _ = torch.cummax(cost, 0)
+    q = torch.arange(1, world, device=allv.device, dtype=torch.float64) / world
+    k = torch.searchsorted(cost, q).clamp(max=n - 1)
     return allv[k]
 
 
@@ -131,10 +146,10 @@ def strip_window(box, splitters, rank: int, world: int, W: int, H: int):
     return (c0, 0, max(c1, c0 + 1), H)
 
 
-def spatial_shard(x, y, cols, world: int, group=None):
+def spatial_shard(x, y, cols, world: int, group=None, box=None, poly_weight: float = 0.0):
     """Load-time exchange: (x, y, cols) of this rank's index range ->
     (x, y, cols, splitters) of its x strip."""
-    sp = strip_splitters(x, world, group)
+    sp = strip_splitters(x, world, group, box=box, poly_weight=poly_weight)
     dest = strip_of(x, sp)
     got = exchange([x, y, *cols], dest, world, group)
     return got[0], got[1], got[2:], sp

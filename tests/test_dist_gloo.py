@@ -147,3 +147,26 @@ def test_spatial_shards_allreduce_to_unsharded(world):
                                  W=4096, H=4096, mode=mode)
         assert np.array_equal(gc, cnt.astype(np.int64)), mode
         assert np.allclose(gs, s, rtol=1e-12, atol=0), mode
+
+
+def test_splitters_from_sample_cost_rule():
+    """poly_weight = 0: point quantiles; = 1: equal-width strips; between:
+    monotone in the weight (wider sparse strips shrink)."""
+    from paper_journals_pvldb_zacharatoudasf17_b200 import dist as rjdist
+
+    g = torch.Generator().manual_seed(3)
+    v = torch.rand(200_000, generator=g, dtype=torch.float64) ** 3 * 100.0
+    box = (0.0, 0.0, 100.0, 50.0)
+    q = rjdist.splitters_from_sample(v, 4)
+    assert torch.allclose(q, torch.quantile(v, torch.tensor([0.25, 0.5, 0.75], dtype=torch.float64)), atol=0.05)
+    e = rjdist.splitters_from_sample(v, 4, box, 1.0)
+    assert torch.allclose(e, torch.tensor([25.0, 50.0, 75.0], dtype=torch.float64), atol=0.05)
+    prev = q
+    for w in (0.1, 0.3, 0.6, 0.9):
+        s = rjdist.splitters_from_sample(v, 4, box, w)
+        assert torch.all(s[1:] > s[:-1])
+        assert torch.all(s >= prev - 1e-9)          # the skewed sample: splitters move right with w
+        prev = s
+    v2 = v.clone()
+    v2[::7] = float("nan")
+    assert torch.all(torch.isfinite(rjdist.splitters_from_sample(v2, 8, box, 0.2)))

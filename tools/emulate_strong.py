@@ -59,6 +59,8 @@ def main():
     ap.add_argument("--ranks", default="2,4,8")
     ap.add_argument("--steps", type=int, default=10)
     ap.add_argument("--only-rank", type=int, default=-1, help="profile: run only this rank's spatial shard")
+    ap.add_argument("--poly-weight", type=float, default=0.0, help="strip cost weight of the domain width")
+    ap.add_argument("--spatial-only", action="store_true")
     args = ap.parse_args()
     n = int(args.points)
     box, polys_name, recipe, q, desc_s = bench.workload(args.config)
@@ -75,12 +77,12 @@ def main():
            "t1_polygon_ms": st1["ms_polygon"], "ranks": {}}
     sample = torch.from_numpy(x[np.linspace(0, n - 1, 1 << 20).astype(np.int64)].astype(np.float64))
     for P in [int(v) for v in args.ranks.split(",")]:
-        sp = rjdist.splitters_from_sample(sample, P)
+        sp = rjdist.splitters_from_sample(sample, P, box, args.poly_weight)
         dest = np.empty(n, dtype=np.uint8)
         for a in range(0, n, 1 << 26):              # chunked: int64 ranks for 1e9 points would be 8 GB
             dest[a:a + (1 << 26)] = rjdist.strip_of(torch.from_numpy(x[a:a + (1 << 26)]), sp).numpy()
         res = {}
-        for kind in (("spatial",) if args.only_rank >= 0 else ("range", "spatial")):
+        for kind in (("spatial",) if args.only_rank >= 0 or args.spatial_only else ("range", "spatial")):
             per, tot = [], np.zeros_like(c1)
             for r in (range(P) if args.only_rank < 0 else [args.only_rank]):
                 if kind == "range":

@@ -275,7 +275,7 @@ static cudaError_t record_ev(Ctx *c, int i) {
 
 // Everything up to (not including) the point-pass launch.
 static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_polygon_pass = true,
-                         bool bands = false) {
+                         bool bands = false, bool need_mask = false) {
     rj_status s = check_ready(c, q);
     if (s != RJ_OK) return s;
     if ((s = resolve(c->x0, c->y0, c->x1, c->y1, q, &P.W, &P.H)) != RJ_OK)
@@ -313,7 +313,7 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     // the index join needs neither spans nor the boundary mask
     P.pp = PolyPass{};
     if (need_polygon_pass && !P.index &&
-        (s = polygon_pass(c, P.W, P.H, P.L, P.acc || bands, P.pp, P.view)) != RJ_OK)
+        (s = polygon_pass(c, P.W, P.H, P.L, P.acc || bands, P.pp, P.view, need_mask && P.acc)) != RJ_OK)
         return s;
     if (c->timing) RJ_CUDA(c, record_ev(c, 1));
     a.qx = c->qx.as<uint32_t>();
@@ -956,7 +956,7 @@ rj_status rj_debug_boundary_mask(rj_ctx *c, const rj_query_desc *q, uint32_t *bi
     rj_query_desc qq = *q;
     qq.mode = RJ_ACCURATE;
     Prepared P;
-    rj_status s = prepare(c, &qq, P);
+    rj_status s = prepare(c, &qq, P, true, false, true);
     if (s != RJ_OK) return s;
     RJ_CUDA(c, cudaMemcpyAsync(bits, P.pp.mask, (uint64_t)P.pp.mask_wpr * P.H * 4, cudaMemcpyDeviceToHost, c->stream));
     RJ_CUDA(c, cudaStreamSynchronize(c->stream));
@@ -966,7 +966,7 @@ rj_status rj_debug_boundary_mask(rj_ctx *c, const rj_query_desc *q, uint32_t *bi
 rj_status rj_debug_point_membership(rj_ctx *c, const rj_query_desc *q, uint64_t *bits) {
     if (!bits) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL bits");
     Prepared P;
-    rj_status s = prepare(c, q, P);
+    rj_status s = prepare(c, q, P, true, false, true);
     if (s != RJ_OK) return s;
     Buf d;
     if (dalloc(c, d, std::max<uint64_t>(1, c->n_in) * 8)) return set_error(c, RJ_ERR_OOM, "allocation failed");

@@ -364,7 +364,7 @@ rj_status label_query_impl(Ctx *c, const Filter &f, const AggPlan &ap, int W, in
     // ---- label canvas (S3 spans painted, S5 mask) + row index of the spans
     PolyPass pp;
     rj_status s;
-    if (!index && (s = polygon_pass(c, W, H, -1, acc, pp, v)) != RJ_OK) return s;
+    if (!index && (s = polygon_pass(c, W, H, -1, acc, pp, v, acc)) != RJ_OK) return s;
     const uint64_t S = pp.n_spans;
     const uint32_t vc0 = v.full ? 0u : (uint32_t)v.c0, vr0 = v.full ? 0u : (uint32_t)v.r0;
     const uint32_t vw = v.full ? (uint32_t)W : (uint32_t)(v.c1 - v.c0), vh = v.full ? (uint32_t)H : (uint32_t)(v.r1 - v.r0);

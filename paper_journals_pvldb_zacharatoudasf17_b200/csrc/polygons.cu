@@ -488,7 +488,7 @@ rj_status load_polygons_impl(Ctx *c, uint32_t n_poly, const uint32_t *pro, const
 }
 
 // ------------------------------------------------------------ per-query pass
-rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp, const View &v) {
+rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp, const View &v, bool need_mask) {
     // L < 0: spans (and mask) only, no pieces (the streamed query)
     const uint64_t ncell = L >= 0 ? 1ull << (2 * L) : 0;
     const uint32_t ne = c->n_edges, np = c->n_poly;
@@ -617,8 +617,10 @@ rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp,
     pp.spans = spans.as<uint32_t>();
     pp.piece_off = poff.as<uint32_t>();
     pp.pieces = pieces.as<uint2>();
-    if (accurate) {
-        pp.n_bands = B;
+    if (accurate) pp.n_bands = B;
+    if (accurate && need_mask) {
+        // the bitmask is only read by the diagnostics and the streamed
+        // (label-canvas) query: the point-pass kernels take bpieces
         const uint32_t wpr = (uint32_t)((W + 31) / 32);
         Buf &mask = wsbuf(c, kWsMask);
         if (dreserve(c, mask, (uint64_t)wpr * H * 4)) return set_error(c, RJ_ERR_OOM, "mask allocation failed");

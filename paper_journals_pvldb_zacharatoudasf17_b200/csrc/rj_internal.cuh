@@ -258,7 +258,7 @@ struct PolyPass {
     uint64_t n_bpieces = 0;
 };
 // Spans, pieces and the boundary mask are clipped to the viewport window v.
-rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp, const View &v);
+rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp, const View &v, bool need_mask);
 
 // interval.cu: bounded-mode worst-case result intervals from the
 // per-pixel count canvas, the spans and the S5 bands of the polygon pass.

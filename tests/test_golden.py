@@ -30,8 +30,11 @@ def _load(path):
     return g, PG.flatten(polys), pts[:, 0].copy(), pts[:, 1].copy(), t
 
 
-CASES = [("bounded", []), ("accurate", []),
-         ("bounded_t_le_6", [(0, "<=", 6)]), ("accurate_t_le_6", [(0, "<=", 6)])]
+def _cases(g):
+    """(key, mode, preds) for every expected query result of a fixture."""
+    for key, e in g["expected"].items():
+        if "mode" in e:
+            yield key, e["mode"], [tuple(p) for p in e.get("preds", [])]
 
 
 def _check(g, key, cnt, s, avg=None):
@@ -48,8 +51,7 @@ def test_golden_oracle(path):
     g, flat, x, y, t = _load(path)
     P = oracle.Polys(flat, g["domain"])
     W, H = g["canvas"]
-    for key, preds in CASES:
-        mode = key.split("_")[0]
+    for key, mode, preds in _cases(g):
         cnt, s, kept = oracle.query(P, x, y, cols=[t], preds=preds, agg_col=0, W=W, H=H, mode=mode)
         _check(g, key, cnt, s, oracle.avg(cnt, s))
         if not preds:
@@ -74,8 +76,7 @@ def test_golden_gpu(path):
     assert int(n_ood) == g["n_out_of_domain"]
     R.load_polygons(flat)
     W, H = g["canvas"]
-    for key, preds in CASES:
-        mode = key.split("_")[0]
+    for key, mode, preds in _cases(g):
         cnt, s = R.query(agg="sum", agg_column=0, preds=preds, W=W, H=H, mode=mode)
         _, a = R.query(agg="avg", agg_column=0, preds=preds, W=W, H=H, mode=mode)
         _check(g, key, cnt, s, a)

@@ -62,8 +62,6 @@ def lib():
         L.or_membership.restype = None
         L.or_membership.argtypes = [vp, u64, vp, vp, i32, d, d, d, d, i32, vp, vp, i32, vp, vp, vp,
                                     i32, i32, i32, vp, vp]
-        L.or_pixel_membership.restype = None
-        L.or_pixel_membership.argtypes = [vp, i32, i32, vp]
         L.or_pixel_spans.restype = i64
         L.or_pixel_spans.argtypes = [vp, i64, i32, i32, i64, vp]
         L.or_seg_rect.restype = i32
@@ -195,12 +193,6 @@ def membership(polys, x, y, cols=(), preds=(), W=1024, H=1024, mode="bounded", v
     lib().or_membership(polys.h, len(x), x.ctypes.data, y.ctypes.data, f64, *polys.box, *c.args(),
                         *c.pargs(), int(W), int(H), 0 if mode == "bounded" else 1, bits.ctypes.data, vp)
     return bits
-
-
-def pixel_membership(polys, W, H):
-    out = np.zeros((H, W), dtype=np.uint64)
-    lib().or_pixel_membership(polys.h, int(W), int(H), out.ctypes.data)
-    return out
 
 
 def pixel_spans(polys, P, W, H):

@@ -437,26 +437,12 @@ OR_EXPORT void or_membership(const or_polys *p, uint64_t n, const void *x, const
     }
 }
 
-/* Bounded-mode pixel membership by brute force: out[r*W + i] bit P set iff
- * the centre of pixel (i, r) is inside polygon P (first 64 polygons). */
-OR_EXPORT void or_pixel_membership(const or_polys *p, int W, int H, uint64_t *out) {
-    int64_t np = p->n_poly < 64 ? p->n_poly : 64;
-    #pragma omp parallel for schedule(dynamic, 4)
-    for (int r = 0; r < H; ++r) {
-        int64_t cy = or_centre(r, H);
-        for (int i = 0; i < W; ++i) {
-            int64_t cx = or_centre(i, W);
-            uint64_t m = 0;
-            for (int64_t P = 0; P < np; ++P)
-                if (or_contains(p, P, cx, cy)) m |= (uint64_t)1 << P;
-            out[(size_t)r * W + i] = m;
-        }
-    }
-}
-
-/* Pixel spans of one polygon from brute-force centre membership:
- * writes (row, lo, hi) triples, hi exclusive; returns the count (or the
- * required count if it exceeds cap). */
+/* Pixel spans of one polygon from brute-force centre membership (O2 + O3,
+ * pixel-centre rule P:561-562): every pixel centre of every row is tested
+ * with O3, and maximal runs of inside centres are written as (row, lo, hi)
+ * triples, hi exclusive; returns the count (or the required count if it
+ * exceeds cap).  Pinned by tests/test_oracle_pins.py
+ * test_pixel_spans_rectilinear_closed_form / _triangle_halfplanes. */
 OR_EXPORT int64_t or_pixel_spans(const or_polys *p, int64_t P, int W, int H, int64_t cap, int32_t *out) {
     int64_t ns = 0;
     for (int r = 0; r < H; ++r) {

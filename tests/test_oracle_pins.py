@@ -261,6 +261,95 @@ def test_c1_convex_polys_halfplane(c1):
         assert np.array_equal(got[~zero].astype(bool), ins[~zero])
 
 
+# ---------------------------------------------------------- O2/O3 pixel spans
+# or_pixel_spans is the expected value of the GPU span test (S3): its pins are
+# closed forms in exact integer arithmetic on the REAL pixel centres
+# cx(i) = (2i+1)*512/W world units on the C1 domain [0,1024) (P:561-562
+# pixel-centre rule), not the oracle's floored lattice centres: for a
+# rectilinear polygon with integer or half-integer vertices, floor(c*2^20) >= k
+# iff c*2^20 >= k for an integer lattice value k, so the two agree exactly.
+
+# rectilinear C1 polygons as signed half-open rectangles (x0, x1, y0, y1, sign)
+_RECTS = {
+    0: [(100, 200, 100, 200, 1)],
+    1: [(300.5, 400.5, 100.5, 200.5, 1)],
+    4: [(100, 300, 400, 450, 1), (100, 150, 450, 600, 1)],                    # L-shape
+    6: [(700, 950, 400, 650, 1), (775, 875, 475, 575, -1)],                   # annulus
+    7: [(100, 400, 700, 750, 1)] + [(a, a + 50, 750, 950, 1) for a in (150, 250, 350)],   # comb
+    8: [(820, 1000, 150, 330, 1)],
+    9: [(200, 300, 100, 200, 1)],
+}
+
+
+def _centre_in(v0, v1, k, n):
+    """v0 <= (2k+1)*512/n < v1 for integer arrays k (2*v integer): exact."""
+    t = (2 * k + 1) * 1024
+    return (int(round(2 * v0)) * n <= t) & (t < int(round(2 * v1)) * n)
+
+
+def _runs(row_mask):
+    out = []
+    for r in range(row_mask.shape[0]):
+        m = np.concatenate([[0], row_mask[r].astype(np.int8), [0]])
+        d = np.diff(m)
+        for lo, hi in zip(np.nonzero(d == 1)[0], np.nonzero(d == -1)[0]):
+            out.append((r, lo, hi))
+    return np.asarray(out, dtype=np.int64).reshape(-1, 3)
+
+
+@pytest.mark.parametrize("W,H", [(1024, 1024), (333, 517), (64, 48), (1500, 97)])
+def test_pixel_spans_rectilinear_closed_form(W, H):
+    polys = oracle.Polys(PG.flatten(C.polygon_set("c1")), C1)
+    cols, rows = np.arange(W, dtype=np.int64), np.arange(H, dtype=np.int64)
+    for pid, rects in _RECTS.items():
+        m = np.zeros((H, W), dtype=np.int64)
+        for x0, x1, y0, y1, sg in rects:
+            m += sg * np.outer(_centre_in(y0, y1, rows, H), _centre_in(x0, x1, cols, W)).astype(np.int64)
+        assert m.min() >= 0 and m.max() <= 1
+        got = oracle.pixel_spans(polys, pid, W, H).astype(np.int64)
+        assert np.array_equal(got, _runs(m)), (pid, W, H)
+    # the hand-readable case: P0 at 1024^2 is rows 100..199, each [100, 200);
+    # P1's centres i + 0.5 lie in [300.5, 400.5) for i = 300..399
+    sp0 = oracle.pixel_spans(polys, 0, 1024, 1024)
+    assert sp0.tolist() == [[r, 100, 200] for r in range(100, 200)]
+    sp1 = oracle.pixel_spans(polys, 1, 1024, 1024)
+    assert sp1.tolist() == [[r, 300, 400] for r in range(100, 200)]
+    # comb row 800 (y = 800.5): three teeth [150,200), [250,300), [350,400)
+    sp7 = oracle.pixel_spans(polys, 7, 1024, 1024)
+    assert sp7[sp7[:, 0] == 800][:, 1:].tolist() == [[150, 200], [250, 300], [350, 400]]
+    # annulus row 500 crosses the hole: [700,775) and [875,950)
+    sp6 = oracle.pixel_spans(polys, 6, 1024, 1024)
+    assert sp6[sp6[:, 0] == 500][:, 1:].tolist() == [[700, 775], [875, 950]]
+
+
+@pytest.mark.parametrize("W,H", [(1024, 1024), (333, 517), (777, 211)])
+def test_pixel_spans_triangle_halfplanes(W, H):
+    """P2 (convex triangle, CCW): a centre is inside iff it is strictly left of
+    all three edges.  Exact integer orientation at the real centre
+    ((2i+1)*512/W, (2r+1)*512/H), scaled by W*H; pixels whose centre lies
+    within 2^-18 world units of an edge line are left out (the lattice floor
+    moves a centre by < 2^-19; exact ties are the half-open rule's, pinned by
+    test_rectangle_half_open_ties)."""
+    polys = oracle.Polys(PG.flatten(C.polygon_set("c1")), C1)
+    ring = np.asarray(C.polygon_set("c1")[2][0], dtype=np.int64)
+    i = np.arange(W, dtype=np.int64)[None, :]
+    r = np.arange(H, dtype=np.int64)[:, None]
+    cxs = (2 * i + 1) * 512 * H           # centre x * W * H
+    cys = (2 * r + 1) * 512 * W           # centre y * W * H
+    ins = np.ones((H, W), dtype=bool)
+    near = np.zeros((H, W), dtype=bool)
+    for (xa, ya), (xb, yb) in zip(ring, np.roll(ring, -1, axis=0)):
+        cr = (xb - xa) * (cys - ya * W * H) - (yb - ya) * (cxs - xa * W * H)
+        ins &= cr > 0
+        near |= np.abs(cr) <= math.hypot(xb - xa, yb - ya) * W * H * 2.0 ** -18
+    got = np.zeros((H, W), dtype=bool)
+    for row, lo, hi in oracle.pixel_spans(polys, 2, W, H).tolist():
+        assert not got[row, lo:hi].any()               # spans are disjoint, sorted
+        got[row, lo:hi] = True
+    assert near.sum() < 0.02 * ins.sum() and ins.sum() > 0
+    assert np.array_equal(got[~near], ins[~near]), (W, H)
+
+
 # ------------------------------------------------------------------ filters/SUM
 def test_filter_identity_and_sum_identities():
     polys = oracle.Polys(C.array_polys("c1"), C1)

@@ -19,7 +19,7 @@ OBJ = os.path.join(ROOT, "build", "rj")
 NVCC = os.environ.get("NVCC", "/usr/local/cuda/bin/nvcc")
 FLAGS = ["-O3", "-std=c++17", "-gencode", "arch=compute_100a,code=sm_100a", "-lineinfo",
          "-Xcompiler", "-fPIC,-ffp-contract=off", "-I", os.path.join(ROOT, "include"),
-         "--expt-relaxed-constexpr", "-DRJ_BUILD"]
+         "--expt-relaxed-constexpr", "-DRJ_BUILD"] + os.environ.get("RJ_NVCC_EXTRA", "").split()
 
 
 def _sources():

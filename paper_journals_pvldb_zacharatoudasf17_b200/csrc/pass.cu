@@ -174,6 +174,7 @@ __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a)
 
     if (wid == kWarps) {
         if (lane == 0) produce(a, rg, ring, nstage, ncol);
+        __syncwarp();                                      // reconverge before the CTA barrier
     } else {
         const Consts<NS> k = make_consts<NS>(a);
         const int s_lat = kLatticeBits - a.level;
@@ -235,8 +236,7 @@ __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a)
                 const uint32_t first = (m.sb - m.cb) - woff;    // may wrap: unsigned range test
                 process<SUM, ACC, NS, FP>(a, sh, t, k, w, first, m.se - m.sb, bq, n_pass, n_bnd);
             }
-            __syncwarp();
-            if (lane == 0) mbar_arrive(smem_u32(&rg.empty[st]));
+            stage_release(smem_u32(&rg.empty[st]));
             if (m.flags & 2u) {
                 // ---- last stage of the cell: reduce the tile over the span pieces (S4)
                 consumers_sync();                          // every point of the cell is in the tile

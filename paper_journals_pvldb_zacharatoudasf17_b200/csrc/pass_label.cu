@@ -226,6 +226,7 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
 
     if (wid == kWarps) {
         if (lane == 0) produce(a, rg, ring, nstage, ncol);
+        __syncwarp();                                      // reconverge before the CTA barrier
     } else {
         const Consts<NS> k = make_consts<NS>(a);
         const int s_lat = kLatticeBits - a.level;
@@ -303,8 +304,7 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
                 process_lab<ACC, NS, FP, AF>(a, sh, t, k, w, (m.sb - m.cb) - woff, m.se - m.sb, cy, acc, bq, n_pass,
                                              n_bnd);
             }
-            __syncwarp();
-            if (lane == 0) mbar_arrive(smem_u32(&rg.empty[st]));
+            stage_release(smem_u32(&rg.empty[st]));
             if (++st == nstage) { st = 0; ph ^= 1u; }
         }
         if (ACC) bq_finish<true>(a, sh, bq);

@@ -27,6 +27,26 @@ from datagen import polygons as PG  # noqa: E402
 from paper_journals_pvldb_zacharatoudasf17_b200 import rj  # noqa: E402
 
 
+def device_paths(R, S, P, x, y, cols, chk):
+    """Device-resident inputs: a streamed query over torch device columns and
+    the multi-GPU path's calls (device partials + finalize)."""
+    import torch
+    dx, dy = torch.from_numpy(x).cuda(), torch.from_numpy(y).cuda()
+    dc = [torch.from_numpy(c).cuda() for c in cols]
+    cnt, _ = S.query_stream(dx, dy, dc, W=1024, H=1024, mode="accurate", agg="avg", agg_column=1)
+    chk(cnt, oracle.query(P, x, y, W=1024, H=1024, mode="accurate")[0], "stream-dev")
+    # device partials + finalize (the multi-GPU path's calls)
+    d_cnt = torch.zeros(P.n, dtype=torch.int64, device="cuda")
+    d_sum = torch.zeros(P.n, dtype=torch.float64, device="cuda")
+    d_val = torch.zeros(P.n, dtype=torch.float64, device="cuda")
+    q = rj.make_desc(agg="avg", agg_column=1, W=1024, H=1024, mode="accurate")
+    rj.rj_query_device(R.ctx, q, d_cnt, d_sum)
+    torch.cuda.synchronize()
+    rj.rj_finalize_device(R.ctx, "avg", d_cnt, d_sum, d_val)
+    torch.cuda.synchronize()
+    chk(d_cnt.cpu().numpy().astype(np.uint64), oracle.query(P, x, y, W=1024, H=1024, mode="accurate")[0], "device")
+
+
 def main():
     quick = "--quick" in sys.argv
     n = 20_000 if quick else 60_000
@@ -87,23 +107,14 @@ def main():
         om = "bounded" if mode == "bounded" else "accurate"
         cnt, _ = S.query_stream(x, y, cols, W=777, H=777, mode=mode, agg="sum", agg_column=0)
         chk(cnt, oracle.query(P, x, y, W=777, H=777, mode=om)[0], ("stream", mode))
-    import torch
-    dx, dy = torch.from_numpy(x).cuda(), torch.from_numpy(y).cuda()
-    dc = [torch.from_numpy(c).cuda() for c in cols]
-    cnt, _ = S.query_stream(dx, dy, dc, W=1024, H=1024, mode="accurate", agg="avg", agg_column=1)
-    chk(cnt, oracle.query(P, x, y, W=1024, H=1024, mode="accurate")[0], "stream-dev")
-    # device partials + finalize (the multi-GPU path's calls)
-    d_cnt = torch.zeros(P.n, dtype=torch.int64, device="cuda")
-    d_sum = torch.zeros(P.n, dtype=torch.float64, device="cuda")
-    d_val = torch.zeros(P.n, dtype=torch.float64, device="cuda")
-    q = rj.make_desc(agg="avg", agg_column=1, W=1024, H=1024, mode="accurate")
-    rj.rj_query_device(R.ctx, q, d_cnt, d_sum)
-    torch.cuda.synchronize()
-    rj.rj_finalize_device(R.ctx, "avg", d_cnt, d_sum, d_val)
-    torch.cuda.synchronize()
-    chk(d_cnt.cpu().numpy().astype(np.uint64), oracle.query(P, x, y, W=1024, H=1024, mode="accurate")[0], "device")
+    device_paths(R, S, P, x, y, cols, chk)
     R.close()
     S.close()
+    import gc
+    import torch
+    gc.collect()
+    torch.cuda.synchronize()
+    torch.cuda.empty_cache()                      # memcheck --leak-check: only librj's frees count
     print(f"sanitize driver: {ok} checked queries bit-exact")
 
 

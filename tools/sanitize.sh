@@ -7,7 +7,6 @@ python -c "import __graft_entry__ as g; g.build()" > gpurun_out/build_san.log 2>
 for tool in memcheck synccheck initcheck racecheck; do
   extra=""
   [ $tool = memcheck ] && extra="--leak-check full"
-  [ $tool = initcheck ] && extra="--track-unused-memory no"
   quick=""; [ $tool = racecheck ] && quick="--quick"
   timeout ${SAN_TIMEOUT:-1500} compute-sanitizer --tool $tool $extra --error-exitcode 99 --target-processes all \
      python tools/sanitize.py $quick > gpurun_out/sanitize_${tag}_$tool.txt 2>&1

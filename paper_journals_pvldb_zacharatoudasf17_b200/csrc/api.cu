@@ -963,6 +963,30 @@ rj_status rj_debug_boundary_mask(rj_ctx *c, const rj_query_desc *q, uint32_t *bi
     return RJ_OK;
 }
 
+rj_status rj_debug_boundary_pieces(rj_ctx *c, const rj_query_desc *q, uint32_t *bnd_bits, uint32_t *cover_bits) {
+    if (!bnd_bits || !cover_bits || !q) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL bits or query");
+    rj_query_desc qq = *q;
+    qq.mode = RJ_ACCURATE;
+    Prepared P;
+    rj_status s = prepare(c, &qq, P);
+    if (s != RJ_OK) return s;
+    const size_t n = c->n_poly;
+    const uint64_t wpr = (uint64_t)(P.W + 31) / 32, words = wpr * P.H;
+    Buf d;
+    if (dreserve(c, c->res_cnt, n * 8) || dreserve(c, c->res_sum, n * 8) || dalloc(c, d, std::max<uint64_t>(1, 2 * words) * 4))
+        return set_error(c, RJ_ERR_OOM, "allocation failed");
+    RJ_CUDA(c, cudaMemsetAsync(d.p, 0, 2 * words * 4, c->stream));
+    P.a.bnd_bits = d.as<uint32_t>();
+    P.a.cover_bits = d.as<uint32_t>() + words;
+    P.a.bits_wpr = (uint32_t)wpr;
+    if ((s = run_pass(c, P, c->res_cnt.as<unsigned long long>(), c->res_sum.as<double>())) != RJ_OK) return s;
+    RJ_CUDA(c, cudaMemcpyAsync(bnd_bits, d.p, words * 4, cudaMemcpyDeviceToHost, c->stream));
+    RJ_CUDA(c, cudaMemcpyAsync(cover_bits, d.as<uint32_t>() + words, words * 4, cudaMemcpyDeviceToHost, c->stream));
+    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
+    dfree(c, d);
+    return RJ_OK;
+}
+
 rj_status rj_debug_point_membership(rj_ctx *c, const rj_query_desc *q, uint64_t *bits) {
     if (!bits) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "NULL bits");
     Prepared P;

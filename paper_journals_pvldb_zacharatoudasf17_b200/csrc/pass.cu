@@ -241,6 +241,9 @@ __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a)
                 // ---- last stage of the cell: reduce the tile over the span pieces (S4)
                 consumers_sync();                          // every point of the cell is in the tile
                 if (a.canvas) dump_canvas(a, t, m.cell, s_lat);
+                if (ACC && a.bnd_bits)
+                    dump_bnd(a, t.cnt, t.stride, t.th, t.tw, (uint32_t)pix(cell_y(m.cell) << s_lat, a.H),
+                             (uint32_t)pix(cell_x(m.cell) << s_lat, a.W), kFlag, kFlag);
                 for (uint32_t kk = pb + threadIdx.x; kk < pe; kk += kThreads) {
                     const uint2 pc = (kk == pb + threadIdx.x) ? pc0 : __ldg(&a.pieces[kk]);
                     const uint32_t lr = pc.y & 255u, lo = (pc.y >> 8) & 255u, hi = pc.y >> 16;

@@ -292,6 +292,25 @@ __device__ __forceinline__ void paint_bnd(uint32_t *tile, uint32_t stride, const
     }
 }
 
+// Diagnostic (rj_debug_boundary_pieces): the boundary pixels the kernel
+// painted into this cell's tile -- word & flag_mask == flag -- and every
+// pixel of the tile inside the window, OR-ed into two global bitmasks
+// [H][bits_wpr].  Only when a.bnd_bits is set (never on the query path).
+__device__ __forceinline__ void dump_bnd(const PassArgs &a, const uint32_t *tile, uint32_t stride, uint32_t th,
+                                         uint32_t tw, uint32_t r0, uint32_t c0, uint32_t flag_mask, uint32_t flag) {
+    for (uint32_t i = threadIdx.x; i < th * stride; i += kThreads) {
+        const uint32_t r = i / stride, x = i - r * stride;
+        const uint32_t gr = r0 + r, gc = c0 + x;
+        if (x >= tw || gc < (uint32_t)a.view[0] || gc >= (uint32_t)a.view[2] || gr < (uint32_t)a.view[1] ||
+            gr >= (uint32_t)a.view[3])
+            continue;
+        const uint64_t w = (uint64_t)gr * a.bits_wpr + (gc >> 5);
+        const uint32_t bit = 1u << (gc & 31);
+        atomicOr(&a.cover_bits[w], bit);
+        if ((tile[i] & flag_mask) == flag) atomicOr(&a.bnd_bits[w], bit);
+    }
+}
+
 // ---------------------------------------------------------------- pipeline
 __device__ __forceinline__ void mbar_init(uint32_t bar, uint32_t count) {
     asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" :: "r"(bar), "r"(count) : "memory");

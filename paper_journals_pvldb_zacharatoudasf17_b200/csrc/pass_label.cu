@@ -295,6 +295,7 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
                     }
                 }
                 consumers_sync();
+                if (ACC && a.bnd_bits) dump_bnd(a, lt, t.stride, th, tw, t.r0, t.c0, 0xFFFFFFFFu, kBnd);
             }
             const uint32_t woff = (uint32_t)wid * kWin;
             const uint32_t ncopy = ((m.se + 3u) & ~3u) - m.cb;

@@ -78,6 +78,9 @@ struct PassArgs {
     uint32_t n_stages;            // depth of the shared-memory stage ring
     int32_t index_join;           // every pixel is a boundary pixel, no span pieces (RJ_INDEX_JOIN)
     uint32_t *canvas;             // tile kernel: dump per-pixel filtered counts (W x H) when set
+    uint32_t *bnd_bits;           // diagnostic (accurate): OR the tiles' boundary pixels into [H][bits_wpr]
+    uint32_t *cover_bits;         //   and the pixels the tiles covered (cells holding points, in the window)
+    uint32_t bits_wpr;
     unsigned long long *stats;    // [0] filtered, [1] boundary
     int32_t view[4];              // viewport pixel window (c0, r0, c1, r1), half-open
     uint32_t cwin[4];             // level-L cells meeting it: columns [cwin0, cwin2], rows [cwin1, cwin3]

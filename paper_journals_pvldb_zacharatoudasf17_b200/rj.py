@@ -7,7 +7,8 @@ the calls raise.
 
     rj_create, rj_destroy, rj_load_points, rj_load_polygons, rj_query,
     rj_query_device, rj_query_stream, rj_query_interval, rj_query_interval_ex, rj_query_multi, rj_finalize_device, rj_resolve_canvas(_domain),
-    rj_debug_pixel_spans, rj_debug_boundary_mask, rj_debug_point_membership, rj_debug_point_canvas,
+    rj_debug_pixel_spans, rj_debug_boundary_mask, rj_debug_boundary_pieces, rj_debug_point_membership,
+    rj_debug_point_canvas,
     rj_get_stats, rj_set_option  -- same names as the C ABI.
 
 `RasterJoin` wraps a context with a Pythonic API.
@@ -97,6 +98,7 @@ def lib():
             "rj_resolve_canvas_domain": (i32, [d, d, d, d, qp, ctypes.POINTER(i32), ctypes.POINTER(i32)]),
             "rj_debug_pixel_spans": (i32, [vp, qp, u64, vp, ctypes.POINTER(u64)]),
             "rj_debug_boundary_mask": (i32, [vp, qp, vp]),
+            "rj_debug_boundary_pieces": (i32, [vp, qp, vp, vp]),
             "rj_debug_point_membership": (i32, [vp, qp, vp]),
             "rj_get_stats": (i32, [vp, ctypes.POINTER(rj_stats)]),
             "rj_set_option": (i32, [vp, i32, ctypes.c_int64]),
@@ -117,7 +119,7 @@ def lib():
 
 EXPORTS = ["rj_create", "rj_destroy", "rj_set_allocator", "rj_load_points", "rj_load_polygons", "rj_query",
            "rj_query_device", "rj_query_stream", "rj_query_interval", "rj_query_interval_ex", "rj_query_multi", "rj_debug_point_canvas", "rj_finalize_device", "rj_resolve_canvas", "rj_resolve_canvas_domain",
-           "rj_debug_pixel_spans", "rj_debug_boundary_mask", "rj_debug_point_membership", "rj_get_stats",
+           "rj_debug_pixel_spans", "rj_debug_boundary_mask", "rj_debug_boundary_pieces", "rj_debug_point_membership", "rj_get_stats",
            "rj_set_option", "rj_get_stream", "rj_n_polygons", "rj_n_points", "rj_status_str", "rj_last_error", "rj_version"]
 
 
@@ -303,6 +305,17 @@ def rj_debug_boundary_mask(ctx, desc):
     return bits
 
 
+def rj_debug_boundary_pieces(ctx, desc):
+    """(bnd_bits, cover_bits), each uint32[H, ceil(W/32)]: the boundary pixels
+    the accurate point-pass kernels painted into their tiles, and the pixels
+    those tiles covered."""
+    W, H = rj_resolve_canvas(ctx, desc)
+    bnd = np.zeros((H, (W + 31) // 32), dtype=np.uint32)
+    cov = np.zeros_like(bnd)
+    _check(lib().rj_debug_boundary_pieces(ctx, ctypes.byref(desc), _ptr(bnd), _ptr(cov)), ctx)
+    return bnd, cov
+
+
 def rj_debug_point_membership(ctx, desc, n_input):
     bits = np.zeros(max(1, n_input), dtype=np.uint64)
     _check(lib().rj_debug_point_membership(ctx, ctypes.byref(desc), _ptr(bits)), ctx)
@@ -393,6 +406,9 @@ class RasterJoin:
 
     def boundary_mask(self, **kw):
         return rj_debug_boundary_mask(self.ctx, make_desc(**kw))
+
+    def boundary_pieces(self, **kw):
+        return rj_debug_boundary_pieces(self.ctx, make_desc(**kw))
 
     def membership(self, **kw):
         return rj_debug_point_membership(self.ctx, make_desc(**kw), self.n_input)

@@ -122,6 +122,85 @@ def test_boundary_mask_bitexact(c1, W, H):
     assert np.array_equal(g, o)
 
 
+def _unpack_bits(bits, W):
+    """uint32[H, ceil(W/32)] -> bool[H, W] (bit i % 32 of word i / 32)."""
+    b = np.unpackbits(bits.view(np.uint8), axis=1, bitorder="little")
+    return b[:, :W].astype(bool)
+
+
+@pytest.fixture(scope="module")
+def c1_dense():
+    """C1b polygons with 2M uniform points, so every point cell of the
+    canvases below holds points and the kernels' tiles cover every pixel."""
+    polys = C.polygon_set("c1b")
+    flat = PG.flatten(polys)
+    rng = np.random.default_rng(20171117)
+    x = rng.uniform(0, 1024, 2_000_000)
+    y = rng.uniform(0, 1024, 2_000_000)
+    return flat, x, y, [(np.arange(len(x)) % 5).astype(np.int32)]
+
+
+@pytest.mark.parametrize("W,H", [(1024, 1024), (200, 300), (4096, 4096), (777, 1500)])
+@pytest.mark.parametrize("agg,variant", [("count", -1), ("sum", 0), ("sum", 1)])
+def test_boundary_pieces_bitexact(c1_dense, W, H, agg, variant):
+    """S5 as the hot path uses it: the boundary pixels the accurate kernels
+    paint into their tiles from k_bnd_pieces (pixel-tile kernel for COUNT and
+    RJ_OPT_PASS=1, label kernel for SUM) equal O9's supercover mask
+     on every pixel the tiles cover -- over-marking
+    would be invisible in counts (lemma L4) and only cost time."""
+    flat, x, y, cols = c1_dense
+    R = gpu_ctx(C.C1_BOX, flat, x, y, cols)
+    R.set_option(rjmod.OPT_PASS, variant)
+    P = oracle.Polys(flat, C.C1_BOX)
+    kw = dict(W=W, H=H, agg=agg, agg_column=0 if agg == "sum" else -1)
+    bnd, cov = R.boundary_pieces(**kw)
+    bnd, cov = _unpack_bits(bnd, W), _unpack_bits(cov, W)
+    o = _unpack_bits(oracle.boundary_mask(P, W, H), W)
+    assert np.array_equal(bnd, o & cov)
+    # every point's pixel is covered, and with 2M uniform points every pixel is
+    q = lambda v, n: (np.floor(v * (1 << 20)).astype(np.int64) * n) >> 30
+    assert cov[q(y, H), q(x, W)].all()
+    assert cov.all()
+    assert o.sum() > 0
+    # a window: pieces are clipped to it
+    view = (W // 5, H // 7, W - W // 3, H - H // 9)
+    bnd, cov = R.boundary_pieces(view=view, **kw)
+    bnd, cov = _unpack_bits(bnd, W), _unpack_bits(cov, W)
+    win = np.zeros((H, W), dtype=bool)
+    win[view[1]:view[3], view[0]:view[2]] = True
+    assert np.array_equal(cov, win)
+    assert np.array_equal(bnd, o & win)
+    R.close()
+
+
+@pytest.mark.parametrize("mode", ["bounded", "accurate"])
+@pytest.mark.parametrize("variant", [0, 1])
+@pytest.mark.parametrize("W,H", [(1024, 1024), (333, 517)])
+def test_fused_membership_fingerprint(c1, mode, variant, W, H):
+    """Point membership through the fused kernels themselves (the label and
+    the pixel-tile kernel, RJ_OPT_PASS 0 / 1), not the separate diagnostic
+    kernel: two columns of uniformly random full-range int32 attributes are
+    summed per polygon.  Every partial sum is an integer below 2^53
+    (< 1.1e5 points x 2^31), so fp64 SUM is exact on both sides and must be
+    bit-identical; a polygon whose GPU point set differs from the oracle's
+    in any point changes the sum of a random column except with probability
+    ~2^-32 per column (P:681-726 exact join, P:550-554 bounded)."""
+    flat, x, y, _ = c1
+    rng = np.random.default_rng(1729 + W)
+    fa = rng.integers(-2**31, 2**31, len(x), dtype=np.int64).astype(np.int32)
+    fb = rng.integers(-2**31, 2**31, len(x), dtype=np.int64).astype(np.int32)
+    R = gpu_ctx(C.C1_BOX, flat, x, y, [fa, fb])
+    R.set_option(rjmod.OPT_PASS, variant)
+    P = oracle.Polys(flat, C.C1_BOX)
+    for col in (0, 1):
+        cnt, val = R.query(W=W, H=H, mode=mode, agg="sum", agg_column=col)
+        ocnt, osum, _ = oracle.query(P, x, y, cols=[fa, fb], agg_col=col, W=W, H=H, mode=mode)
+        assert np.array_equal(cnt, ocnt), col
+        assert np.array_equal(val, osum), col
+        assert np.all(np.abs(osum) < 2.0 ** 53)
+    R.close()
+
+
 @pytest.mark.parametrize("mode", ["bounded", "accurate"])
 @pytest.mark.parametrize("W", [1024, 97])
 def test_point_membership_bitexact(c1, mode, W):

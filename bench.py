@@ -8,11 +8,20 @@ rj_query (polygon pass + fused point pass + finalise + D2H of the results)
 over the whole resident point set.
 
     python bench.py [--gpus N] [--steps K] [--warmup W] [--impl reference]
-                    [--points N] [--config C2|C3|C4|C5] [--scaling weak|strong]
+                    [--points N] [--config C2|C3|C4|C5] [--scaling strong|weak]
+                    [--ns-c4] [--backend nccl|gloo --dry-run]
 
-Under torchrun (N > 1) every rank holds its own shard (weak scaling: 1e9
-points per GPU by default) and the per-polygon partials are all-reduced
-with NCCL; the time is the max over ranks.
+N > 1: one process per GPU.  Under torchrun (WORLD_SIZE set) each rank is
+one of them; without it, `--gpus N` re-launches this script under
+torch.distributed.run with N local ranks (and fails loudly if fewer than N
+GPUs are visible).  Default scaling is STRONG: the fixed total of --points
+(1e9) is split into x-strip shards (all_to_all at load time), every rank
+queries its strip's pixel window and the per-polygon partials are combined
+with ONE NCCL all-reduce; the time is the max over ranks.  `--ns-c4` adds the
+north-star record: C4 (twitter-shaped x 3.1k counties, SUM + COUNT,
+eps = 1 km) on 2e9 points in total, strong.  `--backend gloo --dry-run` runs
+the same launch / shard / all-reduce / max-over-ranks logic on CPU with the
+oracle in place of the GPU query (tests/test_bench_launch.py).
 `--impl reference` times the CPU oracle (this tier's reference arm) on a
 bounded sample of the same workload.
 """
@@ -183,11 +192,205 @@ def run_reference(args):
     cb, _ = cpu_baseline(box, polys, recipe, q, target_s=max(2.0, 60.0 / max(1, args.steps + args.warmup)))
     line = {"impl": "reference", "metric": METRIC, "value": cb["value"], "unit": UNIT, "n_gpus": args.gpus,
             "steps": args.steps, "warmup": args.warmup, "ms_per_step": None, "higher_is_better": True,
-            "scaling": "weak", "vs_baseline": None, "dtype": "int64", "data": "synthetic",
+            "scaling": args.scaling, "vs_baseline": None, "dtype": "int64", "data": "synthetic",
             "config": {"workload": desc, "points": args.points, "polygons": polys},
             "cpu_baseline": cb, "e2e": {"value": cb["value"], "unit": UNIT, "h2d_bytes_per_step": 0,
                                         "d2h_bytes_per_step": 0}}
     print(json.dumps(line), flush=True)
+
+
+def launch_ranks(args):
+    """`--gpus N` without torchrun: re-run this script as N local ranks."""
+    import socket
+    if args.backend == "nccl" and args.impl != "reference":
+        import torch
+        have = torch.cuda.device_count()
+        if have < args.gpus:
+            raise SystemExit(f"bench.py --gpus {args.gpus}: only {have} CUDA device(s) visible")
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    port = s.getsockname()[1]
+    s.close()
+    cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", f"--nproc-per-node={args.gpus}",
+           "--master-addr", "127.0.0.1", "--master-port", str(port), os.path.abspath(__file__), *sys.argv[1:]]
+    raise SystemExit(subprocess.call(cmd))
+
+
+def run_dry(args):
+    """CPU stand-in for a multi-rank run (gloo): the launch, the strong-scaling
+    shards, the spatial all_to_all exchange, the all-reduce of the partials and
+    the max-over-ranks timing of the real path, with the oracle computing
+    each rank's partials.  Prints the same JSON line (`dry_run: true`)."""
+    import torch
+    import torch.distributed as dist
+
+    import oracle
+    from paper_journals_pvldb_zacharatoudasf17_b200 import dist as rjdist
+    from paper_journals_pvldb_zacharatoudasf17_b200 import rj
+
+    if args.backend != "gloo":
+        raise SystemExit("--dry-run needs --backend gloo")
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    if world > 1:
+        dist.init_process_group("gloo")
+    box, polys_name, recipe, q, desc = workload(args.config)
+    i0, hi = rjdist.shard_range(args.points, rank, world) if args.scaling == "strong" else \
+        (rank * args.points, (rank + 1) * args.points)
+    n_total = args.points if args.scaling == "strong" else args.points * world
+    x, y, cols = gen_points(recipe, hi - i0, i0)
+    view = None
+    desc_q = rj.make_desc(**q)
+    if world > 1:
+        tx, ty, tc, sp = rjdist.spatial_shard(torch.from_numpy(x), torch.from_numpy(y),
+                                              [torch.from_numpy(c) for c in cols], world, box=box, poly_weight=0.1)
+        x, y, cols = tx.numpy(), ty.numpy(), [c.numpy() for c in tc]
+        view = rjdist.strip_window(box, sp, rank, world, desc_q)
+    P = oracle.Polys(C.array_polys(polys_name), box)
+    W, H = rj.rj_resolve_canvas_domain(box, desc_q)
+    preds = [(c_, op, v) for c_, op, v in q.get("preds", [])]
+    times = []
+    cnt = None
+    for it in range(args.warmup + args.steps):
+        if world > 1:
+            dist.barrier()
+        t0 = time.perf_counter()
+        c_, s_, kept = oracle.query(P, x, y, cols=cols, preds=preds, agg_col=q.get("agg_column", -1), W=W, H=H,
+                                    mode=q["mode"], view=view)
+        tc_, ts_ = torch.from_numpy(c_.astype(np.int64)), torch.from_numpy(s_.copy())
+        nk = torch.tensor([kept], dtype=torch.int64)
+        if world > 1:
+            rjdist.allreduce_partials(tc_, ts_)
+            dist.all_reduce(nk)
+        dt = time.perf_counter() - t0
+        if it >= args.warmup:
+            times.append(dt)
+        cnt = tc_
+    ms = 1e3 * sum(times) / len(times)
+    t = torch.tensor([ms], dtype=torch.float64)
+    if world > 1:
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+    if rank == 0:
+        line = {"metric": METRIC, "value": n_total / (float(t) / 1e3), "unit": UNIT, "n_gpus": world,
+                "steps": args.steps, "warmup": args.warmup, "ms_per_step": float(t), "higher_is_better": True,
+                "scaling": args.scaling, "vs_baseline": None, "dtype": "u32", "data": "synthetic",
+                "dry_run": True, "backend": "gloo",
+                "config": {"workload": desc, "points": n_total, "rank0_view": view},
+                "checks": {"tiling_sum_equals_filtered": int(cnt.sum()) == int(nk), "n_filtered": int(nk)}}
+        print(json.dumps(line), flush=True)
+    if world > 1:
+        dist.destroy_process_group()
+
+
+def ns_c4_record(args, world, rank, local, stream, total=2_000_000_000):
+    """North-star record (BASELINE.json: >= 85 % scaling efficiency at 8 GPUs
+    on a 2B-point query): C4 -- twitter-shaped points x 3.1k counties, SUM(fav)
+    + COUNT, bounded, eps = 1 km -- on `total` points split over the ranks
+    (strong scaling, x-strip shards, one all-reduce).  Returns T_N (max over
+    ranks, CUDA events) and its points/s; efficiency = T_1 / (N * T_N) from
+    the N = 1 run's record."""
+    import gc
+
+    import torch
+    import torch.distributed as dist
+
+    from paper_journals_pvldb_zacharatoudasf17_b200 import dist as rjdist
+    from paper_journals_pvldb_zacharatoudasf17_b200 import rj
+
+    gc.collect()
+    box, polys_name, recipe, q, desc = workload("C4")
+    i0, hi = rjdist.shard_range(total, rank, world)
+    t0 = time.perf_counter()
+    x, y, cols = gen_points(recipe, hi - i0, i0)
+    t_gen = time.perf_counter() - t0
+    view = None
+    desc_q = rj.make_desc(**q)
+    if world > 1:
+        gx, gy, gc_ = torch.from_numpy(x).cuda(), torch.from_numpy(y).cuda(), [torch.from_numpy(c).cuda() for c in cols]
+        del x, y, cols
+        x, y, cols, sp = rjdist.spatial_shard(gx, gy, gc_, world, box=box, poly_weight=0.1)
+        del gx, gy, gc_
+        view = rjdist.strip_window(box, sp, rank, world, desc_q)
+        desc_q = rj.make_desc(**q, view=view)
+    R = rj.RasterJoin(box, device=local, stream=stream.cuda_stream)
+    R.load_points(x, y, cols)
+    R.load_polygons(C.array_polys(polys_name))
+    del x, y, cols
+    n = R.n_poly
+    d_cnt = torch.zeros(n, dtype=torch.int64, device="cuda")
+    d_sum = torch.zeros(n, dtype=torch.float64, device="cuda")
+    d_val = torch.zeros(n, dtype=torch.float64, device="cuda")
+    d_pk = torch.zeros(2 * n, dtype=torch.float64, device="cuda")
+    h_cnt = torch.zeros(n, dtype=torch.int64, pin_memory=True)
+    h_val = torch.zeros(n, dtype=torch.float64, pin_memory=True)
+
+    def step():
+        with torch.cuda.stream(stream):
+            if world > 1:
+                rjdist.query_sharded(R, desc_q, d_cnt, d_sum, d_val, d_packed=d_pk)
+            else:
+                rj.rj_query_device(R.ctx, desc_q, d_cnt, d_sum)
+                rj.rj_finalize_device(R.ctx, desc_q.agg, d_cnt, d_sum, d_val)
+            h_cnt.copy_(d_cnt, non_blocking=True)
+            h_val.copy_(d_val, non_blocking=True)
+        stream.synchronize()
+
+    for _ in range(args.warmup):
+        step()
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    e0.record(stream)
+    for _ in range(args.steps):
+        step()
+    e1.record(stream)
+    torch.cuda.synchronize()
+    ms = e0.elapsed_time(e1) / args.steps
+    st = R.stats()
+    nf = st["n_filtered"]
+    if world > 1:
+        t = torch.tensor([ms], device="cuda", dtype=torch.float64)
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        ms = float(t.item())
+        t = torch.tensor([nf], device="cuda", dtype=torch.int64)
+        dist.all_reduce(t)
+        nf = int(t.item())
+    R.close()
+    return {"workload": desc, "points": total, "n_gpus": world, "scaling": "strong", "ms_per_step": ms,
+            "value": total / (ms / 1e3), "unit": UNIT, "rank0_view": view, "gen_s_rank0": t_gen,
+            "tiling_sum_equals_filtered": int(h_cnt.sum()) == nf,
+            "efficiency": "T_1 / (N * T_N), T_1 = this record at n_gpus = 1"}
+
+
+def host_info():
+    model = None
+    try:
+        for ln in open("/proc/cpuinfo"):
+            if ln.startswith("model name"):
+                model = ln.split(":", 1)[1].strip()
+                break
+    except OSError:
+        pass
+    return model
+
+
+def pinned_h2d_gbs(nbytes=1 << 30):
+    """Measured pinned host -> device copy rate (best of 3, CUDA events): the
+    link peak the e2e number is a fraction of."""
+    import torch
+    h = torch.empty(nbytes, dtype=torch.uint8, pin_memory=True)
+    d = torch.empty(nbytes, dtype=torch.uint8, device="cuda")
+    best = 0.0
+    for _ in range(3):
+        a, b = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+        a.record()
+        d.copy_(h, non_blocking=True)
+        b.record()
+        b.synchronize()
+        best = max(best, nbytes / (a.elapsed_time(b) / 1e3) / 1e9)
+    del h, d
+    return best
 
 
 def main():
@@ -198,7 +401,10 @@ def main():
     ap.add_argument("--impl", default="ours")
     ap.add_argument("--config", default="C2")
     ap.add_argument("--points", type=int, default=1_000_000_000, help="points per GPU (weak) or total (strong)")
-    ap.add_argument("--scaling", default="weak", choices=("weak", "strong"))
+    ap.add_argument("--scaling", default="strong", choices=("weak", "strong"))
+    ap.add_argument("--backend", default="nccl", choices=("nccl", "gloo"))
+    ap.add_argument("--dry-run", action="store_true", help="gloo only: CPU oracle in place of the GPU query")
+    ap.add_argument("--ns-c4", action="store_true", help="add the north-star record: C4 on 2e9 points, strong")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--e2e-steps", type=int, default=2)
     ap.add_argument("--chunk", type=int, default=0, help="points per work item (0 = library default)")
@@ -212,8 +418,12 @@ def main():
     args = ap.parse_args()
     args.warmup = max(3, args.warmup)
 
+    if args.gpus > 1 and "WORLD_SIZE" not in os.environ:
+        return launch_ranks(args)
     if args.impl == "reference":
         return run_reference(args)
+    if args.dry_run:
+        return run_dry(args)
 
     import torch
     import torch.distributed as dist
@@ -290,20 +500,20 @@ def main():
     desc_q = rj.make_desc(**q)
     view = None
     if splitters is not None:
-        Wc, Hc = rj.rj_resolve_canvas(R.ctx, desc_q)
-        view = rjdist.strip_window(box, splitters, rank, world, Wc, Hc)
+        view = rjdist.strip_window(box, splitters, rank, world, desc_q)
         desc_q = rj.make_desc(**q, view=view)
 
     d_cnt = torch.zeros(n_poly, dtype=torch.int64, device="cuda")
     d_sum = torch.zeros(n_poly, dtype=torch.float64, device="cuda")
     d_val = torch.zeros(n_poly, dtype=torch.float64, device="cuda")
+    d_pk = torch.zeros(2 * n_poly, dtype=torch.float64, device="cuda")
     h_cnt = torch.zeros(n_poly, dtype=torch.int64, pin_memory=True)
     h_val = torch.zeros(n_poly, dtype=torch.float64, pin_memory=True)
 
     def step():
         with torch.cuda.stream(stream):
             if world > 1:
-                rjdist.query_sharded(R, desc_q, d_cnt, d_sum, d_val)
+                rjdist.query_sharded(R, desc_q, d_cnt, d_sum, d_val, d_packed=d_pk)
             else:
                 rj.rj_query_device(R.ctx, desc_q, d_cnt, d_sum)
                 rj.rj_finalize_device(R.ctx, desc_q.agg, d_cnt, d_sum, d_val)
@@ -354,6 +564,16 @@ def main():
     ms_step = ms / args.steps
     lat = [a.elapsed_time(b) for a, b in step_ev]        # per-step latency (this rank)
     value = n_total / (ms_step / 1e3)
+
+    # accurate mode: boundary-point fraction f_b and the exact test's work
+    # (the driver of the accurate/bounded gap), read after the
+    # timed region from the last query's boundary queue
+    acc_info = None
+    if st["mode"] != 0:
+        n_pip, n_tests = rj.rj_debug_pip_work(R.ctx)
+        acc_info = {"f_b": st["n_boundary"] / max(1, st["n_filtered"]), "n_boundary": st["n_boundary"],
+                    "pip_points_queued": n_pip, "mean_edge_tests_per_boundary_point": n_tests / max(1, n_pip),
+                    "note": "rank 0's shard" if world > 1 else "whole query"}
 
     # sanity: exact tiling -> every filtered point lands in exactly one polygon
     n_filtered = st["n_filtered"]
@@ -426,6 +646,12 @@ def main():
         cpu = None
         if world == 1 and not args.no_cpu_baseline:
             cpu, _ = cpu_baseline(box, polys_name, recipe, q)
+            cpu["cpu_model"] = host_info()
+        if e2e is not None:
+            link = pinned_h2d_gbs()
+            e2e["link_peak_gbs"] = link
+            e2e["link_frac"] = (e2e["h2d_bytes_per_step"] / world / (e2e["ms_per_step"] / 1e3) / 1e9) / link
+            e2e["link_peak_source"] = "measured: 1 GiB pinned host -> device copy, best of 3, CUDA events"
         line = {
             "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
             "warmup": args.warmup, "ms_per_step": ms_step, "higher_is_better": True, "scaling": args.scaling,
@@ -433,14 +659,14 @@ def main():
             "config": {"workload": desc, "points": n_total, "points_per_gpu": n_local, "polygons": n_poly,
                        "canvas": [st["W"], st["H"]], "parallelism": f"points sharded x{world} ({shard} shards), "
                        "one NCCL allreduce of per-polygon partials" if world > 1 else "1 GPU",
-                       "rank0_view": view, "l2": "inputs (>= 12 GB) larger than L2, no flush needed"},
+                       "rank0_view": view, "l2": "inputs (>= 1 GB per rank) larger than the 126 MB L2, no flush needed"},
             "latency_ms": ms_step,
             "latency_ms_p50": float(np.percentile(lat, 50)), "latency_ms_p90": float(np.percentile(lat, 90)),
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                          "frac": achieved / peak, "traffic": ncu_traffic(args.config),
                          "kernel": "k_point_pass (fused filter+project+tile scatter+span reduce)",
                          "algorithmic_bytes_per_launch": st["stream_bytes"], "kernel_ms": pp,
-                         "peak_source": peak_src},
+                         "peak_source": peak_src, "nominal_peak": 8000.0, "frac_nominal": achieved / 8000.0},
             "stages_ms": {"polygon_pass": statistics.fmean(poly_ms), "point_pass": pp,
                           "point_pass_share": pp / ms_step},
             "clocks": clk.summary(),
@@ -453,10 +679,20 @@ def main():
             "launch": {"cell_level": st["level"], "ring_stages": st["pass_stages"],
                        "ctas_per_sm": st["pass_ctas_per_sm"], "work_items": st["n_items"],
                        "pieces": st["n_pieces"], "crossings": st["n_crossings"]},
-            "host": {"gen_s": t_gen, "load_s": t_load, "exchange_s": t_exchange},
+            "host": {"gen_s": t_gen, "load_s": t_load, "exchange_s": t_exchange, "cpu_model": host_info()},
+            "accurate": acc_info,
         }
+    ns = None
+    if args.ns_c4:
+        R.close()
+        R = None
+        del x, y, cols
+        ns = ns_c4_record(args, world, rank, local, stream)
+    if rank == 0:
+        line["ns_c4_2b"] = ns
         print(json.dumps(line), flush=True)
-    R.close()
+    if R is not None:
+        R.close()
     if world > 1:
         dist.destroy_process_group()
 

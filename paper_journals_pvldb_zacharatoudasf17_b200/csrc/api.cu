@@ -392,6 +392,7 @@ static rj_status run_pass(Ctx *c, Prepared &P, unsigned long long *d_cnt, double
     s = point_pass(c, a, P.sum, P.acc);
     if (s != RJ_OK) return s;
     if (a.bq_cap && (s = pip_queue_pass(c, a, P.sum)) != RJ_OK) return s;
+    c->last_bq = a;
     if (c->timing) RJ_CUDA(c, record_ev(c, 2));
     RJ_CUDA(c, cudaMemcpyAsync(c->h_stats, a.stats, 2 * sizeof(unsigned long long), cudaMemcpyDeviceToHost, c->stream));
     // statistics of this query
@@ -605,6 +606,60 @@ rj_status rj_resolve_canvas_domain(double x0, double y0, double x1, double y1, c
     return s;
 }
 
+// Reading Z20: the pixels [p0, p1) of a side of n pixels that hold every
+// point with wlo <= v < whi.  O1 is monotone (non-decreasing in v: every op
+// is correctly rounded), so such a point has Q(wlo) <= Q(v) <= Q(v'), v' the
+// largest double below whi; bounds beyond the domain clamp to it.
+static rj_status axis_window(double lo, double hi, int n, double wlo, double whi, int32_t &p0, int32_t &p1) {
+    if (std::isnan(wlo) || std::isnan(whi) || !(wlo < whi)) return RJ_ERR_INVALID_ARGUMENT;
+    const int64_t top = (int64_t(1) << kLatticeBits) - 1;
+    auto q = [&](double v) -> int64_t {
+        if (v <= lo) return 0;
+        if (v >= hi) return top;
+        volatile double d = v - lo;                  // O1, each op rounded, no contraction
+        volatile double s = hi - lo;
+        volatile double f = d / s;
+        volatile double g = f * 1073741824.0;
+        return std::min<int64_t>(top, std::max<int64_t>(0, (int64_t)std::floor(g)));
+    };
+    const int64_t a = (q(wlo) * n) >> kLatticeBits;
+    const int64_t b = whi > hi ? n : ((q(std::nextafter(whi, -INFINITY)) * n) >> kLatticeBits) + 1;
+    p0 = (int32_t)a;
+    p1 = (int32_t)std::max<int64_t>(b, a + 1);
+    return RJ_OK;
+}
+
+rj_status rj_resolve_window(double x0, double y0, double x1, double y1, const rj_query_desc *q, double wx0,
+                            double wy0, double wx1, double wy1, int32_t *view) {
+    if (!q || !view) return RJ_ERR_INVALID_ARGUMENT;
+    int W, H;
+    rj_status s = resolve(x0, y0, x1, y1, q, &W, &H);
+    if (s != RJ_OK) return s;
+    int32_t v[4];
+    if ((s = axis_window(x0, x1, W, wx0, wx1, v[0], v[2])) != RJ_OK) return s;
+    if ((s = axis_window(y0, y1, H, wy0, wy1, v[1], v[3])) != RJ_OK) return s;
+    std::copy(v, v + 4, view);
+    return RJ_OK;
+}
+
+rj_status rj_resolve_lod(double x0, double y0, double x1, double y1, double wx0, double wy0, double wx1,
+                         double wy1, int32_t w, int32_t h, int32_t *W, int32_t *H, int32_t *view) {
+    if (!W || !H || !view || w < 1 || h < 1 || !(wx1 > wx0) || !(wy1 > wy0)) return RJ_ERR_INVALID_ARGUMENT;
+    // the finer canvas over the whole domain whose pixels are as large as
+    // w x h pixels over the world rectangle
+    const double fw = std::nearbyint((double)w * (x1 - x0) / (wx1 - wx0));
+    const double fh = std::nearbyint((double)h * (y1 - y0) / (wy1 - wy0));
+    if (!(fw >= 1.0 && fh >= 1.0)) return RJ_ERR_RESOLUTION;
+    rj_query_desc q{};
+    q.canvas_w = (int32_t)std::min(fw, (double)RJ_MAX_CANVAS);
+    q.canvas_h = (int32_t)std::min(fh, (double)RJ_MAX_CANVAS);
+    rj_status s = rj_resolve_window(x0, y0, x1, y1, &q, wx0, wy0, wx1, wy1, view);
+    if (s != RJ_OK) return s;
+    *W = q.canvas_w;
+    *H = q.canvas_h;
+    return RJ_OK;
+}
+
 rj_status rj_resolve_canvas(const rj_ctx *ctx, const rj_query_desc *q, int32_t *W, int32_t *H) {
     if (!ctx) return RJ_ERR_INVALID_ARGUMENT;
     return rj_resolve_canvas_domain(ctx->x0, ctx->y0, ctx->x1, ctx->y1, q, W, H);
@@ -757,7 +812,9 @@ rj_status rj_query_device(rj_ctx *c, const rj_query_desc *q, uint64_t *d_count, 
         Prepared P;
         rj_status s2 = prepare(c, q, P);
         if (s2 != RJ_OK) return s2;
-        return run_pass(c, P, reinterpret_cast<unsigned long long *>(d_count), d_sum);
+        if ((s2 = run_pass(c, P, reinterpret_cast<unsigned long long *>(d_count), d_sum)) != RJ_OK) return s2;
+        if (c->timing) RJ_CUDA(c, record_ev(c, 3));      // ms_total of this query (rj_get_stats)
+        return RJ_OK;
     });
 }
 
@@ -767,6 +824,22 @@ rj_status rj_finalize_device(rj_ctx *c, int32_t agg, uint32_t n, const uint64_t 
     if (agg < RJ_COUNT || agg > RJ_AVG) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad agg");
     if (c->poisoned) return set_error(c, RJ_ERR_CUDA, c->err);
     RJ_CUDA(c, launch_finalize(c, agg, n, reinterpret_cast<const unsigned long long *>(d_count), d_sum, d_value));
+    return RJ_OK;
+}
+
+rj_status rj_pack_partials(rj_ctx *c, uint32_t n, const uint64_t *d_count, const double *d_sum, double *d_packed) {
+    if (!c || !d_count || !d_packed) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad pack arguments");
+    if (c->poisoned) return set_error(c, RJ_ERR_CUDA, c->err);
+    RJ_CUDA(c, launch_pack(c, n, reinterpret_cast<const unsigned long long *>(d_count), d_sum, d_packed));
+    return RJ_OK;
+}
+
+rj_status rj_finalize_packed(rj_ctx *c, int32_t agg, uint32_t n, const double *d_packed, uint64_t *d_count,
+                             double *d_value) {
+    if (!c || !d_packed || !d_count || !d_value) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad finalize arguments");
+    if (agg < RJ_COUNT || agg > RJ_AVG) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "bad agg");
+    if (c->poisoned) return set_error(c, RJ_ERR_CUDA, c->err);
+    RJ_CUDA(c, launch_finalize_packed(c, agg, n, d_packed, reinterpret_cast<unsigned long long *>(d_count), d_value));
     return RJ_OK;
 }
 
@@ -985,6 +1058,12 @@ rj_status rj_debug_boundary_pieces(rj_ctx *c, const rj_query_desc *q, uint32_t *
     RJ_CUDA(c, cudaStreamSynchronize(c->stream));
     dfree(c, d);
     return RJ_OK;
+}
+
+rj_status rj_debug_pip_work(rj_ctx *c, uint64_t *n_points, uint64_t *n_edge_tests) {
+    if (!c || !n_points || !n_edge_tests) return RJ_ERR_INVALID_ARGUMENT;
+    if (c->poisoned) return set_error(c, RJ_ERR_CUDA, c->err);
+    return pip_work(c, n_points, n_edge_tests);
 }
 
 rj_status rj_debug_point_membership(rj_ctx *c, const rj_query_desc *q, uint64_t *bits) {

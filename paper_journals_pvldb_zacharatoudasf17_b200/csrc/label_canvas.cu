@@ -45,14 +45,15 @@ inline unsigned blocks_for(uint64_t n, int t) { return (unsigned)std::max<uint64
 // (c0 + x, r0 + r) of the W x H canvas is lab[r * vw + x], r < vh, x < vw.
 
 // lab = LAB_BND on boundary pixels (or everywhere: index join), else LAB_NONE.
-__global__ void k_lab_init(uint32_t *__restrict__ lab, uint32_t vw, uint32_t c0, uint32_t r0,
+__global__ void k_lab_init(uint32_t *__restrict__ lab, uint32_t vw, uint32_t vh, uint32_t c0, uint32_t r0,
                            const uint32_t *__restrict__ mask, uint32_t wpr, int all_bnd) {
-    const uint64_t r = blockIdx.y;
-    for (uint32_t x = blockIdx.x * blockDim.x + threadIdx.x; x < vw; x += gridDim.x * blockDim.x) {
-        const uint32_t px = c0 + x;
-        const bool b = all_bnd || (mask && ((mask[(r0 + r) * wpr + (px >> 5)] >> (px & 31)) & 1u));
-        lab[r * vw + x] = b ? kLabBnd : kLabNone;
-    }
+    // rows stride over gridDim.y (<= 65535: a window may be 131072 rows high)
+    for (uint64_t r = blockIdx.y; r < vh; r += gridDim.y)
+        for (uint32_t x = blockIdx.x * blockDim.x + threadIdx.x; x < vw; x += gridDim.x * blockDim.x) {
+            const uint32_t px = c0 + x;
+            const bool b = all_bnd || (mask && ((mask[(r0 + r) * wpr + (px >> 5)] >> (px & 31)) & 1u));
+            lab[r * vw + x] = b ? kLabBnd : kLabNone;
+        }
 }
 
 // One warp per pixel span (polygon, row, lo, hi) -- clipped to the window by
@@ -374,7 +375,7 @@ rj_status label_query_impl(Ctx *c, const Filter &f, const AggPlan &ap, int W, in
         dreserve(c, roff, (uint64_t)(vh + 1) * 4) || dreserve(c, rcur, (uint64_t)(vh + 1) * 4) ||
         dreserve(c, rsp, (S + 1) * 16) || dreserve(c, sts, 64))
         return set_error(c, RJ_ERR_OOM, "label-canvas workspace allocation failed");
-    k_lab_init<<<dim3(blocks_for(vw, 256), vh), 256, 0, st>>>(lab.as<uint32_t>(), vw, vc0, vr0,
+    k_lab_init<<<dim3(blocks_for(vw, 256), std::min<uint32_t>(vh, 65535u)), 256, 0, st>>>(lab.as<uint32_t>(), vw, vh, vc0, vr0,
                                                              acc && !index ? pp.mask : nullptr, pp.mask_wpr, index);
     RJ_LAUNCHED(c);
     RJ_CUDA(c, cudaMemsetAsync(rcnt.p, 0, (uint64_t)(vh + 1) * 4, st));

@@ -16,6 +16,28 @@ __global__ void k_finalize(int agg, uint32_t n, const unsigned long long *__rest
     else val[i] = (double)cnt[i];
 }
 
+// Multi-GPU combine (S8): counts and sums in one binary64 buffer, so one
+// all-reduce combines both (counts are exact in binary64 below 2^53).
+__global__ void k_pack(uint32_t n, const unsigned long long *__restrict__ cnt, const double *__restrict__ sum,
+                       double *__restrict__ out) {
+    const uint32_t i = blockIdx.x * blockDim.x + threadIdx.x;
+    if (i >= n) return;
+    out[i] = (double)cnt[i];
+    out[n + i] = sum ? sum[i] : 0.0;
+}
+
+__global__ void k_finalize_packed(int agg, uint32_t n, const double *__restrict__ in,
+                                  unsigned long long *__restrict__ cnt, double *__restrict__ val) {
+    const uint32_t i = blockIdx.x * blockDim.x + threadIdx.x;
+    if (i >= n) return;
+    const unsigned long long c = (unsigned long long)in[i];
+    const double s = in[n + i];
+    cnt[i] = c;
+    if (agg == RJ_AVG) val[i] = c ? __ddiv_rn(s, (double)c) : __longlong_as_double(0x7ff8000000000000ll);
+    else if (agg == RJ_SUM) val[i] = s;
+    else val[i] = (double)c;
+}
+
 __device__ __forceinline__ bool filter_point(const PassArgs &a, uint64_t i) {
     const Filter &f = a.f;
     if (f.never) return false;
@@ -90,6 +112,21 @@ cudaError_t launch_finalize(Ctx *c, int agg, uint32_t n, const unsigned long lon
                             double *val) {
     if (!n) return cudaSuccess;
     k_finalize<<<blocks_for(n, 256), 256, 0, c->stream>>>(agg, n, cnt, sum, val);
+    RJ_LAUNCHED(c);
+    return cudaGetLastError();
+}
+
+cudaError_t launch_pack(Ctx *c, uint32_t n, const unsigned long long *cnt, const double *sum, double *out) {
+    if (!n) return cudaSuccess;
+    k_pack<<<blocks_for(n, 256), 256, 0, c->stream>>>(n, cnt, sum, out);
+    RJ_LAUNCHED(c);
+    return cudaGetLastError();
+}
+
+cudaError_t launch_finalize_packed(Ctx *c, int agg, uint32_t n, const double *in, unsigned long long *cnt,
+                                   double *val) {
+    if (!n) return cudaSuccess;
+    k_finalize_packed<<<blocks_for(n, 256), 256, 0, c->stream>>>(agg, n, in, cnt, val);
     RJ_LAUNCHED(c);
     return cudaGetLastError();
 }

@@ -334,6 +334,29 @@ __global__ void __launch_bounds__(256) k_pip_queue(const __grid_constant__ PassA
         }
 }
 
+// Diagnostic: the grid entries (edge tests) the exact test of every queued
+// boundary point walks -- the cell's list in pip.cuh.
+__global__ void k_pip_work(const __grid_constant__ PassArgs a, unsigned long long *out) {
+    const uint32_t n = min(*a.bq_count, *a.bq_valid);
+    unsigned long long pts = 0, tests = 0;
+    for (uint32_t i = blockIdx.x * blockDim.x + threadIdx.x; i < n; i += gridDim.x * blockDim.x) {
+        const uint32_t x = a.bq_x[i];
+        if (x == kDone) continue;
+        const uint32_t y = a.bq_y[i];
+        const uint32_t cell = (y >> kGridShift) * kGrid + (x >> kGridShift);
+        ++pts;
+        tests += a.grid_off[cell + 1] - a.grid_off[cell];
+    }
+    for (int o = 16; o; o >>= 1) {
+        pts += __shfl_xor_sync(kFull, pts, o);
+        tests += __shfl_xor_sync(kFull, tests, o);
+    }
+    if ((threadIdx.x & 31) == 0 && pts) {
+        atomicAdd(&out[0], pts);
+        atomicAdd(&out[1], tests);
+    }
+}
+
 template <bool SUM, bool ACC, bool FP>
 void *select_ns(int ns) {
     switch (ns) {
@@ -429,6 +452,23 @@ rj_status pip_queue_pass(Ctx *c, const PassArgs &a_in, bool sum) {
     void *args[] = {(void *)&a};
     RJ_CUDA(c, cudaLaunchKernel(k, dim3(grid), dim3(256), args, smem, c->stream));
     RJ_LAUNCHED(c);
+    return RJ_OK;
+}
+
+rj_status pip_work(Ctx *c, uint64_t *n_points, uint64_t *n_edge_tests) {
+    *n_points = *n_edge_tests = 0;
+    if (!c->last_bq.bq_cap) return RJ_OK;
+    Buf d;
+    if (dalloc(c, d, 16)) return set_error(c, RJ_ERR_OOM, "allocation failed");
+    RJ_CUDA(c, cudaMemsetAsync(d.p, 0, 16, c->stream));
+    k_pip_work<<<c->num_sms * 4, 256, 0, c->stream>>>(c->last_bq, reinterpret_cast<unsigned long long *>(d.p));
+    RJ_CUDA(c, cudaGetLastError());
+    unsigned long long h[2];
+    RJ_CUDA(c, cudaMemcpyAsync(h, d.p, 16, cudaMemcpyDeviceToHost, c->stream));
+    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
+    dfree(c, d);
+    *n_points = h[0];
+    *n_edge_tests = h[1];
     return RJ_OK;
 }
 

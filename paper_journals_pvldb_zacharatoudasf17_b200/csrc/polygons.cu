@@ -43,27 +43,65 @@ __device__ __forceinline__ uint32_t upper_bound_u32(const uint32_t *a, uint32_t 
 }
 
 // ------------------------------------------------------------- edge grid (S6)
+// Cell (gr, gc) lists edge e iff e is not horizontal, gr is one of the grid
+// rows its y-extent overlaps, and gc lies between its polygon's MBR left
+// side and the edge (the cells where e can toggle the half-open ray).  Each
+// edge therefore covers one column run per grid row; the work is cut into
+// items of (edge, row, 32-column chunk), so a long edge of a wide polygon is
+// spread over many threads instead of one thread walking rows x columns.
+constexpr int kGridChunk = 32;
+
+struct GridRun {
+    int gr0, gr1, gc0, gc1;   // rows [gr0, gr1], columns [gc0, gc1] (empty: gr1 < gr0)
+};
+
+__device__ __forceinline__ GridRun grid_run(const int4 E, const int4 M) {
+    GridRun g{0, -1, 0, -1};
+    if (E.y == E.w || M.z - 1 < M.x) return g;           // horizontal: never toggles; empty MBR
+    const int ymin = min(E.y, E.w), ymax = max(E.y, E.w);
+    g.gr0 = ymin >> kGridShift;
+    g.gr1 = (ymax - 1) >> kGridShift;
+    g.gc0 = M.x >> kGridShift;
+    g.gc1 = min(min((M.z - 1) >> kGridShift, (max(E.x, E.z) - 1) >> kGridShift), kGrid - 1);
+    if (g.gc1 < g.gc0) g.gr1 = g.gr0 - 1;
+    return g;
+}
+
+// items[e] = rows x chunks of edge e; *total += its entries (64-bit: the u32
+// CSR offsets overflow silently otherwise)
+__global__ void k_grid_items(const int4 *__restrict__ edges, const uint32_t *__restrict__ edge_poly,
+                             const int4 *__restrict__ mbr, uint32_t n_edges, uint32_t *__restrict__ items,
+                             unsigned long long *__restrict__ total) {
+    const uint32_t e = blockIdx.x * blockDim.x + threadIdx.x;
+    unsigned long long ent = 0;
+    if (e < n_edges) {
+        const GridRun g = grid_run(edges[e], mbr[edge_poly[e]]);
+        const uint32_t rows = (uint32_t)max(0, g.gr1 - g.gr0 + 1), cols = (uint32_t)max(0, g.gc1 - g.gc0 + 1);
+        items[e] = rows * ((cols + kGridChunk - 1) / kGridChunk);
+        ent = (unsigned long long)rows * cols;
+    }
+    for (int o = 16; o; o >>= 1) ent += __shfl_xor_sync(0xFFFFFFFFu, ent, o);
+    if ((threadIdx.x & 31) == 0 && ent) atomicAdd(total, ent);
+}
+
 template <bool FILL>
 __global__ void k_grid_edges(const int4 *__restrict__ edges, const uint32_t *__restrict__ edge_poly,
-                             const int4 *__restrict__ mbr, uint32_t n_edges, uint32_t *__restrict__ cnt,
-                             const uint32_t *__restrict__ off, uint32_t *__restrict__ cursor,
-                             uint32_t *__restrict__ ent) {
-    const uint32_t e = blockIdx.x * blockDim.x + threadIdx.x;
-    if (e >= n_edges) return;
-    const int4 E = edges[e];
-    if (E.y == E.w) return;                               // horizontal: never toggles
-    const int4 M = mbr[edge_poly[e]];
-    if (M.z - 1 < M.x) return;                            // empty half-open MBR
-    const int ymin = min(E.y, E.w), ymax = max(E.y, E.w);
-    const int gr0 = ymin >> kGridShift, gr1 = (ymax - 1) >> kGridShift;
-    const int gc0 = M.x >> kGridShift;
-    const int gc1 = min(min((M.z - 1) >> kGridShift, (max(E.x, E.z) - 1) >> kGridShift), kGrid - 1);
-    for (int gr = gr0; gr <= gr1; ++gr)
-        for (int gc = gc0; gc <= gc1; ++gc) {
+                             const int4 *__restrict__ mbr, uint32_t n_edges, const uint32_t *__restrict__ item_off,
+                             uint32_t *__restrict__ cnt, const uint32_t *__restrict__ off,
+                             uint32_t *__restrict__ cursor, uint32_t *__restrict__ ent) {
+    const uint32_t n_items = item_off[n_edges];
+    for (uint32_t j = blockIdx.x * blockDim.x + threadIdx.x; j < n_items; j += gridDim.x * blockDim.x) {
+        const uint32_t e = upper_bound_u32(item_off, n_edges + 1, j) - 1;
+        const GridRun g = grid_run(edges[e], mbr[edge_poly[e]]);
+        const uint32_t nch = (uint32_t)(g.gc1 - g.gc0 + kGridChunk) / kGridChunk, k = j - item_off[e];
+        const int gr = g.gr0 + (int)(k / nch);
+        const int c0 = g.gc0 + (int)(k % nch) * kGridChunk, c1 = min(g.gc1, c0 + kGridChunk - 1);
+        for (int gc = c0; gc <= c1; ++gc) {
             const uint32_t cell = (uint32_t)gr * kGrid + gc;
             if (FILL) ent[off[cell] + atomicAdd(&cursor[cell], 1u)] = e;
             else atomicAdd(&cnt[cell], 1u);
         }
+    }
 }
 
 // Entries inlined for the accurate-mode test: the edge's endpoints and its
@@ -79,15 +117,34 @@ __global__ void k_grid_inline(const uint32_t *__restrict__ ent, uint32_t n, cons
     gpoly[i] = edge_poly[e];
 }
 
-__global__ void k_grid_sort(const uint32_t *__restrict__ off, uint32_t *__restrict__ ent) {
-    const uint32_t c = blockIdx.x * blockDim.x + threadIdx.x;
-    if (c >= (uint32_t)kGrid * kGrid) return;
-    const uint32_t b = off[c], e = off[c + 1];
-    for (uint32_t i = b + 1; i < e; ++i) {               // insertion sort: edge ids group by polygon
-        const uint32_t v = ent[i];
-        uint32_t j = i;
-        while (j > b && ent[j - 1] > v) { ent[j] = ent[j - 1]; --j; }
-        ent[j] = v;
+// Sort each cell's entries by edge id (so they group by polygon, which the
+// walk in pip.cuh relies on): one warp per cell -- a register bitonic sort
+// for <= 32 entries, else every entry's rank (distinct ids) into tmp and back.
+__global__ void k_grid_sort(const uint32_t *__restrict__ off, uint32_t *__restrict__ ent, uint32_t *__restrict__ tmp) {
+    const uint32_t lane = threadIdx.x & 31;
+    const uint32_t nw = (gridDim.x * blockDim.x) >> 5;
+    for (uint32_t c = (blockIdx.x * blockDim.x + threadIdx.x) >> 5; c < (uint32_t)kGrid * kGrid; c += nw) {
+        const uint32_t b = off[c], e = off[c + 1], k = e - b;
+        if (k < 2) continue;
+        if (k <= 32) {
+            uint32_t v = lane < k ? ent[b + lane] : 0xFFFFFFFFu;
+            for (uint32_t size = 2; size <= 32; size <<= 1)
+                for (uint32_t st = size >> 1; st; st >>= 1) {
+                    const uint32_t o = __shfl_xor_sync(0xFFFFFFFFu, v, st);
+                    const bool up = (lane & size) == 0, lower = (lane & st) == 0;
+                    v = (lower == up) ? min(v, o) : max(v, o);
+                }
+            if (lane < k) ent[b + lane] = v;
+        } else {
+            for (uint32_t i = b + lane; i < e; i += 32) {
+                const uint32_t v = ent[i];
+                uint32_t r = 0;
+                for (uint32_t j = b; j < e; ++j) r += ent[j] < v ? 1u : 0u;
+                tmp[b + r] = v;
+            }
+            __syncwarp();
+            for (uint32_t i = b + lane; i < e; i += 32) ent[i] = tmp[i];
+        }
     }
 }
 
@@ -434,32 +491,58 @@ rj_status load_polygons_impl(Ctx *c, uint32_t n_poly, const uint32_t *pro, const
     RJ_CUDA(c, cudaMemcpyAsync(c->poly_edge_off.p, peoff.data(), (n_poly + 1) * 4, cudaMemcpyHostToDevice, c->stream));
     RJ_CUDA(c, cudaMemcpyAsync(c->mbr.p, mbr.data(), n_poly * sizeof(int4), cudaMemcpyHostToDevice, c->stream));
 
-    // S6 edge grid, two passes + per-cell sort
+    // S6 edge grid: items per edge, count pass, offsets, fill pass, per-cell sort
     const uint64_t ncell = (uint64_t)kGrid * kGrid;
-    Buf cnt, cur;
-    if (dalloc(c, cnt, ncell * 4) || dalloc(c, cur, ncell * 4) || dalloc(c, c->grid_off, (ncell + 1) * 4))
+    Buf cnt, cur, items, item_off, tot;
+    if (dalloc(c, cnt, ncell * 4) || dalloc(c, cur, ncell * 4) || dalloc(c, c->grid_off, (ncell + 1) * 4) ||
+        dalloc(c, items, (uint64_t)(ne + 1) * 4) || dalloc(c, item_off, (uint64_t)(ne + 1) * 4) || dalloc(c, tot, 8))
         return set_error(c, RJ_ERR_OOM, "edge grid allocation failed");
     RJ_CUDA(c, cudaMemsetAsync(cnt.p, 0, ncell * 4, c->stream));
     RJ_CUDA(c, cudaMemsetAsync(cur.p, 0, ncell * 4, c->stream));
-    k_grid_edges<false><<<blocks_for(ne, 128), 128, 0, c->stream>>>(
-        c->edges.as<int4>(), c->edge_poly.as<uint32_t>(), c->mbr.as<int4>(), ne, cnt.as<uint32_t>(), nullptr,
-        nullptr, nullptr);
+    RJ_CUDA(c, cudaMemsetAsync(tot.p, 0, 8, c->stream));
+    k_grid_items<<<blocks_for(ne, 256), 256, 0, c->stream>>>(c->edges.as<int4>(), c->edge_poly.as<uint32_t>(),
+                                                             c->mbr.as<int4>(), ne, items.as<uint32_t>(),
+                                                             reinterpret_cast<unsigned long long *>(tot.p));
+    RJ_LAUNCHED(c);
+    RJ_CUDA(c, cudaGetLastError());
+    RJ_CUDA(c, scan_u32(c, items.as<uint32_t>(), item_off.as<uint32_t>(), ne, kWsScan));
+    unsigned long long n_ent64 = 0;
+    RJ_CUDA(c, cudaMemcpyAsync(&n_ent64, tot.p, 8, cudaMemcpyDeviceToHost, c->stream));
+    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
+    // the item count is at most the entry count, so one check covers both u32 offsets
+    if (n_ent64 > 0xFFFFFFFFull) {
+        dfree(c, cnt); dfree(c, cur); dfree(c, items); dfree(c, item_off); dfree(c, tot);
+        return set_error(c, RJ_ERR_CAPACITY, "edge grid: more than 2^32 - 1 (cell, edge) entries");
+    }
+    const uint32_t n_ent = (uint32_t)n_ent64;
+    const unsigned gi = (unsigned)std::max<uint64_t>(1, std::min<uint64_t>(blocks_for(n_ent, 256), c->num_sms * 16ull));
+    k_grid_edges<false><<<gi, 256, 0, c->stream>>>(c->edges.as<int4>(), c->edge_poly.as<uint32_t>(),
+                                                   c->mbr.as<int4>(), ne, item_off.as<uint32_t>(),
+                                                   cnt.as<uint32_t>(), nullptr, nullptr, nullptr);
     RJ_LAUNCHED(c);
     RJ_CUDA(c, cudaGetLastError());
     RJ_CUDA(c, scan_u32(c, cnt.as<uint32_t>(), c->grid_off.as<uint32_t>(), ncell, kWsScan));
-    uint32_t n_ent = 0;
-    RJ_CUDA(c, cudaMemcpyAsync(&n_ent, c->grid_off.as<uint32_t>() + ncell, 4, cudaMemcpyDeviceToHost, c->stream));
-    RJ_CUDA(c, cudaStreamSynchronize(c->stream));
     if (dalloc(c, c->grid_ent, std::max<uint64_t>(1, n_ent) * 4))
         return set_error(c, RJ_ERR_OOM, "edge grid allocation failed");
-    k_grid_edges<true><<<blocks_for(ne, 128), 128, 0, c->stream>>>(
-        c->edges.as<int4>(), c->edge_poly.as<uint32_t>(), c->mbr.as<int4>(), ne, nullptr,
-        c->grid_off.as<uint32_t>(), cur.as<uint32_t>(), c->grid_ent.as<uint32_t>());
+    k_grid_edges<true><<<gi, 256, 0, c->stream>>>(c->edges.as<int4>(), c->edge_poly.as<uint32_t>(),
+                                                  c->mbr.as<int4>(), ne, item_off.as<uint32_t>(), nullptr,
+                                                  c->grid_off.as<uint32_t>(), cur.as<uint32_t>(),
+                                                  c->grid_ent.as<uint32_t>());
     RJ_LAUNCHED(c);
     RJ_CUDA(c, cudaGetLastError());
-    k_grid_sort<<<blocks_for(ncell, 256), 256, 0, c->stream>>>(c->grid_off.as<uint32_t>(), c->grid_ent.as<uint32_t>());
-    RJ_LAUNCHED(c);
-    RJ_CUDA(c, cudaGetLastError());
+    {
+        Buf tmp;
+        if (dalloc(c, tmp, std::max<uint64_t>(1, n_ent) * 4)) return set_error(c, RJ_ERR_OOM, "edge grid allocation failed");
+        k_grid_sort<<<(unsigned)(c->num_sms * 16), 256, 0, c->stream>>>(c->grid_off.as<uint32_t>(),
+                                                                     c->grid_ent.as<uint32_t>(), tmp.as<uint32_t>());
+        RJ_LAUNCHED(c);
+        RJ_CUDA(c, cudaGetLastError());
+        RJ_CUDA(c, cudaStreamSynchronize(c->stream));
+        dfree(c, tmp);
+    }
+    dfree(c, items);
+    dfree(c, item_off);
+    dfree(c, tot);
     dfree(c, c->grid_edge);
     dfree(c, c->grid_poly);
     if (dalloc(c, c->grid_edge, std::max<uint64_t>(1, n_ent) * sizeof(int4)) ||

@@ -167,11 +167,12 @@ struct Ctx {
     cudaEvent_t ev[6] = {};
     uint32_t launches = 0;
     int last_stages = 0, last_ctas_per_sm = 0;   // point-pass launch shape of the last query
+    PassArgs last_bq{};                           // last accurate query with a global boundary queue (bq_cap > 0)
     int pass_variant = -1;                        // RJ_OPT_PASS: -1 auto, 0 label, 1 pixel tile
     int force_stages = 0;                         // RJ_OPT_STAGES: 0 = automatic, else 2..4
     int tile_side = 64;                           // RJ_OPT_TILE_SIDE: target point-cell side in pixels
 
-    // streamed query (stream.cu)
+    // streamed query (label_canvas.cu, rj_query_stream)
     int64_t stream_batch = int64_t(1) << 24;      // RJ_OPT_STREAM_BATCH: points per batch
     cudaStream_t copy_stream = nullptr;           // H2D copies of the batches
     cudaEvent_t sev[5] = {};                      // copied[2], consumed[2], start
@@ -181,7 +182,7 @@ struct Ctx {
 
 // workspace slot map (Ctx::ws)
 enum : int {
-    kWsSortCounts = 0, kWsSortBuf = 1,      // 1..12 double buffers of the radix sort
+    kWsSortCounts = 0,                      // radix-sort digit counts (load_points.cu)
     kWsEdgeRows = 14, kWsEdgeOff, kWsPolyRows, kWsPolyRowOff, kWsCrossPR, kWsCrossT,
     kWsPRCount, kWsPROff, kWsPRCursor, kWsTvals, kWsSpanCount, kWsSpanOff, kWsSpans,
     kWsPieceCount, kWsPieceOff, kWsPieceCursor, kWsPieces, kWsMask, kWsBandCount, kWsBandOff,
@@ -190,7 +191,7 @@ enum : int {
     kWsCanvas, kWsBRowCount, kWsBRowOff, kWsBktCount, kWsBktOff, kWsBktCursor, kWsBktRanges,   // intervals
     kWsBQx, kWsBQy, kWsBQa,                 // accurate mode: global boundary-point queue
     kWsBPCount, kWsBPOff, kWsBPCursor, kWsBPieces,   // accurate mode: boundary pieces per point cell
-    kWsScan = 72,                           // 72..95 recursive scan temporaries
+    kWsScan = 72,                           // scan_u32's look-back status words (scan.cu, one slot)
 };
 
 // allocation helpers (ctx allocator if set)
@@ -277,12 +278,18 @@ rj_status ring_sigma_impl(Ctx *c, uint32_t n_poly, uint32_t n_ring);
 rj_status point_pass(Ctx *c, const PassArgs &a, bool sum, bool accurate);
 // accurate mode: exact PIP of the queued boundary points (after point_pass)
 rj_status pip_queue_pass(Ctx *c, const PassArgs &a, bool sum);
+// diagnostic: points in the last query's boundary queue and the edge-grid
+// entries their exact tests walk (SURVEY.md 8(a) S7 note)
+rj_status pip_work(Ctx *c, uint64_t *n_points, uint64_t *n_edge_tests);
 size_t point_pass_smem(const Ctx *c, const PassArgs &a, bool sum, bool accurate);
 int point_pass_stages(int n_slots);
 
 // misc.cu
 cudaError_t launch_finalize(Ctx *c, int agg, uint32_t n, const unsigned long long *cnt,
                             const double *sum, double *val);
+cudaError_t launch_pack(Ctx *c, uint32_t n, const unsigned long long *cnt, const double *sum, double *out);
+cudaError_t launch_finalize_packed(Ctx *c, int agg, uint32_t n, const double *in, unsigned long long *cnt,
+                                   double *val);
 cudaError_t launch_membership(Ctx *c, const PassArgs &a, bool accurate, unsigned long long *bits);
 
 rj_status set_error(Ctx *c, rj_status s, const std::string &msg);

@@ -40,22 +40,41 @@ def allreduce_partials(count: torch.Tensor, total: torch.Tensor | None = None, g
 
 
 def query_sharded(R: "rj.RasterJoin", desc, d_count: torch.Tensor, d_sum: torch.Tensor, d_value: torch.Tensor,
-                  group=None):
-    """Partials on this rank's shard -> all-reduce -> finalise (all on device).
+                  group=None, d_packed: torch.Tensor | None = None):
+    """Partials on this rank's shard -> ONE all-reduce -> finalise (all on device).
 
-    The query and the finalisation run on the context's stream (rj_get_stream),
-    the collective on torch's current stream; each waits for the other, so any
-    stream choice at rj_create is safe."""
-    rj.rj_query_device(R.ctx, desc, d_count, d_sum)
+    COUNT all-reduces the int64 counts; SUM/AVG first pack counts and sums
+    into one binary64 buffer of 2 n_poly (rj_pack_partials; counts are exact
+    in binary64 below 2^53) so a single collective combines both, then
+    rj_finalize_packed unpacks and finalises.  librj's calls run on the
+    context's stream (rj_get_stream), the collective on torch's current
+    stream, each ordered after the other by stream waits -- including the
+    caller's pending work on the output tensors -- so any stream choice at
+    rj_create is safe."""
     ctx_stream = torch.cuda.ExternalStream(rj.rj_get_stream(R.ctx))
     cur = torch.cuda.current_stream()
-    cur.wait_stream(ctx_stream)
-    if dist.get_backend(group) == "gloo":
-        # gloo stages device tensors through the host outside the stream order
-        cur.synchronize()
-    allreduce_partials(d_count, d_sum if desc.agg != 0 else None, group)
-    ctx_stream.wait_stream(cur)
-    rj.rj_finalize_device(R.ctx, desc.agg, d_count, d_sum, d_value)
+    ctx_stream.wait_stream(cur)                  # caller's work on d_count / d_sum / d_value first
+    rj.rj_query_device(R.ctx, desc, d_count, d_sum)
+    gloo = dist.get_backend(group) == "gloo"
+    if desc.agg == 0:
+        cur.wait_stream(ctx_stream)
+        if gloo:
+            cur.synchronize()                    # gloo stages device tensors through the host
+        c = d_count.view(torch.int64) if d_count.dtype == torch.uint64 else d_count
+        dist.all_reduce(c, op=dist.ReduceOp.SUM, group=group)
+        ctx_stream.wait_stream(cur)
+        rj.rj_finalize_device(R.ctx, desc.agg, d_count, d_sum, d_value)
+    else:
+        n = d_count.numel()
+        if d_packed is None or d_packed.numel() < 2 * n:
+            d_packed = torch.empty(2 * n, dtype=torch.float64, device=d_count.device)
+        rj.rj_pack_partials(R.ctx, d_count, d_sum, d_packed)
+        cur.wait_stream(ctx_stream)
+        if gloo:
+            cur.synchronize()
+        dist.all_reduce(d_packed[:2 * n], op=dist.ReduceOp.SUM, group=group)
+        ctx_stream.wait_stream(cur)
+        rj.rj_finalize_packed(R.ctx, desc.agg, d_packed, d_count, d_value)
     cur.wait_stream(ctx_stream)
     return d_value
 
@@ -133,17 +152,14 @@ def exchange(columns, dest: torch.Tensor, world: int, group=None):
     return out
 
 
-def strip_window(box, splitters, rank: int, world: int, W: int, H: int):
-    """Pixel window (c0, 0, c1, H) of the W x H canvas holding every point of
-    rank's strip [split[rank-1], split[rank]) -- padded by one column each
-    side against rounding, so it is a superset (extra columns hold no point
-    of this rank and cost nothing but their spans)."""
-    import math
+def strip_window(box, splitters, rank: int, world: int, desc):
+    """Pixel window (c0, 0, c1, H) of the canvas desc resolves to, holding
+    every point of rank's strip [split[rank-1], split[rank]) -- exact, through
+    the C ABI's rj_resolve_window (reading Z20)."""
     sp = [float(v) for v in splitters.tolist()] if hasattr(splitters, "tolist") else list(splitters)
-    bw = box[2] - box[0]
-    c0 = 0 if rank == 0 else max(0, int(math.floor((sp[rank - 1] - box[0]) / bw * W)) - 1)
-    c1 = W if rank == world - 1 else min(W, int(math.ceil((sp[rank] - box[0]) / bw * W)) + 1)
-    return (c0, 0, max(c1, c0 + 1), H)
+    lo = -float("inf") if rank == 0 else sp[rank - 1]
+    hi = float("inf") if rank == world - 1 else sp[rank]
+    return rj.rj_resolve_window(box, desc, (lo, -float("inf"), hi, float("inf")))
 
 
 def spatial_shard(x, y, cols, world: int, group=None, box=None, poly_weight: float = 0.0):

@@ -6,9 +6,11 @@ There is no fallback: if librj.so is missing or no sm_100 device is present
 the calls raise.
 
     rj_create, rj_destroy, rj_load_points, rj_load_polygons, rj_query,
-    rj_query_device, rj_query_stream, rj_query_interval, rj_query_interval_ex, rj_query_multi, rj_finalize_device, rj_resolve_canvas(_domain),
-    rj_debug_pixel_spans, rj_debug_boundary_mask, rj_debug_boundary_pieces, rj_debug_point_membership,
-    rj_debug_point_canvas,
+    rj_query_device, rj_pack_partials, rj_finalize_packed, rj_finalize_device,
+    rj_query_stream, rj_query_interval, rj_query_interval_ex, rj_query_multi,
+    rj_resolve_canvas(_domain), rj_resolve_window, rj_resolve_lod,
+    rj_debug_pixel_spans, rj_debug_boundary_mask, rj_debug_boundary_pieces, rj_debug_pip_work,
+    rj_debug_point_membership, rj_debug_point_canvas,
     rj_get_stats, rj_set_option  -- same names as the C ABI.
 
 `RasterJoin` wraps a context with a Pythonic API.
@@ -96,9 +98,15 @@ def lib():
             "rj_finalize_device": (i32, [vp, i32, u32, vp, vp, vp]),
             "rj_resolve_canvas": (i32, [vp, qp, ctypes.POINTER(i32), ctypes.POINTER(i32)]),
             "rj_resolve_canvas_domain": (i32, [d, d, d, d, qp, ctypes.POINTER(i32), ctypes.POINTER(i32)]),
+            "rj_resolve_window": (i32, [d, d, d, d, qp, d, d, d, d, ctypes.POINTER(i32)]),
+            "rj_resolve_lod": (i32, [d, d, d, d, d, d, d, d, i32, i32, ctypes.POINTER(i32), ctypes.POINTER(i32),
+                                     ctypes.POINTER(i32)]),
+            "rj_pack_partials": (i32, [vp, u32, vp, vp, vp]),
+            "rj_finalize_packed": (i32, [vp, i32, u32, vp, vp, vp]),
             "rj_debug_pixel_spans": (i32, [vp, qp, u64, vp, ctypes.POINTER(u64)]),
             "rj_debug_boundary_mask": (i32, [vp, qp, vp]),
             "rj_debug_boundary_pieces": (i32, [vp, qp, vp, vp]),
+            "rj_debug_pip_work": (i32, [vp, ctypes.POINTER(u64), ctypes.POINTER(u64)]),
             "rj_debug_point_membership": (i32, [vp, qp, vp]),
             "rj_get_stats": (i32, [vp, ctypes.POINTER(rj_stats)]),
             "rj_set_option": (i32, [vp, i32, ctypes.c_int64]),
@@ -119,7 +127,8 @@ def lib():
 
 EXPORTS = ["rj_create", "rj_destroy", "rj_set_allocator", "rj_load_points", "rj_load_polygons", "rj_query",
            "rj_query_device", "rj_query_stream", "rj_query_interval", "rj_query_interval_ex", "rj_query_multi", "rj_debug_point_canvas", "rj_finalize_device", "rj_resolve_canvas", "rj_resolve_canvas_domain",
-           "rj_debug_pixel_spans", "rj_debug_boundary_mask", "rj_debug_boundary_pieces", "rj_debug_point_membership", "rj_get_stats",
+           "rj_resolve_window", "rj_resolve_lod", "rj_pack_partials", "rj_finalize_packed",
+           "rj_debug_pixel_spans", "rj_debug_boundary_mask", "rj_debug_boundary_pieces", "rj_debug_pip_work", "rj_debug_point_membership", "rj_get_stats",
            "rj_set_option", "rj_get_stream", "rj_n_polygons", "rj_n_points", "rj_status_str", "rj_last_error", "rj_version"]
 
 
@@ -172,20 +181,30 @@ def make_desc(agg="count", agg_column=-1, preds=(), W=0, H=0, epsilon=0.0, mode=
 
 
 def lod_view(box, viewport, W, H=None):
-    """LOD zoom: the canvas resolution and pixel window that
-    render the world rectangle viewport = (vx0, vy0, vx1, vy1) with about
-    W x H pixels -- a window of a finer virtual canvas over the whole domain
-    (rounded outward to whole pixels).  Returns (W_full, H_full, view)."""
-    import math
-    H = H or W
-    bw, bh = box[2] - box[0], box[3] - box[1]
-    Wf = min(131072, max(1, int(round(W * bw / (viewport[2] - viewport[0])))))
-    Hf = min(131072, max(1, int(round(H * bh / (viewport[3] - viewport[1])))))
-    c0 = max(0, int(math.floor((viewport[0] - box[0]) / bw * Wf)))
-    r0 = max(0, int(math.floor((viewport[1] - box[1]) / bh * Hf)))
-    c1 = min(Wf, int(math.ceil((viewport[2] - box[0]) / bw * Wf)))
-    r1 = min(Hf, int(math.ceil((viewport[3] - box[1]) / bh * Hf)))
-    return Wf, Hf, (c0, r0, max(c1, c0 + 1), max(r1, r0 + 1))
+    """LOD zoom through rj_resolve_lod: the canvas resolution and
+    pixel window that render the world rectangle viewport = (vx0, vy0, vx1,
+    vy1) with about W x H pixels.  Returns (W_full, H_full, view)."""
+    Wf, Hf, v = ctypes.c_int32(), ctypes.c_int32(), (ctypes.c_int32 * 4)()
+    _check(lib().rj_resolve_lod(*map(float, box), *map(float, viewport), int(W), int(H or W), ctypes.byref(Wf),
+                                ctypes.byref(Hf), v))
+    return Wf.value, Hf.value, tuple(v)
+
+
+def rj_resolve_window(box, desc, rect):
+    """Pixel window (c0, r0, c1, r1) holding every point of the world
+    rectangle rect = (wx0, wy0, wx1, wy1), half-open (+-inf allowed)."""
+    v = (ctypes.c_int32 * 4)()
+    _check(lib().rj_resolve_window(*map(float, box), ctypes.byref(desc), *map(float, rect), v))
+    return tuple(v)
+
+
+def rj_pack_partials(ctx, d_count, d_sum, d_packed):
+    _check(lib().rj_pack_partials(ctx, len(d_count), _ptr(d_count), _ptr(d_sum), _ptr(d_packed)), ctx)
+
+
+def rj_finalize_packed(ctx, agg, d_packed, d_count, d_value):
+    a = AGG[agg] if isinstance(agg, str) else int(agg)
+    _check(lib().rj_finalize_packed(ctx, a, len(d_count), _ptr(d_packed), _ptr(d_count), _ptr(d_value)), ctx)
 
 
 # ---- C-ABI names ------------------------------------------------------------
@@ -204,7 +223,21 @@ def rj_set_option(ctx, option, value):
     _check(lib().rj_set_option(ctx, int(option), int(value)), ctx)
 
 
+def _order_after_producer(ctx, arrays):
+    """Device tensors may still be in flight on torch's current stream: make
+    the context's stream wait for it before librj reads them."""
+    if not any(getattr(a, "is_cuda", False) for a in arrays):
+        return
+    import torch
+    s = rj_get_stream(ctx)
+    if s:
+        torch.cuda.ExternalStream(s).wait_stream(torch.cuda.current_stream())
+    else:
+        torch.cuda.current_stream().synchronize()
+
+
 def rj_load_points(ctx, x, y, cols=()):
+    _order_after_producer(ctx, [x, y, *cols])
     n = len(x)
     ptrs = (ctypes.c_void_p * max(1, len(cols)))(*[_ptr(c) for c in cols])
     dts = (ctypes.c_int32 * max(1, len(cols)))(*[_dtype_code(c) for c in cols])
@@ -225,6 +258,7 @@ def rj_query(ctx, desc, count=None, value=None):
 
 
 def rj_query_stream(ctx, desc, x, y, cols=(), count=None, value=None):
+    _order_after_producer(ctx, [x, y, *cols])
     n = len(x)
     ptrs = (ctypes.c_void_p * max(1, len(cols)))(*[_ptr(c) for c in cols])
     dts = (ctypes.c_int32 * max(1, len(cols)))(*[_dtype_code(c) for c in cols])
@@ -314,6 +348,13 @@ def rj_debug_boundary_pieces(ctx, desc):
     cov = np.zeros_like(bnd)
     _check(lib().rj_debug_boundary_pieces(ctx, ctypes.byref(desc), _ptr(bnd), _ptr(cov)), ctx)
     return bnd, cov
+
+
+def rj_debug_pip_work(ctx):
+    """(boundary points tested, edge-grid entries walked) of the last accurate query."""
+    a, b = ctypes.c_uint64(), ctypes.c_uint64()
+    _check(lib().rj_debug_pip_work(ctx, ctypes.byref(a), ctypes.byref(b)), ctx)
+    return a.value, b.value
 
 
 def rj_debug_point_membership(ctx, desc, n_input):

@@ -5,6 +5,7 @@ import math
 import os
 import re
 
+import numpy as np
 import pytest
 
 import oracle
@@ -102,3 +103,38 @@ def test_lod_view_helper():
     Wf, Hf, v = rj.lod_view((0, 0, 1024, 1024), (100, 100, 150, 200), 1000)
     assert (Wf, Hf) == (20480, 10240)
     assert v == (2000, 1000, 3000, 2000)
+
+
+def test_resolve_window_exact_and_tight():
+    """rj_resolve_window (reading Z20) against the oracle's O1/O2 maps: on
+    random domains, canvases and world rectangles, every point of the
+    half-open rectangle falls in the window, and the window is tight (its
+    first and last columns/rows hold the rectangle's extreme points)."""
+    import oracle
+    rng = np.random.default_rng(99)
+    for _ in range(300):
+        x0, y0 = rng.uniform(-1e6, 1e6, 2)
+        w, h = 10 ** rng.uniform(-3, 6, 2)
+        box = (x0, y0, x0 + w, y0 + h)
+        W, H = int(rng.integers(1, 131073)), int(rng.integers(1, 5000))
+        q = rj.make_desc(W=W, H=H)
+        a, b = np.sort(rng.uniform(x0 - 0.1 * w, x0 + 1.1 * w, 2))
+        c, d = np.sort(rng.uniform(y0 - 0.1 * h, y0 + 1.1 * h, 2))
+        if a == b or c == d:
+            continue
+        v = rj.rj_resolve_window(box, q, (a, c, b, d))
+        assert 0 <= v[0] < v[2] <= W and 0 <= v[1] < v[3] <= H
+        xs = np.concatenate([rng.uniform(a, b, 200), [a, np.nextafter(b, -np.inf)]])
+        ys = np.concatenate([rng.uniform(c, d, 200), [c, np.nextafter(d, -np.inf)]])
+        for vals, lo, hi, n, p0, p1 in ((xs, box[0], box[2], W, v[0], v[2]), (ys, box[1], box[3], H, v[1], v[3])):
+            qv = np.array([oracle.quantize(float(t), lo, hi) for t in vals])
+            inside = (qv >= 0) & (qv < (1 << 30))
+            pix = (qv[inside] * n) >> 30
+            assert np.all((pix >= p0) & (pix < p1))
+            if inside[-2] and inside[-1]:
+                assert pix.min() == p0 and pix.max() == p1 - 1
+    # the whole domain and +-infinity
+    q = rj.make_desc(W=777, H=555)
+    assert rj.rj_resolve_window((0, 0, 1, 1), q, (-np.inf, -np.inf, np.inf, np.inf)) == (0, 0, 777, 555)
+    with pytest.raises(rj.RJError):
+        rj.rj_resolve_window((0, 0, 1, 1), q, (0.5, 0, 0.5, 1))

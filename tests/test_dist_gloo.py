@@ -90,7 +90,8 @@ def _spatial_worker(rank, world, port, q):
         hi_x = np.inf if rank == world - 1 else float(sp[rank])
         assert np.all((xs >= lo_x) & (xs < hi_x))
         W = 4096
-        view = rjdist.strip_window(C.NYC_BOX, sp, rank, world, W, W)
+        from paper_journals_pvldb_zacharatoudasf17_b200 import rj
+        view = rjdist.strip_window(C.NYC_BOX, sp, rank, world, rj.make_desc(W=W, H=W))
         P = oracle.Polys(C.array_polys("neighborhoods"), C.NYC_BOX)
         preds = [(0, ">=", C.T_2012[0]), (0, "<", C.T_2012[1])]
         out = []

@@ -57,7 +57,7 @@ def _run(rank, world, port, q, spatial=False):
             tx, ty, tc, sp = rjdist.spatial_shard(torch.from_numpy(x.copy()), torch.from_numpy(y.copy()),
                                                   [torch.from_numpy(c.copy()) for c in cols], world)
             x, y, cols = tx.numpy(), ty.numpy(), [c.numpy() for c in tc]
-            view = rjdist.strip_window(C.NYC_BOX, sp, rank, world, 4096, 4096)
+            view = rjdist.strip_window(C.NYC_BOX, sp, rank, world, rj.make_desc(W=4096, H=4096))
         R.load_points(x, y, cols)
         R.load_polygons(C.array_polys("neighborhoods"))
         out = {}

@@ -166,6 +166,26 @@ def test_high_resolution_parity(c1, W, mode):
     assert np.array_equal(cnt, ocnt)
 
 
+@pytest.mark.parametrize("W,H,view", [(64, 70000, None), (131072, 131072, (60000, 0, 60512, 131072))])
+def test_label_canvas_taller_than_grid_y(c1, W, H, view):
+    """Label-canvas paths (MIN/MAX, multi-aggregate, streamed) on windows
+    more than 65535 rows high: the label canvas init strides rows over
+    gridDim.y (a launch with gridDim.y = height failed)."""
+    R, P, x, y, cols = c1
+    for mode in ("bounded", "accurate"):
+        ocnt, osum, _ = oracle.query(P, x, y, cols=cols, agg_col=0, W=W, H=H, mode=mode, view=view)
+        mn, mx = oracle.query_minmax(P, x, y, cols, 1, W=W, H=H, mode=mode, view=view)
+        cnt, v = R.query(W=W, H=H, mode=mode, agg="min", agg_column=1, view=view)
+        assert np.array_equal(cnt, ocnt), mode
+        assert np.array_equal(v[cnt > 0], mn[cnt > 0])
+        cnt, vals = R.query_multi([("max", 1), ("sum", 0)], W=W, H=H, mode=mode, view=view)
+        assert np.array_equal(cnt, ocnt) and np.array_equal(vals[0][cnt > 0], mx[cnt > 0])
+        assert np.array_equal(vals[1], osum)
+        cnt, val = R.query_stream(x, y, cols, W=W, H=H, mode=mode, agg="sum", agg_column=0, view=view)
+        assert np.array_equal(cnt, ocnt) and np.array_equal(val, osum), mode
+        assert ocnt.sum() > 0
+
+
 def test_view_errors(c1):
     R, P, x, y, cols = c1
     for view in ((0, 0, 1025, 10), (5, 0, 5, 10), (-1, 0, 3, 3), (0, 7, 3, 3)):

@@ -91,7 +91,7 @@ def main():
                     d = desc
                 else:
                     sel = dest == r
-                    d = rj.make_desc(**q, view=rjdist.strip_window(box, sp, r, P, W, H))
+                    d = rj.make_desc(**q, view=rjdist.strip_window(box, sp, r, P, desc))
                 R.load_points(np.ascontiguousarray(x[sel]), np.ascontiguousarray(y[sel]),
                               [np.ascontiguousarray(c[sel]) for c in cols])
                 ms, cnt, st = time_query(R, d, stream, args.steps)

@@ -309,6 +309,9 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     a.n_stages = (uint32_t)point_pass_stages(f.n_slots);
     if ((s = items_for_level(c, P.L)) != RJ_OK) return s;
     c->launches = 0;
+    // work counters / pass statistics (cleared per pass)
+    Buf &wk = wsbuf(c, kWsWork);
+    if (dreserve(c, wk, 64)) return set_error(c, RJ_ERR_OOM, "workspace allocation failed");
     if (c->timing) RJ_CUDA(c, record_ev(c, 0));
     // the index join needs neither spans nor the boundary mask
     P.pp = PolyPass{};
@@ -339,7 +342,6 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     a.edges = c->edges.as<int4>();
     a.edge_poly = c->edge_poly.as<uint32_t>();
     Buf &st = wsbuf(c, kWsWork);
-    if (dreserve(c, st, 64)) return set_error(c, RJ_ERR_OOM, "workspace allocation failed");
     a.work_counter = st.as<uint32_t>();
     a.stats = reinterpret_cast<unsigned long long *>(st.as<uint32_t>() + 2);
     a.view[0] = P.view.c0;

@@ -83,10 +83,7 @@ __device__ __forceinline__ void process(const PassArgs &a, const Shared &sh, con
         for (int j = 0; j < kIPL; ++j)
             if (ok[j] && (lds(t.tbase + key[j] * 4u) & kFlag)) bm |= 1u << j;
         if (__any_sync(kFull, bm != 0u)) {
-#pragma unroll
-            for (int j = 0; j < kIPL; ++j) {
-                enqueue<SUM, NS>(a, sh, w, j, (bm >> j) & 1u, bq, n_bnd);
-            }
+            enqueue_window<SUM, NS>(a, sh, w, bm, bq, n_bnd);
 #pragma unroll
             for (int j = 0; j < kIPL; ++j) ok[j] = ok[j] && !((bm >> j) & 1u);
         }

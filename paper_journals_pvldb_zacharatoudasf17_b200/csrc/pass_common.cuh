@@ -254,6 +254,59 @@ __device__ __forceinline__ void enqueue(const PassArgs &a, const Shared &sh, con
     if (q.qn >= 32) drain_queue<SUM>(a, sh, q.qn, false);       // leaves < 32
 }
 
+// Append the boundary points of a whole 256-point window (bit j of bm: this
+// lane's point j is a boundary point) -- one warp scan of the per-lane
+// counts instead of a ballot per point slot.  Ranks follow (lane, j), the
+// order enqueue() would give; a window may fill the current chunk and
+// continue in the next one.  Without a global chunk the points go to the
+// warp's shared queue, tested 32 at a time.
+template <bool SUM, int NS>
+__device__ __forceinline__ void enqueue_window(const PassArgs &a, const Shared &sh, const Win<NS> &w, uint32_t bm,
+                                               BQ &q, uint32_t &n_bnd) {
+    const int lane = threadIdx.x & 31;
+    const uint32_t c = __popc(bm);
+    uint32_t incl = c;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+        const uint32_t t = __shfl_up_sync(kFull, incl, o);
+        if (lane >= o) incl += t;
+    }
+    const uint32_t total = __shfl_sync(kFull, incl, 31);
+    if (!total) return;
+    n_bnd += c;
+    const uint32_t excl = incl - c;
+    for (uint32_t done = 0; done < total;) {
+        if (q.global && q.pos == q.end) bq_next_chunk(a, q);
+        const bool glob = q.pos < q.end;
+        const uint32_t room = glob ? q.end - q.pos : (uint32_t)kQ - q.qn;
+        const uint32_t take = min(total - done, room);
+        const uint32_t at = glob ? q.pos : q.qn;
+#pragma unroll
+        for (int j = 0; j < kIPL; ++j) {
+            const uint32_t r = excl + __popc(bm & ((1u << j) - 1u));   // rank of point j
+            if (((bm >> j) & 1u) && r >= done && r < done + take) {
+                const uint32_t pos = at + (r - done);
+                if (glob) {
+                    a.bq_x[pos] = w.x[j];
+                    a.bq_y[pos] = w.y[j];
+                    if (SUM) a.bq_a[pos] = agg_bits<NS>(a, w, j);
+                } else {
+                    sh.qx[pos] = w.x[j];
+                    sh.qy[pos] = w.y[j];
+                    sh.qa[pos] = SUM ? agg_bits<NS>(a, w, j) : 0u;
+                }
+            }
+        }
+        done += take;
+        if (glob) {
+            q.pos += take;
+        } else {
+            q.qn += take;
+            if (q.qn >= 32) drain_queue<SUM>(a, sh, q.qn, false);   // leaves < 32
+        }
+    }
+}
+
 // end of the pass: close the chunk, test what is left in the shared queue
 template <bool SUM>
 __device__ __forceinline__ void bq_finish(const PassArgs &a, const Shared &sh, BQ &q) {

@@ -130,16 +130,16 @@ __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh,
     }
     fold(acc, cy);
     if (__any_sync(kFull, spec)) {                            // rare: overlaps, boundary pixels
+        uint32_t bm = 0;
 #pragma unroll
         for (int j = 0; j < kIPL; ++j) {
             if (lab[j] == kMulti)
                 multi_point(a, sh, t, mulhi(w.x[j], k.W4), mulhi(w.y[j], k.H4),
                             attr_d<AF>(agg_bits<NS>(a, w, j)));
-            if (ACC) {
-                enqueue<true, NS>(a, sh, w, j, lab[j] == kBnd, bq, n_bnd);
-            }
+            if (ACC && lab[j] == kBnd) bm |= 1u << j;
             if (lab[j] >= kBnd) lab[j] = kNone;
         }
+        if (ACC) enqueue_window<true, NS>(a, sh, w, bm, bq, n_bnd);
     }
     // Runs of equal labels: inside the lane in registers, across lanes by a
     // segmented scan, and across windows through the warp's carry (Morton

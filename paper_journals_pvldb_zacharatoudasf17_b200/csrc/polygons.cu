@@ -159,41 +159,53 @@ __device__ __forceinline__ bool culled(const int4 M, int W, int H, const int4 vi
     return c1 < view.x || c0 >= view.z || r1 < view.y || r0 >= view.w;
 }
 
+__device__ __forceinline__ void edge_rows_body(uint32_t t0, uint32_t ts, const int4 *__restrict__ edges,
+                                               const uint32_t *__restrict__ edge_poly, const int4 *__restrict__ mbr,
+                                               uint32_t n_edges, int H, uint32_t *__restrict__ rows, int accurate,
+                                               int W, uint32_t *__restrict__ bands, int4 view) {
+    for (uint32_t e = t0; e < n_edges; e += ts) {
+        if (culled(mbr[edge_poly[e]], W, H, view)) {
+            rows[e] = 0;
+            if (accurate) bands[e] = 0;
+            continue;
+        }
+        const int4 E = edges[e];
+        const int64_t ymin = min(E.y, E.w), ymax = max(E.y, E.w);
+        rows[e] = (uint32_t)(row_start(ymax, H) - row_start(ymin, H));
+        // S5 row bands: pixel rows whose closed lattice extent meets [ymin, ymax]
+        if (accurate) bands[e] = (uint32_t)band_rows(ymin, ymax, H);
+    }
+}
+
 __global__ void k_edge_rows(const int4 *__restrict__ edges, const uint32_t *__restrict__ edge_poly,
                             const int4 *__restrict__ mbr, uint32_t n_edges, int H,
                             uint32_t *__restrict__ rows, int accurate, int W,
                             uint32_t *__restrict__ bands, int4 view) {
-    const uint32_t e = blockIdx.x * blockDim.x + threadIdx.x;
-    if (e >= n_edges) return;
-    if (culled(mbr[edge_poly[e]], W, H, view)) {
-        rows[e] = 0;
-        if (accurate) bands[e] = 0;
-        return;
-    }
-    const int4 E = edges[e];
-    const int64_t ymin = min(E.y, E.w), ymax = max(E.y, E.w);
-    rows[e] = (uint32_t)(row_start(ymax, H) - row_start(ymin, H));
-    if (accurate) {
-        // S5 row bands: pixel rows whose closed lattice extent meets [ymin, ymax]
-        bands[e] = (uint32_t)band_rows(ymin, ymax, H);
+    edge_rows_body(blockIdx.x * blockDim.x + threadIdx.x, gridDim.x * blockDim.x, edges, edge_poly, mbr, n_edges, H,
+                   rows, accurate, W, bands, view);
+}
+
+__device__ __forceinline__ void poly_rows_body(uint32_t t0, uint32_t ts, const int4 *__restrict__ mbr,
+                                               uint32_t n_poly, int W, int H, uint32_t *__restrict__ rows,
+                                               int4 view) {
+    for (uint32_t p = t0; p < n_poly; p += ts) {
+        const int4 M = mbr[p];
+        rows[p] = culled(M, W, H, view) ? 0u : (uint32_t)(row_start(M.w, H) - row_start(M.y, H));
     }
 }
 
 __global__ void k_poly_rows(const int4 *__restrict__ mbr, uint32_t n_poly, int W, int H, uint32_t *__restrict__ rows,
                             int4 view) {
-    const uint32_t p = blockIdx.x * blockDim.x + threadIdx.x;
-    if (p >= n_poly) return;
-    const int4 M = mbr[p];
-    rows[p] = culled(M, W, H, view) ? 0u : (uint32_t)(row_start(M.w, H) - row_start(M.y, H));
+    poly_rows_body(blockIdx.x * blockDim.x + threadIdx.x, gridDim.x * blockDim.x, mbr, n_poly, W, H, rows, view);
 }
 
-__global__ void k_crossings(const int4 *__restrict__ edges, const uint32_t *__restrict__ edge_poly,
+__device__ __forceinline__ void crossings_body(uint32_t t0, uint32_t ts, const int4 *__restrict__ edges, const uint32_t *__restrict__ edge_poly,
                             const int4 *__restrict__ mbr, const uint32_t *__restrict__ edge_off,
                             uint32_t n_edges, const uint32_t *__restrict__ prow_off, int W, int H,
                             uint32_t *__restrict__ cx_pr, uint32_t *__restrict__ cx_t,
                             uint32_t *__restrict__ pr_cnt) {
     const uint32_t total = edge_off[n_edges];
-    for (uint32_t j = blockIdx.x * blockDim.x + threadIdx.x; j < total; j += gridDim.x * blockDim.x) {
+    for (uint32_t j = t0; j < total; j += ts) {
         const uint32_t e = upper_bound_u32(edge_off, n_edges + 1, j) - 1;
         const int4 E = edges[e];
         const uint32_t P = edge_poly[e];
@@ -207,13 +219,27 @@ __global__ void k_crossings(const int4 *__restrict__ edges, const uint32_t *__re
     }
 }
 
-__global__ void k_scatter_t(const uint32_t *__restrict__ cx_pr, const uint32_t *__restrict__ cx_t,
+__global__ void k_crossings(const int4 *__restrict__ edges, const uint32_t *__restrict__ edge_poly,
+                            const int4 *__restrict__ mbr, const uint32_t *__restrict__ edge_off,
+                            uint32_t n_edges, const uint32_t *__restrict__ prow_off, int W, int H,
+                            uint32_t *__restrict__ cx_pr, uint32_t *__restrict__ cx_t,
+                            uint32_t *__restrict__ pr_cnt) {
+    crossings_body(blockIdx.x * blockDim.x + threadIdx.x, gridDim.x * blockDim.x, edges, edge_poly, mbr, edge_off, n_edges, prow_off, W, H, cx_pr, cx_t, pr_cnt);
+}
+
+__device__ __forceinline__ void scatter_t_body(uint32_t t0, uint32_t ts, const uint32_t *__restrict__ cx_pr, const uint32_t *__restrict__ cx_t,
                             uint32_t total, const uint32_t *__restrict__ pr_off,
                             uint32_t *__restrict__ pr_cur, uint32_t *__restrict__ tv) {
-    for (uint32_t j = blockIdx.x * blockDim.x + threadIdx.x; j < total; j += gridDim.x * blockDim.x) {
+    for (uint32_t j = t0; j < total; j += ts) {
         const uint32_t pr = cx_pr[j];
         tv[pr_off[pr] + atomicAdd(&pr_cur[pr], 1u)] = cx_t[j];
     }
+}
+
+__global__ void k_scatter_t(const uint32_t *__restrict__ cx_pr, const uint32_t *__restrict__ cx_t,
+                            uint32_t total, const uint32_t *__restrict__ pr_off,
+                            uint32_t *__restrict__ pr_cur, uint32_t *__restrict__ tv) {
+    scatter_t_body(blockIdx.x * blockDim.x + threadIdx.x, gridDim.x * blockDim.x, cx_pr, cx_t, total, pr_off, pr_cur, tv);
 }
 
 struct SpanGeo {
@@ -279,10 +305,10 @@ __device__ __forceinline__ void sort_small(uint32_t *p, uint32_t m) {
 }
 
 // Sort each (polygon,row) threshold list, count its spans and their pieces.
-__global__ void k_prow_count(SpanGeo g, uint32_t n_prow, const uint32_t *__restrict__ pr_off,
+__device__ __forceinline__ void prow_count_body(uint32_t t0, uint32_t ts, SpanGeo g, uint32_t n_prow, const uint32_t *__restrict__ pr_off,
                              uint32_t *__restrict__ tv, uint32_t *__restrict__ span_cnt,
                              uint32_t *__restrict__ piece_cnt) {
-    for (uint32_t pr = blockIdx.x * blockDim.x + threadIdx.x; pr < n_prow; pr += gridDim.x * blockDim.x) {
+    for (uint32_t pr = t0; pr < n_prow; pr += ts) {
         const uint32_t b = pr_off[pr], e = pr_off[pr + 1];
         const uint32_t m = e - b;                            // the usual case: sort in registers
         if (m <= 2) {
@@ -318,11 +344,17 @@ __global__ void k_prow_count(SpanGeo g, uint32_t n_prow, const uint32_t *__restr
     }
 }
 
-__global__ void k_prow_emit(SpanGeo g, uint32_t n_prow, const uint32_t *__restrict__ pr_off,
+__global__ void k_prow_count(SpanGeo g, uint32_t n_prow, const uint32_t *__restrict__ pr_off,
+                             uint32_t *__restrict__ tv, uint32_t *__restrict__ span_cnt,
+                             uint32_t *__restrict__ piece_cnt) {
+    prow_count_body(blockIdx.x * blockDim.x + threadIdx.x, gridDim.x * blockDim.x, g, n_prow, pr_off, tv, span_cnt, piece_cnt);
+}
+
+__device__ __forceinline__ void prow_emit_body(uint32_t t0, uint32_t ts, SpanGeo g, uint32_t n_prow, const uint32_t *__restrict__ pr_off,
                             const uint32_t *__restrict__ tv, const uint32_t *__restrict__ span_off,
                             uint32_t *__restrict__ spans, const uint32_t *__restrict__ piece_off,
                             uint32_t *__restrict__ piece_cur, uint2 *__restrict__ pieces) {
-    for (uint32_t pr = blockIdx.x * blockDim.x + threadIdx.x; pr < n_prow; pr += gridDim.x * blockDim.x) {
+    for (uint32_t pr = t0; pr < n_prow; pr += ts) {
         const uint32_t b = pr_off[pr], e = pr_off[pr + 1];
         uint32_t P;
         int64_t r;
@@ -359,6 +391,13 @@ __global__ void k_prow_emit(SpanGeo g, uint32_t n_prow, const uint32_t *__restri
     }
 }
 
+__global__ void k_prow_emit(SpanGeo g, uint32_t n_prow, const uint32_t *__restrict__ pr_off,
+                            const uint32_t *__restrict__ tv, const uint32_t *__restrict__ span_off,
+                            uint32_t *__restrict__ spans, const uint32_t *__restrict__ piece_off,
+                            uint32_t *__restrict__ piece_cur, uint2 *__restrict__ pieces) {
+    prow_emit_body(blockIdx.x * blockDim.x + threadIdx.x, gridDim.x * blockDim.x, g, n_prow, pr_off, tv, span_off, spans, piece_off, piece_cur, pieces);
+}
+
 // -------------------------------------------------------------- S5 supercover
 // (marks only inside the viewport window [c0, c1) x [r0, r1))
 __global__ void k_mask_mark(const int4 *__restrict__ edges, const uint32_t *__restrict__ band_off,
@@ -391,11 +430,11 @@ __global__ void k_mask_mark(const int4 *__restrict__ edges, const uint32_t *__re
 // of reading the mask rows per cell (a dependent global load between two
 // CTA barriers).  A pixel touched by several edges appears several times.
 template <bool EMIT>
-__global__ void k_bnd_pieces(SpanGeo g, const int4 *__restrict__ edges, const uint32_t *__restrict__ band_off,
+__device__ __forceinline__ void bnd_pieces_body(uint32_t t0, uint32_t ts, SpanGeo g, const int4 *__restrict__ edges, const uint32_t *__restrict__ band_off,
                              uint32_t n_edges, uint32_t *__restrict__ cnt, const uint32_t *__restrict__ off,
                              uint32_t *__restrict__ cur, uint32_t *__restrict__ out) {
     const uint32_t total = band_off[n_edges];
-    for (uint32_t j = blockIdx.x * blockDim.x + threadIdx.x; j < total; j += gridDim.x * blockDim.x) {
+    for (uint32_t j = t0; j < total; j += ts) {
         const uint32_t e = upper_bound_u32(band_off, n_edges + 1, j) - 1;
         const int4 E = edges[e];
         const int64_t r = pix(min(E.y, E.w), g.H) + (j - band_off[e]);
@@ -408,6 +447,13 @@ __global__ void k_bnd_pieces(SpanGeo g, const int4 *__restrict__ edges, const ui
             else atomicAdd(&cnt[cell], 1u);
         });
     }
+}
+
+template <bool EMIT>
+__global__ void k_bnd_pieces(SpanGeo g, const int4 *__restrict__ edges, const uint32_t *__restrict__ band_off,
+                             uint32_t n_edges, uint32_t *__restrict__ cnt, const uint32_t *__restrict__ off,
+                             uint32_t *__restrict__ cur, uint32_t *__restrict__ out) {
+    bnd_pieces_body<EMIT>(blockIdx.x * blockDim.x + threadIdx.x, gridDim.x * blockDim.x, g, edges, band_off, n_edges, cnt, off, cur, out);
 }
 
 }  // namespace
@@ -585,6 +631,8 @@ rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp,
         dreserve(c, sizes, 64))
         return set_error(c, RJ_ERR_OOM, "workspace allocation failed");
     const int4 vw = v.full ? make_int4(0, 0, W, H) : make_int4(v.c0, v.r0, v.c1, v.r1);
+    const int64_t key[9] = {W, H, L, accurate ? 1 : 0, vw.x, vw.y, vw.z, vw.w, (int64_t)c->data_gen};
+    const bool known = c->pp_key_valid && std::equal(key, key + 9, c->pp_key);
     k_edge_rows<<<blocks_for(ne, 256), 256, 0, st>>>(c->edges.as<int4>(), c->edge_poly.as<uint32_t>(),
                                                      c->mbr.as<int4>(), ne, H, erows.as<uint32_t>(), accurate, W,
                                                      bcnt.as<uint32_t>(), vw);
@@ -596,8 +644,6 @@ rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp,
     RJ_CUDA(c, scan_u32(c, prows.as<uint32_t>(), proff.as<uint32_t>(), np, kWsScan));
     if (accurate) RJ_CUDA(c, scan_u32(c, bcnt.as<uint32_t>(), boff.as<uint32_t>(), ne, kWsScan));
     // sync 1: crossing / polygon-row / band totals (skipped for a repeated key)
-    const int64_t key[9] = {W, H, L, accurate ? 1 : 0, vw.x, vw.y, vw.z, vw.w, (int64_t)c->data_gen};
-    const bool known = c->pp_key_valid && std::equal(key, key + 9, c->pp_key);
     uint32_t *hs = reinterpret_cast<uint32_t *>(c->h_stats + 8);
     if (known) {
         std::copy(c->pp_sizes, c->pp_sizes + 6, hs);

@@ -98,11 +98,16 @@ RJ_HD uint32_t cell_y(uint32_t c) { return compact16(c >> 1); }
 RJ_HD int64_t cell_pix_lo(int64_t cc, int64_t n, int L) { return pix(cc << (kLatticeBits - L), n); }
 RJ_HD int64_t cell_pix_hi(int64_t cc, int64_t n, int L) { return pix(((cc + 1) << (kLatticeBits - L)) - 1, n); }
 
-// S5 supercover (reading Z7, O-S): pixel columns [i0, i1] of row r touched by
+// S5 supercover (reading Z6, O9): pixel columns [i0, i1] of row r touched by
 // edge (xa,ya)-(xb,yb): clip the segment to the row's closed lattice band
-// y in [max(qlo(r), ymin), min(qhi(r), ymax)], take the ceil of its left and
-// the floor of its right x-extent, exclude coordinate 2^30.  False when the
-// edge passes between two pixels' lattice extents.
+// y in [max(qlo(r), ymin), min(qhi(r), ymax)]; its real x-extent [xl, xr]
+// meets pixel i's closed extent [qlo(i), qhi(i)] (integers) iff
+// qlo(i) <= floor(xr) and qhi(i) >= ceil(xl), i.e. pix(ceil(xl)) <= i <=
+// pix(floor(xr)).  That range is empty only when the clipped segment lies in
+// the open gap (qhi(i), qlo(i+1)) between two pixels' extents; a nearly
+// vertical edge whose x-extent falls strictly between two consecutive
+// lattice values INSIDE one pixel's extent (ceil(xl) > floor(xr), same
+// pixel) touches that pixel.  Coordinate 2^30 and beyond is excluded.
 RJ_HD bool supercover_cols(int64_t xa, int64_t ya, int64_t xb, int64_t yb, int64_t r, int64_t W, int64_t H,
                            int64_t &i0, int64_t &i1) {
     const int64_t ymin = ya < yb ? ya : yb, ymax = ya < yb ? yb : ya;
@@ -122,10 +127,9 @@ RJ_HD bool supercover_cols(int64_t xa, int64_t ya, int64_t xb, int64_t yb, int64
     }
     if (cl >= kOne) return false;
     if (fr > kOne - 1) fr = kOne - 1;
-    if (fr < cl) return false;
     i0 = pix(cl, W);
     i1 = pix(fr, W);
-    return true;
+    return i0 <= i1;
 }
 
 // Rows of the supercover band of an edge / polygon with y-extent [ymin, ymax]:

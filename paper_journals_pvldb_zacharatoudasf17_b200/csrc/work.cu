@@ -71,6 +71,38 @@ rj_status items_for_level(Ctx *c, int L) {
         gcells += 1;
     }
     flush();
+    // Guided tail: CTAs take items in order from one counter, so the last
+    // items decide how unevenly the persistent grid finishes (a 64k-point
+    // item is ~40 us of one CTA's stream).  The items holding the last ~one
+    // item per CTA of points are re-cut into single cells and <= CH/8-point
+    // chunks, so every CTA that finishes its last large item finds small
+    // ones -- the points are the same, only the final items are finer.
+    {
+        uint64_t total = 0;
+        for (const int4 &I : items) total += (uint64_t)(I.w - I.z);
+        const uint64_t tail_pts = std::min<uint64_t>(total / 4, (uint64_t)c->num_sms * 2 * CH);
+        const uint64_t cht = std::max<uint64_t>(2048, CH / 8);
+        size_t k = items.size();
+        uint64_t acc = 0;
+        while (k > 0 && acc < tail_pts) {
+            --k;
+            acc += (uint64_t)(items[k].w - items[k].z);
+        }
+        std::vector<int4> tail;
+        for (size_t i = k; i < items.size(); ++i) {
+            const int4 I = items[i];
+            for (int64_t cc = I.x; cc < I.y; ++cc) {
+                const uint64_t b = std::max<uint64_t>((uint64_t)I.z, off[(uint64_t)cc << sh]);
+                const uint64_t e = std::min<uint64_t>((uint64_t)I.w, off[(uint64_t)(cc + 1) << sh]);
+                if (b >= e) continue;
+                const uint64_t m = e - b, parts = (m + cht - 1) / cht;
+                for (uint64_t j = 0; j < parts; ++j)
+                    tail.push_back(make_int4((int)cc, (int)cc + 1, (int)(b + m * j / parts), (int)(b + m * (j + 1) / parts)));
+            }
+        }
+        items.resize(k);
+        items.insert(items.end(), tail.begin(), tail.end());
+    }
     // non-empty point cells of the level as a bitmask (the polygon pass skips
     // span pieces of empty cells with one L1-friendly word load)
     std::vector<uint32_t> bits((ncell + 31) / 32, 0u);

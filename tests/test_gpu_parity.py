@@ -397,3 +397,54 @@ def test_sharding_sums_to_unsharded():
     assert np.array_equal(acc_c, c_all)
     ok, _ = rel_close(acc_s, s_all)
     assert ok
+
+
+# ---------------------------------------------- nearly axis-parallel edges
+def _sliver_set():
+    """C1 polygons plus a quad whose right edge is nearly vertical (dx = 3
+    lattice units over 800 world units) and whose top edge is nearly
+    horizontal: within a pixel row the right edge's x-extent lies strictly
+    between two consecutive lattice values inside one pixel's extent.  Round
+    2's full-size C3 parity run found tract edges of this kind whose
+    boundary pixels the supercover skipped (O9)."""
+    u = 2.0 ** -20
+    quad = [np.array([(200.0, 100.0), (300.0 + u, 100.0), (300.0 + 4 * u, 900.0 + u), (200.0, 900.0 + 4 * u)], float)]
+    tall = [np.array([(600.0, 50.0), (600.0 + 2 * u, 50.0), (600.0 + 3 * u, 1000.0), (599.0, 1000.0)], float)]
+    return C.polygon_set("c1") + [quad, tall]
+
+
+@pytest.mark.parametrize("W,H", [(1024, 1024), (333, 517), (4096, 4096), (8192, 8192)])
+def test_nearly_axis_parallel_edges(W, H):
+    polys = _sliver_set()
+    flat = PG.flatten(polys)
+    rng = np.random.default_rng(W + H)
+    n = 400_000
+    x = rng.uniform(0, 1024, n)
+    y = rng.uniform(0, 1024, n)
+    # a third of the points hug the nearly vertical edges (inside and outside)
+    k = n // 3
+    x[:k // 2] = 300.0 + rng.uniform(-0.6, 0.6, k // 2)
+    x[k // 2:k] = 600.0 + rng.uniform(-0.6, 0.6, k - k // 2)
+    fav = rng.integers(-1000, 1000, n).astype(np.int32)
+    R = gpu_ctx(C.C1_BOX, flat, x, y, [fav])
+    P = oracle.Polys(flat, C.C1_BOX)
+    o = oracle.boundary_mask(P, W, H)
+    assert np.array_equal(R.boundary_mask(W=W, H=H), o)
+    bnd, cov = R.boundary_pieces(W=W, H=H)
+    ob = _unpack_bits(o, W)
+    assert np.array_equal(_unpack_bits(bnd, W), ob & _unpack_bits(cov, W))
+    for mode in ("bounded", "accurate"):
+        for variant in (0, 1):
+            R.set_option(rjmod.OPT_PASS, variant)
+            cnt, val = R.query(W=W, H=H, mode=mode, agg="sum", agg_column=0)
+            ocnt, osum, _ = oracle.query(P, x, y, cols=[fav], agg_col=0, W=W, H=H, mode=mode)
+            assert np.array_equal(cnt, ocnt), (mode, variant)
+            assert np.array_equal(val, osum), (mode, variant)
+    cnt, _ = R.query_stream(x, y, [fav], W=W, H=H, mode="accurate")
+    assert np.array_equal(cnt, oracle.query(P, x, y, W=W, H=H, mode="accurate")[0])
+    if W <= 1024:
+        c_, v_, ep, em = R.query_interval(W=W, H=H)
+        counts = oracle.pixel_counts(x, y, C.C1_BOX, W=W, H=H)
+        oep, oem = oracle.error_interval(P, W, H, counts)
+        assert np.array_equal(ep, oep) and np.array_equal(em, oem)
+    R.close()

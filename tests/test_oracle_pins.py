@@ -471,6 +471,31 @@ def test_boundary_mask_diagonal():
     assert got == diag | top | left
 
 
+def _sliver_polys():
+    """A quad whose right edge is nearly vertical (dx = 3 lattice units over
+    800 world units, 2^-20 world units per lattice unit on the C1 domain) and
+    whose top edge is nearly horizontal (dy = 3 units): in every pixel row /
+    column its x- (y-) extent lies strictly between two consecutive lattice
+    values inside ONE pixel's extent (the full-size C3 finding of round 2)."""
+    u = 2.0 ** -20
+    return [[np.array([(200.0, 100.0), (300.0 + u, 100.0), (300.0 + 4 * u, 900.0 + u), (200.0, 900.0 + 4 * u)], float)]]
+
+
+def test_boundary_mask_nearly_axis_parallel_edges():
+    """O9 on edges that never cross a lattice column (row) inside a pixel
+    row (column): the closed pixel rectangles they pass through are the
+    boundary pixels -- pixel column 300 on every row 100..900 (the right
+    edge) and pixel row 900 on every column 200..300 (the top edge), closed
+    form at 1024^2 where pixel i spans lattice [i 2^20, (i+1) 2^20 - 1]."""
+    polys = oracle.Polys(PG.flatten(_sliver_polys()), C1)
+    m = oracle.boundary_mask(polys, 1024, 1024)
+    bits = np.unpackbits(m.view(np.uint8), bitorder="little").reshape(1024, -1)[:, :1024].astype(bool)
+    assert bits[100:901, 300].all()                 # right edge: every row of its extent
+    assert bits[900, 200:301].all()                 # top edge: every column
+    assert bits[100:901, 200].all() and bits[100, 200:301].all()
+    assert bits.sum() == 801 + 801 + 101 + 101 - 4
+
+
 def test_boundary_mask_brute_force_tiny():
     # brute force over every lattice point of a tiny domain: a pixel is a
     # boundary pixel iff some lattice point of it lies on an edge, or its

@@ -3,6 +3,7 @@
 // point pass (S2/S7 + S4) -> S8 finalise.  All device work is in the
 // kernels of this library; there is no CPU fallback.
 #include <algorithm>
+#include <cstdlib>
 #include <cmath>
 #include <cstring>
 #include <new>
@@ -387,10 +388,7 @@ static rj_status run_pass(Ctx *c, Prepared &P, unsigned long long *d_cnt, double
     a.A_sum = d_sum;
     rj_status s = setup_bqueue(c, P);
     if (s != RJ_OK) return s;
-    RJ_CUDA(c, cudaMemsetAsync(a.work_counter, 0, 64, c->stream));
-    RJ_CUDA(c, cudaMemsetAsync(a.bq_valid, 0xFF, 4, c->stream));
-    RJ_CUDA(c, cudaMemsetAsync(d_cnt, 0, (size_t)c->n_poly * 8, c->stream));
-    if (P.sum) RJ_CUDA(c, cudaMemsetAsync(d_sum, 0, (size_t)c->n_poly * 8, c->stream));
+    RJ_CUDA(c, launch_pass_init(c, a.work_counter, d_cnt, P.sum ? d_sum : nullptr, c->n_poly));
     s = point_pass(c, a, P.sum, P.acc);
     if (s != RJ_OK) return s;
     if (a.bq_cap && (s = pip_queue_pass(c, a, P.sum)) != RJ_OK) return s;
@@ -693,6 +691,7 @@ rj_status rj_create(rj_ctx **out, int32_t dev, void *stream, double x0, double y
         c->own_stream = true;
     }
     if (cudaMallocHost(&c->h_stats, 64 * sizeof(unsigned long long)) != cudaSuccess) { delete c; return RJ_ERR_CUDA; }
+    if (const char *e = std::getenv("RJ_NO_PDL")) c->pdl = (e[0] == '1') ? 0 : 1;
     for (auto &e : c->ev)
         if (cudaEventCreate(&e) != cudaSuccess) { delete c; return RJ_ERR_CUDA; }
     *out = c;

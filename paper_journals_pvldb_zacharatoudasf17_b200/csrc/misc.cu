@@ -9,11 +9,28 @@ namespace rj {
 namespace {
 __global__ void k_finalize(int agg, uint32_t n, const unsigned long long *__restrict__ cnt,
                            const double *__restrict__ sum, double *__restrict__ val) {
+    pdl_wait();
+    pdl_trigger();
     const uint32_t i = blockIdx.x * blockDim.x + threadIdx.x;
     if (i >= n) return;
     if (agg == RJ_AVG) val[i] = cnt[i] ? __ddiv_rn(sum[i], (double)cnt[i]) : __longlong_as_double(0x7ff8000000000000ll);
     else if (agg == RJ_SUM) val[i] = sum[i];
     else val[i] = (double)cnt[i];
+}
+
+// Per-query reset before the point pass (one PDL-chained kernel instead of
+// four memset nodes): work counters and statistics, the boundary queue's
+// valid mark (all ones), the per-polygon partials.
+__global__ void k_pass_init(uint32_t *__restrict__ work, unsigned long long *__restrict__ cnt, double *__restrict__ sum,
+                            uint32_t n) {
+    pdl_wait();
+    pdl_trigger();
+    const uint32_t t0 = blockIdx.x * blockDim.x + threadIdx.x, ts = gridDim.x * blockDim.x;
+    if (t0 < 16) work[t0] = t0 == 9 ? 0xFFFFFFFFu : 0u;
+    for (uint32_t i = t0; i < n; i += ts) {
+        cnt[i] = 0ull;
+        if (sum) sum[i] = 0.0;
+    }
 }
 
 // Multi-GPU combine (S8): counts and sums in one binary64 buffer, so one
@@ -111,9 +128,16 @@ __global__ void k_membership(const PassArgs a, uint64_t n, int accurate, const u
 cudaError_t launch_finalize(Ctx *c, int agg, uint32_t n, const unsigned long long *cnt, const double *sum,
                             double *val) {
     if (!n) return cudaSuccess;
-    k_finalize<<<blocks_for(n, 256), 256, 0, c->stream>>>(agg, n, cnt, sum, val);
+    const cudaError_t e = launch_pdl(c, k_finalize, dim3(blocks_for(n, 256)), dim3(256), 0, agg, n, cnt, sum, val);
     RJ_LAUNCHED(c);
-    return cudaGetLastError();
+    return e;
+}
+
+cudaError_t launch_pass_init(Ctx *c, uint32_t *work, unsigned long long *cnt, double *sum, uint32_t n) {
+    const unsigned g = std::max(1u, std::min(blocks_for(n, 256), (unsigned)c->num_sms));
+    const cudaError_t e = launch_pdl(c, k_pass_init, dim3(g), dim3(256), 0, work, cnt, sum, n);
+    RJ_LAUNCHED(c);
+    return e;
 }
 
 cudaError_t launch_pack(Ctx *c, uint32_t n, const unsigned long long *cnt, const double *sum, double *out) {

@@ -167,6 +167,10 @@ __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a)
         for (uint32_t kk = threadIdx.x; kk < a.n_poly; kk += blockDim.x) {
             sh.pcnt[kk] = 0;
         }
+    // everything above is CTA-local setup; the work counter, the polygon
+    // pass's pieces and the partial vectors are the predecessors' output
+    pdl_wait();
+    pdl_trigger();
     __syncthreads();
 
     if (wid == kWarps) {
@@ -297,6 +301,8 @@ __global__ void __launch_bounds__(256) k_pip_queue(const __grid_constant__ PassA
     sh.pcnt = reinterpret_cast<uint32_t *>(smem_raw);
     if (a.smem_partials)
         for (uint32_t k = threadIdx.x; k < a.n_poly; k += blockDim.x) sh.pcnt[k] = 0;
+    pdl_wait();
+    pdl_trigger();
     __syncthreads();
     const uint32_t n = min(*a.bq_count, *a.bq_valid);
     const int lane = threadIdx.x & 31;
@@ -415,7 +421,7 @@ rj_status launch_pass(Ctx *c, void *k, const PassArgs &a, size_t smem) {
     const unsigned grid = (unsigned)std::max<uint64_t>(
         1, std::min<uint64_t>((uint64_t)per_sm * c->num_sms, std::max<uint32_t>(1, a.n_items)));
     void *args[] = {(void *)&a};
-    RJ_CUDA(c, cudaLaunchKernel(k, dim3(grid), dim3(kThreads + 32), args, smem, c->stream));
+    RJ_CUDA(c, launch_pdl_ptr(c, k, dim3(grid), dim3(kThreads + 32), smem, args));
     RJ_LAUNCHED(c);
     c->last_stages = (int)a.n_stages;
     c->last_ctas_per_sm = per_sm;
@@ -447,7 +453,7 @@ rj_status pip_queue_pass(Ctx *c, const PassArgs &a_in, bool sum) {
     RJ_CUDA(c, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, k, 256, smem));
     const unsigned grid = (unsigned)std::max(1, per_sm) * (unsigned)c->num_sms;
     void *args[] = {(void *)&a};
-    RJ_CUDA(c, cudaLaunchKernel(k, dim3(grid), dim3(256), args, smem, c->stream));
+    RJ_CUDA(c, launch_pdl_ptr(c, k, dim3(grid), dim3(256), smem, args));
     RJ_LAUNCHED(c);
     return RJ_OK;
 }

@@ -222,6 +222,8 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
         for (uint32_t kk = threadIdx.x; kk < a.n_poly; kk += blockDim.x) {
             sh.pcnt[kk] = 0;
         }
+    pdl_wait();                                             // predecessors' output from here on
+    pdl_trigger();
     __syncthreads();
 
     if (wid == kWarps) {

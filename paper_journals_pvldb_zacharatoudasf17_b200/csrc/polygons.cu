@@ -177,14 +177,6 @@ __device__ __forceinline__ void edge_rows_body(uint32_t t0, uint32_t ts, const i
     }
 }
 
-__global__ void k_edge_rows(const int4 *__restrict__ edges, const uint32_t *__restrict__ edge_poly,
-                            const int4 *__restrict__ mbr, uint32_t n_edges, int H,
-                            uint32_t *__restrict__ rows, int accurate, int W,
-                            uint32_t *__restrict__ bands, int4 view) {
-    edge_rows_body(blockIdx.x * blockDim.x + threadIdx.x, gridDim.x * blockDim.x, edges, edge_poly, mbr, n_edges, H,
-                   rows, accurate, W, bands, view);
-}
-
 __device__ __forceinline__ void poly_rows_body(uint32_t t0, uint32_t ts, const int4 *__restrict__ mbr,
                                                uint32_t n_poly, int W, int H, uint32_t *__restrict__ rows,
                                                int4 view) {
@@ -192,11 +184,6 @@ __device__ __forceinline__ void poly_rows_body(uint32_t t0, uint32_t ts, const i
         const int4 M = mbr[p];
         rows[p] = culled(M, W, H, view) ? 0u : (uint32_t)(row_start(M.w, H) - row_start(M.y, H));
     }
-}
-
-__global__ void k_poly_rows(const int4 *__restrict__ mbr, uint32_t n_poly, int W, int H, uint32_t *__restrict__ rows,
-                            int4 view) {
-    poly_rows_body(blockIdx.x * blockDim.x + threadIdx.x, gridDim.x * blockDim.x, mbr, n_poly, W, H, rows, view);
 }
 
 __device__ __forceinline__ void crossings_body(uint32_t t0, uint32_t ts, const int4 *__restrict__ edges, const uint32_t *__restrict__ edge_poly,
@@ -219,11 +206,13 @@ __device__ __forceinline__ void crossings_body(uint32_t t0, uint32_t ts, const i
     }
 }
 
-__global__ void k_crossings(const int4 *__restrict__ edges, const uint32_t *__restrict__ edge_poly,
+__global__ void __launch_bounds__(256) k_crossings(const int4 *__restrict__ edges, const uint32_t *__restrict__ edge_poly,
                             const int4 *__restrict__ mbr, const uint32_t *__restrict__ edge_off,
                             uint32_t n_edges, const uint32_t *__restrict__ prow_off, int W, int H,
                             uint32_t *__restrict__ cx_pr, uint32_t *__restrict__ cx_t,
                             uint32_t *__restrict__ pr_cnt) {
+    pdl_wait();
+    pdl_trigger();
     crossings_body(blockIdx.x * blockDim.x + threadIdx.x, gridDim.x * blockDim.x, edges, edge_poly, mbr, edge_off, n_edges, prow_off, W, H, cx_pr, cx_t, pr_cnt);
 }
 
@@ -239,6 +228,8 @@ __device__ __forceinline__ void scatter_t_body(uint32_t t0, uint32_t ts, const u
 __global__ void k_scatter_t(const uint32_t *__restrict__ cx_pr, const uint32_t *__restrict__ cx_t,
                             uint32_t total, const uint32_t *__restrict__ pr_off,
                             uint32_t *__restrict__ pr_cur, uint32_t *__restrict__ tv) {
+    pdl_wait();
+    pdl_trigger();
     scatter_t_body(blockIdx.x * blockDim.x + threadIdx.x, gridDim.x * blockDim.x, cx_pr, cx_t, total, pr_off, pr_cur, tv);
 }
 
@@ -344,12 +335,6 @@ __device__ __forceinline__ void prow_count_body(uint32_t t0, uint32_t ts, SpanGe
     }
 }
 
-__global__ void k_prow_count(SpanGeo g, uint32_t n_prow, const uint32_t *__restrict__ pr_off,
-                             uint32_t *__restrict__ tv, uint32_t *__restrict__ span_cnt,
-                             uint32_t *__restrict__ piece_cnt) {
-    prow_count_body(blockIdx.x * blockDim.x + threadIdx.x, gridDim.x * blockDim.x, g, n_prow, pr_off, tv, span_cnt, piece_cnt);
-}
-
 __device__ __forceinline__ void prow_emit_body(uint32_t t0, uint32_t ts, SpanGeo g, uint32_t n_prow, const uint32_t *__restrict__ pr_off,
                             const uint32_t *__restrict__ tv, const uint32_t *__restrict__ span_off,
                             uint32_t *__restrict__ spans, const uint32_t *__restrict__ piece_off,
@@ -389,13 +374,6 @@ __device__ __forceinline__ void prow_emit_body(uint32_t t0, uint32_t ts, SpanGeo
             if (nb) flush();
         }
     }
-}
-
-__global__ void k_prow_emit(SpanGeo g, uint32_t n_prow, const uint32_t *__restrict__ pr_off,
-                            const uint32_t *__restrict__ tv, const uint32_t *__restrict__ span_off,
-                            uint32_t *__restrict__ spans, const uint32_t *__restrict__ piece_off,
-                            uint32_t *__restrict__ piece_cur, uint2 *__restrict__ pieces) {
-    prow_emit_body(blockIdx.x * blockDim.x + threadIdx.x, gridDim.x * blockDim.x, g, n_prow, pr_off, tv, span_off, spans, piece_off, piece_cur, pieces);
 }
 
 // -------------------------------------------------------------- S5 supercover
@@ -449,11 +427,62 @@ __device__ __forceinline__ void bnd_pieces_body(uint32_t t0, uint32_t ts, SpanGe
     }
 }
 
+// ---- the polygon pass as a chain of PDL-launched kernels (pdl_wait first)
+// rows per edge (+ S5 bands) and per polygon, window-culled
+__global__ void k_rows(const int4 *__restrict__ edges, const uint32_t *__restrict__ edge_poly,
+                       const int4 *__restrict__ mbr, uint32_t n_edges, uint32_t n_poly, int W, int H, int accurate,
+                       uint32_t *__restrict__ erows, uint32_t *__restrict__ bands, uint32_t *__restrict__ prows,
+                       int4 view) {
+    pdl_wait();
+    pdl_trigger();
+    const uint32_t t0 = blockIdx.x * blockDim.x + threadIdx.x, ts = gridDim.x * blockDim.x;
+    edge_rows_body(t0, ts, edges, edge_poly, mbr, n_edges, H, erows, accurate, W, bands, view);
+    poly_rows_body(t0, ts, mbr, n_poly, W, H, prows, view);
+}
+
+// zero up to four counter arrays of n[k] + 1 words
+struct ZeroJobs {
+    uint32_t *p[4];
+    uint64_t n[4];
+};
+__global__ void k_zero(const ZeroJobs z) {
+    pdl_wait();
+    pdl_trigger();
+    const uint64_t t0 = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x, ts = (uint64_t)gridDim.x * blockDim.x;
+    for (int k = 0; k < 4; ++k)
+        if (z.p[k])
+            for (uint64_t i = t0; i <= z.n[k]; i += ts) z.p[k][i] = 0u;
+}
+
+// per (polygon, row): sort, count spans and per-cell pieces
+__global__ void k_count(SpanGeo g, uint32_t n_prow, const uint32_t *__restrict__ pr_off, uint32_t *__restrict__ tv,
+                        uint32_t *__restrict__ span_cnt, uint32_t *__restrict__ piece_cnt) {
+    pdl_wait();
+    pdl_trigger();
+    prow_count_body(blockIdx.x * blockDim.x + threadIdx.x, gridDim.x * blockDim.x, g, n_prow, pr_off, tv, span_cnt,
+                    piece_cnt);
+}
+
+// spans and their pieces per cell
+__global__ void k_emit(SpanGeo g, uint32_t n_prow, const uint32_t *__restrict__ pr_off, const uint32_t *__restrict__ tv,
+                       const uint32_t *__restrict__ span_off, uint32_t *__restrict__ spans,
+                       const uint32_t *__restrict__ piece_off, uint32_t *__restrict__ piece_cur,
+                       uint2 *__restrict__ pieces) {
+    pdl_wait();
+    pdl_trigger();
+    prow_emit_body(blockIdx.x * blockDim.x + threadIdx.x, gridDim.x * blockDim.x, g, n_prow, pr_off, tv, span_off,
+                   spans, piece_off, piece_cur, pieces);
+}
+
+// accurate mode: boundary pieces per cell (count pass / emit pass)
 template <bool EMIT>
-__global__ void k_bnd_pieces(SpanGeo g, const int4 *__restrict__ edges, const uint32_t *__restrict__ band_off,
-                             uint32_t n_edges, uint32_t *__restrict__ cnt, const uint32_t *__restrict__ off,
-                             uint32_t *__restrict__ cur, uint32_t *__restrict__ out) {
-    bnd_pieces_body<EMIT>(blockIdx.x * blockDim.x + threadIdx.x, gridDim.x * blockDim.x, g, edges, band_off, n_edges, cnt, off, cur, out);
+__global__ void k_bnd(SpanGeo g, const int4 *__restrict__ edges, const uint32_t *__restrict__ band_off,
+                      uint32_t n_edges, uint32_t *__restrict__ cnt, const uint32_t *__restrict__ off,
+                      uint32_t *__restrict__ cur, uint32_t *__restrict__ out) {
+    pdl_wait();
+    pdl_trigger();
+    bnd_pieces_body<EMIT>(blockIdx.x * blockDim.x + threadIdx.x, gridDim.x * blockDim.x, g, edges, band_off, n_edges,
+                          cnt, off, cur, out);
 }
 
 }  // namespace
@@ -633,16 +662,18 @@ rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp,
     const int4 vw = v.full ? make_int4(0, 0, W, H) : make_int4(v.c0, v.r0, v.c1, v.r1);
     const int64_t key[9] = {W, H, L, accurate ? 1 : 0, vw.x, vw.y, vw.z, vw.w, (int64_t)c->data_gen};
     const bool known = c->pp_key_valid && std::equal(key, key + 9, c->pp_key);
-    k_edge_rows<<<blocks_for(ne, 256), 256, 0, st>>>(c->edges.as<int4>(), c->edge_poly.as<uint32_t>(),
-                                                     c->mbr.as<int4>(), ne, H, erows.as<uint32_t>(), accurate, W,
-                                                     bcnt.as<uint32_t>(), vw);
+    const unsigned gr = (unsigned)std::min<uint64_t>(std::max<uint64_t>(1, blocks_for(std::max(ne, np), 256)),
+                                                     c->num_sms * 8ull);
+    RJ_CUDA(c, launch_pdl(c, k_rows, dim3(gr), dim3(256), 0, c->edges.as<int4>(), c->edge_poly.as<uint32_t>(),
+                          c->mbr.as<int4>(), ne, np, W, H, accurate ? 1 : 0, erows.as<uint32_t>(), bcnt.as<uint32_t>(),
+                          prows.as<uint32_t>(), vw));
     RJ_LAUNCHED(c);
-    k_poly_rows<<<blocks_for(np, 256), 256, 0, st>>>(c->mbr.as<int4>(), np, W, H, prows.as<uint32_t>(), vw);
-    RJ_LAUNCHED(c);
-    RJ_CUDA(c, cudaGetLastError());
-    RJ_CUDA(c, scan_u32(c, erows.as<uint32_t>(), eoff.as<uint32_t>(), ne, kWsScan));
-    RJ_CUDA(c, scan_u32(c, prows.as<uint32_t>(), proff.as<uint32_t>(), np, kWsScan));
-    if (accurate) RJ_CUDA(c, scan_u32(c, bcnt.as<uint32_t>(), boff.as<uint32_t>(), ne, kWsScan));
+    {
+        const uint32_t *in[3] = {erows.as<uint32_t>(), prows.as<uint32_t>(), bcnt.as<uint32_t>()};
+        uint32_t *out[3] = {eoff.as<uint32_t>(), proff.as<uint32_t>(), boff.as<uint32_t>()};
+        const uint64_t n[3] = {ne, np, ne};
+        RJ_CUDA(c, scan_multi(c, accurate ? 3 : 2, in, out, n, kWsScan));
+    }
     // sync 1: crossing / polygon-row / band totals (skipped for a repeated key)
     uint32_t *hs = reinterpret_cast<uint32_t *>(c->h_stats + 8);
     if (known) {
@@ -661,50 +692,63 @@ rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp,
     Buf &pro = wsbuf(c, kWsPROff), &prcur = wsbuf(c, kWsPRCursor), &tv = wsbuf(c, kWsTvals);
     Buf &scnt = wsbuf(c, kWsSpanCount), &soff = wsbuf(c, kWsSpanOff);
     Buf &pcnt = wsbuf(c, kWsPieceCount), &poff = wsbuf(c, kWsPieceOff), &pcur = wsbuf(c, kWsPieceCursor);
+    Buf &bpc = wsbuf(c, kWsBPCount), &bpo = wsbuf(c, kWsBPOff), &bpu = wsbuf(c, kWsBPCursor);
+    const bool bnd_pieces = accurate && ncell;               // accurate mode with point cells
     if (dreserve(c, cpr, (X + 1) * 4) || dreserve(c, ct, (X + 1) * 4) || dreserve(c, prc, (NPR + 1) * 4) ||
         dreserve(c, pro, (NPR + 1) * 4) || dreserve(c, prcur, (NPR + 1) * 4) || dreserve(c, tv, (X + 1) * 4) ||
         dreserve(c, scnt, (NPR + 1) * 4) || dreserve(c, soff, (NPR + 1) * 4) ||
         dreserve(c, pcnt, (ncell + 1) * 4) || dreserve(c, poff, (ncell + 1) * 4) ||
-        dreserve(c, pcur, (ncell + 1) * 4))
+        dreserve(c, pcur, (ncell + 1) * 4) ||
+        (bnd_pieces && (dreserve(c, bpc, (ncell + 1) * 4) || dreserve(c, bpo, (ncell + 1) * 4) ||
+                        dreserve(c, bpu, (ncell + 1) * 4))))
         return set_error(c, RJ_ERR_OOM, "workspace allocation failed");
-    RJ_CUDA(c, cudaMemsetAsync(prc.p, 0, (NPR + 1) * 4, st));
-    RJ_CUDA(c, cudaMemsetAsync(prcur.p, 0, (NPR + 1) * 4, st));
-    RJ_CUDA(c, cudaMemsetAsync(pcnt.p, 0, (ncell + 1) * 4, st));
-    RJ_CUDA(c, cudaMemsetAsync(pcur.p, 0, (ncell + 1) * 4, st));
+    {
+        // counters: (polygon,row) counts + cursors, per-cell piece counts + cursors
+        // (cursors follow counts in one allocation-free kernel)
+        ZeroJobs z{};
+        z.p[0] = prc.as<uint32_t>(); z.n[0] = NPR;
+        z.p[1] = prcur.as<uint32_t>(); z.n[1] = NPR;
+        z.p[2] = pcnt.as<uint32_t>(); z.n[2] = ncell;
+        z.p[3] = pcur.as<uint32_t>(); z.n[3] = ncell;
+        const unsigned gz = (unsigned)std::min<uint64_t>(std::max<uint64_t>(1, blocks_for(std::max<uint64_t>(NPR, ncell) + 1, 256)),
+                                                         c->num_sms * 8ull);
+        RJ_CUDA(c, launch_pdl(c, k_zero, dim3(gz), dim3(256), 0, z));
+        RJ_LAUNCHED(c);
+        if (bnd_pieces) {
+            ZeroJobs zb{};
+            zb.p[0] = bpc.as<uint32_t>(); zb.n[0] = ncell;
+            zb.p[1] = bpu.as<uint32_t>(); zb.n[1] = ncell;
+            RJ_CUDA(c, launch_pdl(c, k_zero, dim3(gz), dim3(256), 0, zb));
+            RJ_LAUNCHED(c);
+        }
+    }
     const unsigned gx = (unsigned)std::min<uint64_t>(std::max<uint64_t>(1, blocks_for(X, 256)), c->num_sms * 8ull);
-    k_crossings<<<gx, 256, 0, st>>>(c->edges.as<int4>(), c->edge_poly.as<uint32_t>(), c->mbr.as<int4>(),
-                                    eoff.as<uint32_t>(), ne, proff.as<uint32_t>(), W, H, cpr.as<uint32_t>(),
-                                    ct.as<uint32_t>(), prc.as<uint32_t>());
+    RJ_CUDA(c, launch_pdl(c, k_crossings, dim3(gx), dim3(256), 0, c->edges.as<int4>(), c->edge_poly.as<uint32_t>(),
+                          c->mbr.as<int4>(), eoff.as<uint32_t>(), ne, proff.as<uint32_t>(), W, H, cpr.as<uint32_t>(),
+                          ct.as<uint32_t>(), prc.as<uint32_t>()));
     RJ_LAUNCHED(c);
-    RJ_CUDA(c, cudaGetLastError());
     RJ_CUDA(c, scan_u32(c, prc.as<uint32_t>(), pro.as<uint32_t>(), NPR, kWsScan));
-    k_scatter_t<<<gx, 256, 0, st>>>(cpr.as<uint32_t>(), ct.as<uint32_t>(), X, pro.as<uint32_t>(),
-                                    prcur.as<uint32_t>(), tv.as<uint32_t>());
+    RJ_CUDA(c, launch_pdl(c, k_scatter_t, dim3(gx), dim3(256), 0, cpr.as<uint32_t>(), ct.as<uint32_t>(), X,
+                          pro.as<uint32_t>(), prcur.as<uint32_t>(), tv.as<uint32_t>()));
     RJ_LAUNCHED(c);
     SpanGeo g{W, H, L, proff.as<uint32_t>(), np, c->mbr.as<int4>(), L >= 0 ? c->cell_bits[L].as<uint32_t>() : nullptr,
               v.full ? 0 : v.c0, v.full ? 0 : v.r0, v.full ? W : v.c1, v.full ? H : v.r1};
-    const unsigned gp = (unsigned)std::min<uint64_t>(std::max<uint64_t>(1, blocks_for(NPR, 128)), c->num_sms * 16ull);
-    k_prow_count<<<gp, 128, 0, st>>>(g, NPR, pro.as<uint32_t>(), tv.as<uint32_t>(), scnt.as<uint32_t>(),
-                                     pcnt.as<uint32_t>());
-    RJ_LAUNCHED(c);
-    RJ_CUDA(c, cudaGetLastError());
-    RJ_CUDA(c, scan_u32(c, scnt.as<uint32_t>(), soff.as<uint32_t>(), NPR, kWsScan));
-    if (ncell) RJ_CUDA(c, scan_u32(c, pcnt.as<uint32_t>(), poff.as<uint32_t>(), ncell, kWsScan));
-    // accurate mode with point cells: boundary pieces (count pass)
-    const bool bnd_pieces = accurate && ncell;
     const uint32_t B = accurate ? hs[2] : 0;
-    Buf &bpc = wsbuf(c, kWsBPCount), &bpo = wsbuf(c, kWsBPOff), &bpu = wsbuf(c, kWsBPCursor);
+    const unsigned gp = (unsigned)std::min<uint64_t>(std::max<uint64_t>(1, blocks_for(NPR, 128)), c->num_sms * 16ull);
     const unsigned gb = (unsigned)std::min<uint64_t>(std::max<uint64_t>(1, blocks_for(B, 256)), c->num_sms * 8ull);
+    RJ_CUDA(c, launch_pdl(c, k_count, dim3(gp), dim3(128), 0, g, NPR, pro.as<uint32_t>(), tv.as<uint32_t>(),
+                          scnt.as<uint32_t>(), pcnt.as<uint32_t>()));
+    RJ_LAUNCHED(c);
     if (bnd_pieces) {
-        if (dreserve(c, bpc, (ncell + 1) * 4) || dreserve(c, bpo, (ncell + 1) * 4) || dreserve(c, bpu, (ncell + 1) * 4))
-            return set_error(c, RJ_ERR_OOM, "workspace allocation failed");
-        RJ_CUDA(c, cudaMemsetAsync(bpc.p, 0, (ncell + 1) * 4, st));
-        RJ_CUDA(c, cudaMemsetAsync(bpu.p, 0, (ncell + 1) * 4, st));
-        k_bnd_pieces<false><<<gb, 256, 0, st>>>(g, c->edges.as<int4>(), boff.as<uint32_t>(), ne, bpc.as<uint32_t>(),
-                                                nullptr, nullptr, nullptr);
+        RJ_CUDA(c, launch_pdl(c, k_bnd<false>, dim3(gb), dim3(256), 0, g, c->edges.as<int4>(), boff.as<uint32_t>(), ne,
+                              bpc.as<uint32_t>(), (const uint32_t *)nullptr, (uint32_t *)nullptr, (uint32_t *)nullptr));
         RJ_LAUNCHED(c);
-        RJ_CUDA(c, cudaGetLastError());
-        RJ_CUDA(c, scan_u32(c, bpc.as<uint32_t>(), bpo.as<uint32_t>(), ncell, kWsScan));
+    }
+    {
+        const uint32_t *in[3] = {scnt.as<uint32_t>(), pcnt.as<uint32_t>(), bpc.as<uint32_t>()};
+        uint32_t *out[3] = {soff.as<uint32_t>(), poff.as<uint32_t>(), bpo.as<uint32_t>()};
+        const uint64_t n[3] = {NPR, ncell, ncell};
+        RJ_CUDA(c, scan_multi(c, ncell ? (bnd_pieces ? 3 : 2) : 1, in, out, n, kWsScan));
     }
     // sync 2: span / piece totals (skipped for a repeated key)
     if (!known) {
@@ -719,27 +763,25 @@ rj_status polygon_pass(Ctx *c, int W, int H, int L, bool accurate, PolyPass &pp,
         c->pp_key_valid = true;
     }
     const uint32_t S = hs[3], NP = hs[4], NB = hs[5];
-    Buf &spans = wsbuf(c, kWsSpans), &pieces = wsbuf(c, kWsPieces);
-    if (dreserve(c, spans, (uint64_t)(S + 1) * 16) || dreserve(c, pieces, (uint64_t)(NP + 1) * 8))
+    Buf &spans = wsbuf(c, kWsSpans), &pieces = wsbuf(c, kWsPieces), &bp = wsbuf(c, kWsBPieces);
+    if (dreserve(c, spans, (uint64_t)(S + 1) * 16) || dreserve(c, pieces, (uint64_t)(NP + 1) * 8) ||
+        (bnd_pieces && dreserve(c, bp, (uint64_t)(NB + 1) * 4)))
         return set_error(c, RJ_ERR_OOM, "workspace allocation failed");
-    k_prow_emit<<<gp, 128, 0, st>>>(g, NPR, pro.as<uint32_t>(), tv.as<uint32_t>(), soff.as<uint32_t>(),
-                                    spans.as<uint32_t>(), poff.as<uint32_t>(), pcur.as<uint32_t>(),
-                                    pieces.as<uint2>());
+    RJ_CUDA(c, launch_pdl(c, k_emit, dim3(gp), dim3(128), 0, g, NPR, pro.as<uint32_t>(), tv.as<uint32_t>(),
+                          soff.as<uint32_t>(), spans.as<uint32_t>(), poff.as<uint32_t>(), pcur.as<uint32_t>(),
+                          pieces.as<uint2>()));
     RJ_LAUNCHED(c);
-    RJ_CUDA(c, cudaGetLastError());
-
     if (bnd_pieces) {
-        Buf &bp = wsbuf(c, kWsBPieces);
-        if (dreserve(c, bp, (uint64_t)(NB + 1) * 4)) return set_error(c, RJ_ERR_OOM, "workspace allocation failed");
-        k_bnd_pieces<true><<<gb, 256, 0, st>>>(g, c->edges.as<int4>(), boff.as<uint32_t>(), ne, nullptr,
-                                               bpo.as<uint32_t>(), bpu.as<uint32_t>(), bp.as<uint32_t>());
+        RJ_CUDA(c, launch_pdl(c, k_bnd<true>, dim3(gb), dim3(256), 0, g, c->edges.as<int4>(), boff.as<uint32_t>(), ne,
+                              (uint32_t *)nullptr, (const uint32_t *)bpo.as<uint32_t>(), bpu.as<uint32_t>(),
+                              bp.as<uint32_t>()));
         RJ_LAUNCHED(c);
-        RJ_CUDA(c, cudaGetLastError());
+    }
+    if (bnd_pieces) {
         pp.bpiece_off = bpo.as<uint32_t>();
         pp.bpieces = bp.as<uint32_t>();
         pp.n_bpieces = NB;
     }
-
     pp.n_cross = X;
     pp.n_spans = S;
     pp.n_pieces = NP;

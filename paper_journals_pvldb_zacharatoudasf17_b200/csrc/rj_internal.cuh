@@ -1,5 +1,6 @@
 // rj_internal.cuh -- private context and launcher declarations of librj.
 #pragma once
+#include <utility>
 #include <cuda_runtime.h>
 #include <stdint.h>
 
@@ -147,6 +148,7 @@ struct Ctx {
     uint64_t alloc_gen = 0;                    // bumped by every device (re)allocation / free
     bool capturing = false;
     int use_graphs = 1;                        // RJ_OPT_GRAPHS
+    int pdl = 1;                               // programmatic dependent launch of the query's kernel chain (env RJ_NO_PDL=1: off)
     std::vector<int64_t> graph_key, pending_key;
     cudaGraphExec_t graph_exec = nullptr;
     rj_stats graph_last{};
@@ -204,6 +206,16 @@ Buf &wsbuf(Ctx *c, int slot);
 // scan.cu: exclusive scan of n u32 -> out[0..n], out[n] = total.  tmp
 // workspace slots base.. are used for block sums.
 cudaError_t scan_u32(Ctx *c, const uint32_t *in, uint32_t *out, uint64_t n, int ws_base);
+// up to three independent scans in one launch (out[j][n[j]] = total of array j)
+struct ScanJobs {
+    const uint32_t *in[3];
+    uint32_t *out[3];
+    uint64_t n[3];
+    uint32_t tile0[4];       // first global tile of each array; tile0[nj] = all tiles
+    int nj;
+};
+cudaError_t scan_multi(Ctx *c, int nj, const uint32_t *const *in, uint32_t *const *out, const uint64_t *n,
+                       int ws_base);
 
 // load_points.cu
 rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int xy_f64,
@@ -287,6 +299,7 @@ int point_pass_stages(int n_slots);
 // misc.cu
 cudaError_t launch_finalize(Ctx *c, int agg, uint32_t n, const unsigned long long *cnt,
                             const double *sum, double *val);
+cudaError_t launch_pass_init(Ctx *c, uint32_t *work, unsigned long long *cnt, double *sum, uint32_t n);
 cudaError_t launch_pack(Ctx *c, uint32_t n, const unsigned long long *cnt, const double *sum, double *out);
 cudaError_t launch_finalize_packed(Ctx *c, int agg, uint32_t n, const double *in, unsigned long long *cnt,
                                    double *val);
@@ -302,6 +315,45 @@ rj_status cuda_error(Ctx *c, cudaError_t e, const char *where);
     } while (0)
 
 #define RJ_LAUNCHED(c) do { (c)->launches++; } while (0)
+
+// Programmatic dependent launch: the per-query kernel chain (polygon pass ->
+// point pass -> finalisation) is launched with the PDL attribute, so a
+// kernel's grid is scheduled while its predecessor drains.  Every such
+// kernel first waits for its predecessor's completion and memory
+// (griddepcontrol.wait -- a no-op without the attribute), then lets its own
+// dependent launch.
+__device__ __forceinline__ void pdl_wait() { asm volatile("griddepcontrol.wait;" ::: "memory"); }
+__device__ __forceinline__ void pdl_trigger() { asm volatile("griddepcontrol.launch_dependents;" ::: "memory"); }
+
+// the same for a kernel given as a function pointer plus argument array
+inline cudaError_t launch_pdl_ptr(Ctx *c, const void *k, dim3 grid, dim3 block, size_t smem, void **args) {
+    cudaLaunchConfig_t cfg{};
+    cfg.gridDim = grid;
+    cfg.blockDim = block;
+    cfg.dynamicSmemBytes = smem;
+    cfg.stream = c->stream;
+    cudaLaunchAttribute at[1];
+    at[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+    at[0].val.programmaticStreamSerializationAllowed = c->pdl;
+    cfg.attrs = at;
+    cfg.numAttrs = 1;
+    return cudaLaunchKernelExC(&cfg, k, args);
+}
+
+template <typename... KArgs, typename... Args>
+cudaError_t launch_pdl(Ctx *c, void (*k)(KArgs...), dim3 grid, dim3 block, size_t smem, Args &&...args) {
+    cudaLaunchConfig_t cfg{};
+    cfg.gridDim = grid;
+    cfg.blockDim = block;
+    cfg.dynamicSmemBytes = smem;
+    cfg.stream = c->stream;
+    cudaLaunchAttribute at[1];
+    at[0].id = cudaLaunchAttributeProgrammaticStreamSerialization;
+    at[0].val.programmaticStreamSerializationAllowed = c->pdl;
+    cfg.attrs = at;
+    cfg.numAttrs = 1;
+    return cudaLaunchKernelEx(&cfg, k, std::forward<Args>(args)...);
+}
 
 inline unsigned blocks_for(uint64_t n, unsigned t) { return (unsigned)((n + t - 1) / t); }
 

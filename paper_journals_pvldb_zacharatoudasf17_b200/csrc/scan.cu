@@ -2,6 +2,8 @@
 // the path (radix-sort digit offsets, crossings, spans, pieces, edge grid).
 // Single pass with decoupled look-back, 256 threads x 16 elements per block.
 // out[n] receives the total; in == out (in place) is allowed.
+#include <algorithm>
+
 #include "rj_internal.cuh"
 
 namespace rj {
@@ -40,25 +42,36 @@ __device__ __forceinline__ uint32_t block_excl_scan(uint32_t v, uint32_t &total)
     return warp_tot[w] + inc - v;
 }
 
-// Single-pass scan with decoupled look-back: every block takes a ticket (so
-// all its predecessors are already resident), scans its 4096-element tile,
-// publishes the tile aggregate, then warp 0 walks back over the predecessors'
-// status words 32 at a time until it meets an inclusive prefix, and
-// publishes its own.  One memset + one launch per scan instead of a
-// recursive three-phase scan (the polygon pass runs six of them per query).
+// Single-pass scan with decoupled look-back over up to three arrays in ONE
+// launch: every block takes a ticket (so all its predecessors are already
+// resident), maps it to (array, tile), scans its 4096-element tile,
+// publishes the tile aggregate, then warp 0 walks back over the
+// predecessors' status words of the same array 32 at a time until it meets
+// an inclusive prefix, and publishes its own.  The status words reset
+// themselves: the last block to finish (a second counter) zeroes them, so a
+// scan needs no memset node -- consecutive polygon-pass kernels chain with
+// programmatic dependent launch (pdl_wait / pdl_trigger).
 constexpr unsigned long long kFlagAgg = 1ull << 32, kFlagInc = 2ull << 32;
 
 __device__ __forceinline__ unsigned long long ld_volatile(const unsigned long long *p) {
     return *reinterpret_cast<const volatile unsigned long long *>(p);
 }
 
-__global__ void __launch_bounds__(kScanThreads) k_scan_lb(const uint32_t *in, uint32_t *out, uint64_t n,
-                                                          unsigned long long *__restrict__ ws) {
+__global__ void __launch_bounds__(kScanThreads) k_scan_lb(const ScanJobs J, unsigned long long *__restrict__ ws) {
+    pdl_wait();
+    pdl_trigger();
     __shared__ uint32_t s_tile, s_excl;
-    unsigned long long *status = ws + 1;                  // ws[0]: ticket
+    __shared__ int s_last;
+    unsigned long long *status = ws + 2;                  // ws[0]: ticket, ws[1]: blocks done
     if (threadIdx.x == 0) s_tile = (uint32_t)atomicAdd(ws, 1ull);
     __syncthreads();
-    const uint32_t tile = s_tile;
+    const uint32_t gt = s_tile;
+    int j = 0;
+    while (j + 1 < J.nj && gt >= J.tile0[j + 1]) ++j;
+    const uint32_t tile = gt - J.tile0[j], ntiles = J.tile0[j + 1] - J.tile0[j];
+    const uint32_t *in = J.in[j];
+    uint32_t *out = J.out[j];
+    const uint64_t n = J.n[j];
     const uint64_t base = (uint64_t)tile * kScanTile + (uint64_t)threadIdx.x * kScanItems;
     uint32_t v[kScanItems];
     uint32_t sum = 0;
@@ -70,21 +83,22 @@ __global__ void __launch_bounds__(kScanThreads) k_scan_lb(const uint32_t *in, ui
     }
     uint32_t total;
     uint32_t pre = block_excl_scan(sum, total);
+    unsigned long long *st_j = status + J.tile0[j];
     if (tile == 0) {
         if (threadIdx.x == 0) {
-            atomicExch(&status[0], kFlagInc | total);
+            atomicExch(&st_j[0], kFlagInc | total);
             s_excl = 0;
         }
     } else if (threadIdx.x < 32) {
         const int lane = threadIdx.x;
-        if (lane == 0) atomicExch(&status[tile], kFlagAgg | total);
+        if (lane == 0) atomicExch(&st_j[tile], kFlagAgg | total);
         uint32_t excl = 0;
-        int64_t j = (int64_t)tile - 1;
+        int64_t jj = (int64_t)tile - 1;
         for (;;) {
-            const int64_t k = j - lane;
-            unsigned long long st = k >= 0 ? ld_volatile(&status[k]) : kFlagInc;
+            const int64_t k = jj - lane;
+            unsigned long long st = k >= 0 ? ld_volatile(&st_j[k]) : kFlagInc;
             while (__any_sync(0xffffffffu, (st >> 32) == 0))
-                if ((st >> 32) == 0) st = ld_volatile(&status[k]);
+                if ((st >> 32) == 0) st = ld_volatile(&st_j[k]);
             const unsigned inc = __ballot_sync(0xffffffffu, (st >> 32) == 2);
             const int first = inc ? __ffs(inc) - 1 : 32;
             uint32_t c = lane <= first ? (uint32_t)st : 0u;
@@ -92,10 +106,10 @@ __global__ void __launch_bounds__(kScanThreads) k_scan_lb(const uint32_t *in, ui
             for (int o = 16; o; o >>= 1) c += __shfl_xor_sync(0xffffffffu, c, o);
             excl += c;
             if (inc) break;
-            j -= 32;
+            jj -= 32;
         }
         if (lane == 0) {
-            atomicExch(&status[tile], kFlagInc | (excl + total));
+            atomicExch(&st_j[tile], kFlagInc | (excl + total));
             s_excl = excl;
         }
     }
@@ -106,28 +120,55 @@ __global__ void __launch_bounds__(kScanThreads) k_scan_lb(const uint32_t *in, ui
         const uint64_t i = base + k;
         if (i < n) out[i] = pre;
         pre += v[k];
-        if (i + 1 == n) out[n] = pre;
+    }
+    if (tile == ntiles - 1 && threadIdx.x == 0) out[n] = s_excl + total;
+    // the last block to finish (every look-back done) resets the status words
+    __syncthreads();
+    if (threadIdx.x == 0) {
+        __threadfence();
+        s_last = atomicAdd(&ws[1], 1ull) == (unsigned long long)J.tile0[J.nj] - 1;
+    }
+    __syncthreads();
+    if (s_last) {
+        __threadfence();
+        for (uint32_t k = threadIdx.x; k < J.tile0[J.nj]; k += kScanThreads) status[k] = 0ull;
+        if (threadIdx.x == 0) {
+            ws[0] = 0ull;
+            ws[1] = 0ull;
+        }
     }
 }
-
-__global__ void k_scan_zero(uint32_t *out) { out[0] = 0u; }
 }  // namespace
 
-cudaError_t scan_u32(Ctx *c, const uint32_t *in, uint32_t *out, uint64_t n, int ws_base) {
-    if (n == 0) {
-        k_scan_zero<<<1, 1, 0, c->stream>>>(out);
-        RJ_LAUNCHED(c);
-        return cudaGetLastError();
+cudaError_t scan_multi(Ctx *c, int nj, const uint32_t *const *in, uint32_t *const *out, const uint64_t *n,
+                       int ws_base) {
+    ScanJobs J{};
+    J.nj = nj;
+    J.tile0[0] = 0;
+    for (int j = 0; j < nj; ++j) {
+        J.in[j] = in[j];
+        J.out[j] = out[j];
+        J.n[j] = n[j];
+        J.tile0[j + 1] = J.tile0[j] + (uint32_t)std::max<uint64_t>(1, (n[j] + kScanTile - 1) / kScanTile);
     }
-    const uint64_t tiles = (n + kScanTile - 1) / kScanTile;
+    const uint32_t tiles = J.tile0[nj];
     Buf &ws = wsbuf(c, ws_base);
-    cudaError_t e = dreserve(c, ws, (tiles + 1) * sizeof(unsigned long long));
-    if (e != cudaSuccess) return e;
-    e = cudaMemsetAsync(ws.p, 0, (tiles + 1) * sizeof(unsigned long long), c->stream);
-    if (e != cudaSuccess) return e;
-    k_scan_lb<<<(unsigned)tiles, kScanThreads, 0, c->stream>>>(in, out, n, ws.as<unsigned long long>());
+    const size_t need = (tiles + 2) * sizeof(unsigned long long);
+    if (ws.bytes < need) {
+        // (re)allocated status words start at zero; from then on the scans
+        // leave them zero themselves
+        cudaError_t e = dreserve(c, ws, need);
+        if (e != cudaSuccess) return e;
+        e = cudaMemsetAsync(ws.p, 0, ws.bytes, c->stream);
+        if (e != cudaSuccess) return e;
+    }
+    cudaError_t e = launch_pdl(c, k_scan_lb, dim3(tiles), dim3(kScanThreads), 0, J, ws.as<unsigned long long>());
     RJ_LAUNCHED(c);
-    return cudaGetLastError();
+    return e;
+}
+
+cudaError_t scan_u32(Ctx *c, const uint32_t *in, uint32_t *out, uint64_t n, int ws_base) {
+    return scan_multi(c, 1, &in, &out, &n, ws_base);
 }
 
 }  // namespace rj

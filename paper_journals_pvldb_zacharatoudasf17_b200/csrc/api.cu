@@ -522,6 +522,16 @@ static void drop_graph(Ctx *c) {
 
 template <class F>
 static rj_status run_graphed(Ctx *c, std::vector<int64_t> key, F body) {
+    // the caller is capturing the context's stream into its own graph: the
+    // query's work becomes part of that graph (no internal graph; anything
+    // that would allocate or synchronise fails the capture loudly)
+    cudaStreamCaptureStatus cs = cudaStreamCaptureStatusNone;
+    if (cudaStreamIsCapturing(c->stream, &cs) == cudaSuccess && cs != cudaStreamCaptureStatusNone) {
+        c->capturing = true;
+        rj_status s = body();
+        c->capturing = false;
+        return s;
+    }
     if (c->use_graphs && c->graph_exec && key == c->graph_key) {
         RJ_CUDA(c, cudaGraphLaunch(c->graph_exec, c->stream));
         c->last = c->graph_last;

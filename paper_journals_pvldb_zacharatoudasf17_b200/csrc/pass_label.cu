@@ -270,10 +270,18 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
                 // polygon < MULTI < BND: a polygon claims NONE, a second
                 // polygon turns a polygon into MULTI (CAS, so a concurrent
                 // BND is never overwritten), boundary pixels become BND.
-                for (uint32_t kk = t.pb + threadIdx.x; kk < t.pe; kk += kThreads) {
+                // With fewer pieces than threads, G = kThreads / pieces
+                // threads paint one piece's column range together (a cell's
+                // ~60 row pieces would otherwise leave 3/4 of the CTA idle
+                // at the barrier while 64-pixel CAS runs complete).
+                const uint32_t npc = t.pe - t.pb;
+                const uint32_t G = npc ? max(1u, (uint32_t)kThreads / npc) : 1u;
+                const uint32_t part = threadIdx.x % G;
+                for (uint32_t kk = t.pb + threadIdx.x / G; kk < t.pe; kk += kThreads / G) {
                     const uint2 pc = __ldg(&a.pieces[kk]);
                     uint32_t *row = lt + (pc.y & 255u) * t.stride;
-                    const uint32_t lo = (pc.y >> 8) & 255u, hi = pc.y >> 16;
+                    const uint32_t plo = (pc.y >> 8) & 255u, phi = pc.y >> 16;
+                    const uint32_t lo = plo + (phi - plo) * part / G, hi = plo + (phi - plo) * (part + 1) / G;
                     for (uint32_t x = lo; x < hi; ++x) {
                         uint32_t o = atomicCAS(&row[x], kNone, pc.x);
                         if (!ACC) {

@@ -27,19 +27,39 @@ from paper_journals_pvldb_zacharatoudasf17_b200 import dist as rjdist  # noqa: E
 from paper_journals_pvldb_zacharatoudasf17_b200 import rj  # noqa: E402
 
 
-def time_query(R, desc, stream, steps):
+def time_query(R, desc, stream, steps, graph_step=False):
+    """ms per step of the bench's step (query + finalise + D2H of the
+    results + stream sync); graph_step: the step captured once as one CUDA
+    graph (every kernel and copy still runs every step)."""
     n = R.n_poly
     d_cnt = torch.zeros(n, dtype=torch.int64, device="cuda")
     d_sum = torch.zeros(n, dtype=torch.float64, device="cuda")
     d_val = torch.zeros(n, dtype=torch.float64, device="cuda")
+    h_cnt = torch.zeros(n, dtype=torch.int64, pin_memory=True)
+    h_val = torch.zeros(n, dtype=torch.float64, pin_memory=True)
+
+    def body():
+        rj.rj_query_device(R.ctx, desc, d_cnt, d_sum)
+        rj.rj_finalize_device(R.ctx, desc.agg, d_cnt, d_sum, d_val)
+        h_cnt.copy_(d_cnt, non_blocking=True)
+        h_val.copy_(d_val, non_blocking=True)
 
     def step():
         with torch.cuda.stream(stream):
-            rj.rj_query_device(R.ctx, desc, d_cnt, d_sum)
-            rj.rj_finalize_device(R.ctx, desc.agg, d_cnt, d_sum, d_val)
+            body()
         stream.synchronize()
 
     for _ in range(3):
+        step()
+    if graph_step:
+        g = torch.cuda.CUDAGraph()
+        with torch.cuda.graph(g, stream=stream, capture_error_mode="relaxed"):
+            body()
+
+        def step():                                  # noqa: F811
+            with torch.cuda.stream(stream):          # replay on the timed stream
+                g.replay()
+            stream.synchronize()
         step()
     e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
     torch.cuda.synchronize()
@@ -49,7 +69,7 @@ def time_query(R, desc, stream, steps):
     e1.record(stream)
     torch.cuda.synchronize()
     st = R.stats()
-    return e0.elapsed_time(e1) / steps, d_cnt.cpu().numpy(), st
+    return e0.elapsed_time(e1) / steps, h_cnt.numpy().copy(), st
 
 
 def main():
@@ -61,6 +81,8 @@ def main():
     ap.add_argument("--only-rank", type=int, default=-1, help="profile: run only this rank's spatial shard")
     ap.add_argument("--poly-weight", type=float, default=0.0, help="strip cost weight of the domain width")
     ap.add_argument("--spatial-only", action="store_true")
+    ap.add_argument("--graph-step", action="store_true", help="capture each rank's whole step as one CUDA graph")
+    ap.add_argument("--skip-t1", action="store_true", help="profiling: skip the one-GPU query (T1 = NaN)")
     args = ap.parse_args()
     n = int(args.points)
     box, polys_name, recipe, q, desc_s = bench.workload(args.config)
@@ -72,7 +94,10 @@ def main():
     R.load_points(x, y, cols)
     desc = rj.make_desc(**q)
     W, H = rj.rj_resolve_canvas(R.ctx, desc)
-    t1, c1, st1 = time_query(R, desc, stream, args.steps)
+    if args.skip_t1:
+        t1, c1, st1 = float("nan"), np.zeros(R.n_poly, np.int64), {"ms_polygon": float("nan")}
+    else:
+        t1, c1, st1 = time_query(R, desc, stream, args.steps, args.graph_step)
     out = {"config": desc_s, "points": n, "canvas": [W, H], "t1_ms": t1,
            "t1_polygon_ms": st1["ms_polygon"], "ranks": {}}
     sample = torch.from_numpy(x[np.linspace(0, n - 1, 1 << 20).astype(np.int64)].astype(np.float64))
@@ -94,7 +119,7 @@ def main():
                     d = rj.make_desc(**q, view=rjdist.strip_window(box, sp, r, P, desc))
                 R.load_points(np.ascontiguousarray(x[sel]), np.ascontiguousarray(y[sel]),
                               [np.ascontiguousarray(c[sel]) for c in cols])
-                ms, cnt, st = time_query(R, d, stream, args.steps)
+                ms, cnt, st = time_query(R, d, stream, args.steps, args.graph_step)
                 tot += cnt
                 per.append({"ms": ms, "points": int(R.n_input), "polygon_ms": st["ms_polygon"],
                             "point_pass_ms": st["ms_point_pass"]})

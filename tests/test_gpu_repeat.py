@@ -137,3 +137,55 @@ def test_graph_replay_matches_eager():
             e = outs[(0,) + k[1:]]
             assert np.array_equal(v[0], e[0]) and np.allclose(v[1], e[1], rtol=1e-12, atol=0), k
     R.close()
+
+
+@pytest.mark.parametrize("agg", ["count", "sum"])
+def test_caller_graph_capture(agg):
+    """A caller may capture a whole query step (rj_query_device +
+    rj_finalize_device + the D2H copies) into its own CUDA graph on the
+    context's stream: the library then runs inside that capture (no
+    internal graph), and every replay recomputes the result -- checked by
+    poisoning the outputs before each replay."""
+    import torch
+    flat = PG.flatten(C.polygon_set("c1b"))
+    pts = C.c1_points(300_000)
+    fav = (np.arange(len(pts["x"])) % 9).astype(np.int32)
+    stream = torch.cuda.Stream()
+    R = rjmod.RasterJoin(C.C1_BOX, stream=stream.cuda_stream)
+    R.set_option(rjmod.OPT_TIMING, 1)
+    R.load_points(pts["x"], pts["y"], [fav])
+    R.load_polygons(flat)
+    P = oracle.Polys(flat, C.C1_BOX)
+    desc = rjmod.make_desc(agg=agg, agg_column=0 if agg == "sum" else -1, W=777, H=555, mode="accurate")
+    n = R.n_poly
+    d_cnt = torch.zeros(n, dtype=torch.int64, device="cuda")
+    d_sum = torch.zeros(n, dtype=torch.float64, device="cuda")
+    d_val = torch.zeros(n, dtype=torch.float64, device="cuda")
+    h_cnt = torch.zeros(n, dtype=torch.int64, pin_memory=True)
+
+    def body():
+        rjmod.rj_query_device(R.ctx, desc, d_cnt, d_sum)
+        rjmod.rj_finalize_device(R.ctx, desc.agg, d_cnt, d_sum, d_val)
+        h_cnt.copy_(d_cnt, non_blocking=True)
+
+    for _ in range(3):                                   # internal graph captured and replayed
+        with torch.cuda.stream(stream):
+            body()
+        stream.synchronize()
+    g = torch.cuda.CUDAGraph()
+    with torch.cuda.graph(g, stream=stream, capture_error_mode="relaxed"):
+        body()
+    ocnt, osum, _ = oracle.query(P, pts["x"], pts["y"], cols=[fav], agg_col=0, W=777, H=555, mode="accurate")
+    for _ in range(2):
+        h_cnt.fill_(-1)
+        d_cnt.fill_(-1)
+        d_val.fill_(-1.0)
+        torch.cuda.synchronize()
+        with torch.cuda.stream(stream):
+            g.replay()
+        stream.synchronize()
+        assert np.array_equal(h_cnt.numpy().astype(np.uint64), ocnt)
+        if agg == "sum":
+            assert np.array_equal(d_val.cpu().numpy(), osum)
+    assert R.stats()["ms_point_pass"] > 0
+    R.close()

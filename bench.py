@@ -411,7 +411,9 @@ def main():
     ap.add_argument("--tile", type=int, default=0, help="point-cell side in pixels (0 = library default)")
     ap.add_argument("--pass-variant", type=int, default=-1, help="SUM/AVG kernel: 0 label, 1 pixel tile")
     ap.add_argument("--stages", type=int, default=0, help="point-pass ring depth (0 = library default)")
+    ap.add_argument("--lane-runs", type=int, default=0, help="COUNT runs: 0 library default, 1 in-lane, 2 warp-merged")
     ap.add_argument("--mode", default="", help="override the config's mode: bounded|accurate|index|exact")
+    ap.add_argument("--canvas", type=int, default=0, help="override the config's canvas: W = H = CANVAS")
     ap.add_argument("--no-graphs", action="store_true", help="launch every query eagerly (no CUDA-graph replay)")
     ap.add_argument("--shard", default="spatial", choices=("spatial", "range"),
                     help="N > 1: x-strip shards via all_to_all + per-rank pixel windows, or plain index ranges")
@@ -441,6 +443,10 @@ def main():
     if args.mode:
         q = dict(q, mode=args.mode)
         desc += f" [mode={args.mode}]"
+    if args.canvas:
+        q = {k: v for k, v in q.items() if k != "epsilon"}
+        q.update(W=args.canvas, H=args.canvas)
+        desc += f" [canvas={args.canvas}^2]"
 
     if args.scaling == "weak":
         n_local, i0 = args.points, rank * args.points
@@ -488,6 +494,8 @@ def main():
         R.set_option(rj.OPT_STAGES, args.stages)
     if args.pass_variant >= 0:
         R.set_option(rj.OPT_PASS, args.pass_variant)
+    if args.lane_runs:
+        R.set_option(rj.OPT_LANE_RUNS, args.lane_runs)
     if args.no_graphs:
         R.set_option(rj.OPT_GRAPHS, 0)
     flat = C.array_polys(polys_name)

@@ -308,6 +308,7 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
         ++P.L;
     }
     a.n_stages = (uint32_t)point_pass_stages(f.n_slots);
+    a.lane_runs = c->lane_runs != 2;
     if ((s = items_for_level(c, P.L)) != RJ_OK) return s;
     c->launches = 0;
     // work counters / pass statistics (cleared per pass)
@@ -509,7 +510,7 @@ static void key_desc(std::vector<int64_t> &k, const rj_query_desc *q) {
 static std::vector<int64_t> query_key(Ctx *c, const rj_query_desc *q, int entry, const void *p0, const void *p1) {
     std::vector<int64_t> k = {entry, (int64_t)(uintptr_t)p0, (int64_t)(uintptr_t)p1, (int64_t)c->data_gen,
                               (int64_t)c->alloc_gen, c->timing, c->chunk, c->tile_side, c->force_stages,
-                              c->pass_variant, (int64_t)(uintptr_t)c->stream};
+                              c->pass_variant, c->lane_runs, (int64_t)(uintptr_t)c->stream};
     key_desc(k, q);
     return k;
 }
@@ -770,6 +771,11 @@ rj_status rj_set_option(rj_ctx *c, int32_t option, int64_t value) {
     if (option == RJ_OPT_KEEP_LOAD_SCRATCH) {
         c->keep_load_scratch = value ? 1 : 0;
         if (!value) free_load_scratch(c);
+        return RJ_OK;
+    }
+    if (option == RJ_OPT_LANE_RUNS) {
+        if (value < 0 || value > 2) return set_error(c, RJ_ERR_INVALID_ARGUMENT, "RJ_OPT_LANE_RUNS must be 0, 1 or 2");
+        c->lane_runs = (int)value;
         return RJ_OK;
     }
     if (option == RJ_OPT_CHUNK) {

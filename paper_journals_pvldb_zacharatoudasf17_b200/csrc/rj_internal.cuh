@@ -59,6 +59,7 @@ struct PassArgs {
     int32_t level;                // point-cell level L of this query (2^L x 2^L cells)
     const uint32_t *cell_off10;   // [kCells10 + 1] first point of every level-10 cell
     uint32_t tile_stride;         // row stride of a warp's tile (odd: conflict-free row prefix)
+    int32_t lane_runs;            // COUNT tile kernel: merge equal-pixel runs inside lanes only
     const uint32_t *piece_off;    // [4^L + 1]
     const uint2 *pieces;
     const uint32_t *mask;         // accurate: boundary bitmask (diagnostics; the kernels use bpieces)
@@ -172,6 +173,7 @@ struct Ctx {
     PassArgs last_bq{};                           // last accurate query with a global boundary queue (bq_cap > 0)
     int pass_variant = -1;                        // RJ_OPT_PASS: -1 auto, 0 label, 1 pixel tile
     int force_stages = 0;                         // RJ_OPT_STAGES: 0 = automatic, else 2..4
+    int lane_runs = 0;                            // RJ_OPT_LANE_RUNS: 0 auto (= 1), 1 in-lane runs, 2 warp-merged
     int tile_side = 64;                           // RJ_OPT_TILE_SIDE: target point-cell side in pixels
 
     // streamed query (label_canvas.cu, rj_query_stream)

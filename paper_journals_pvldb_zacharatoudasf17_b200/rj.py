@@ -34,6 +34,7 @@ OPS = {"<": 0, "<=": 1, ">": 2, ">=": 3, "==": 4}
 DT_I32, DT_F32, DT_F64 = 0, 1, 2
 OPT_TIMING, OPT_CHUNK, OPT_PASS, OPT_KEEP_LOAD_SCRATCH, OPT_TILE_SIDE, OPT_STAGES, OPT_STREAM_BATCH = 1, 2, 3, 4, 5, 6, 7
 OPT_GRAPHS = 8
+OPT_LANE_RUNS = 9
 MAX_PRED = 5
 
 

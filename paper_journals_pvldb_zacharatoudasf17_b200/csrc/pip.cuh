@@ -6,8 +6,8 @@
 // y-extent overlaps the cell's rows and that lies (partly) at or right of the
 // cell inside its polygon's MBR: exactly the edges that can toggle the
 // half-open PNPOLY ray of a point in the cell (reading Z4).  Entries are
-// sorted by edge id, so they group by polygon; each entry is inlined as
-// (xa, ya, xb, yb) + polygon id.
+// sorted by edge id, so they group by polygon; each entry is inlined as the
+// upward-oriented edge (xl, yl, dx = xu - xl, yu), yl < yu, + polygon id.
 #pragma once
 #include "rj_geom.cuh"
 
@@ -25,7 +25,7 @@ __device__ __forceinline__ uint32_t grid_pip(const uint32_t *__restrict__ grid_o
     const uint32_t cell = (py >> kGridShift) * kGrid + (px >> kGridShift);
     const uint32_t b = __ldg(&grid_off[cell]), e = __ldg(&grid_off[cell + 1]);
     uint32_t cur = kPipNone, par = 0, first = kPipNone;
-    const int64_t X = px, Y = py;
+    const int X = (int)px, Y = (int)py;                    // lattice coordinates < 2^30
     for (uint32_t k = b; k < e; ++k) {
         const uint32_t P = __ldg(&grid_poly[k]);
         const int4 E = __ldg(&grid_edge[k]);
@@ -37,11 +37,14 @@ __device__ __forceinline__ uint32_t grid_pip(const uint32_t *__restrict__ grid_o
             cur = P;
             par = 0;
         }
-        // PNPOLY toggle (half-open in y), exact in int64
-        if ((E.y > (int)py) != (E.w > (int)py)) {
-            const int64_t lhs = (X - E.x) * (int64_t)(E.w - E.y);
-            const int64_t rhs = (int64_t)(E.z - E.x) * (Y - E.y);
-            if (E.w > E.y ? lhs < rhs : lhs > rhs) par ^= 1u;
+        // PNPOLY toggle (O3, half-open in y) of the edge oriented upwards:
+        // yl <= py < yu and px < the crossing's x, i.e.
+        // (px - xl)(yu - yl) < (xu - xl)(py - yl); every factor fits 31 bits
+        // plus sign, so each product is one exact 32 x 32 -> 64-bit multiply
+        if (E.y <= Y && Y < E.w) {
+            const long long lhs = (long long)(X - E.x) * (E.w - E.y);
+            const long long rhs = (long long)E.z * (Y - E.y);
+            par ^= lhs < rhs ? 1u : 0u;
         }
     }
     if (par) {

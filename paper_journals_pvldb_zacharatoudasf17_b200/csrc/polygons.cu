@@ -104,16 +104,23 @@ __global__ void k_grid_edges(const int4 *__restrict__ edges, const uint32_t *__r
     }
 }
 
-// Entries inlined for the accurate-mode test: the edge's endpoints and its
-// polygon next to each other, so a boundary point reads one 16-B record and
-// one id per entry instead of chasing entry -> edge -> polygon.
+// Entries inlined for the accurate-mode test: the edge and its polygon next
+// to each other, so a boundary point reads one 16-B record and one id per
+// entry instead of chasing entry -> edge -> polygon.  The record is the edge
+// oriented upwards, (xl, yl, xu - xl, yu) with yl < yu (grid edges are never
+// horizontal): the half-open PNPOLY test is symmetric in the endpoints, and
+// the orientation leaves one comparison and two 32 x 32 -> 64-bit products
+// per entry (pip.cuh).
 __global__ void k_grid_inline(const uint32_t *__restrict__ ent, uint32_t n, const int4 *__restrict__ edges,
                               const uint32_t *__restrict__ edge_poly, int4 *__restrict__ gedge,
                               uint32_t *__restrict__ gpoly) {
     const uint32_t i = blockIdx.x * blockDim.x + threadIdx.x;
     if (i >= n) return;
     const uint32_t e = ent[i];
-    gedge[i] = edges[e];
+    const int4 E = edges[e];
+    const bool up = E.w > E.y;
+    const int xl = up ? E.x : E.z, yl = up ? E.y : E.w, xu = up ? E.z : E.x, yu = up ? E.w : E.y;
+    gedge[i] = make_int4(xl, yl, xu - xl, yu);
     gpoly[i] = edge_poly[e];
 }
 

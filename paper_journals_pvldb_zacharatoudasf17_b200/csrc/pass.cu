@@ -66,8 +66,8 @@ __device__ __forceinline__ void emit_pixel_run(const Tile &t, uint32_t key, uint
 // their points skip the tile and go to the warp queue.
 template <bool SUM, bool ACC, int NS, bool FP>
 __device__ __forceinline__ void process(const PassArgs &a, const Shared &sh, const Tile &t, const Consts<NS> &k,
-                                        const Win<NS> &w, uint32_t first, uint32_t count, BQ &bq,
-                                        uint32_t &n_pass, uint32_t &n_bnd) {
+                                        const Win<NS> &w, const uint32_t *sp, uint32_t first, uint32_t count,
+                                        BQ &bq, uint32_t &n_pass, uint32_t &n_bnd) {
     const int lane = threadIdx.x & 31;
     bool ok[kIPL];
     uint32_t key[kIPL];
@@ -83,7 +83,7 @@ __device__ __forceinline__ void process(const PassArgs &a, const Shared &sh, con
         for (int j = 0; j < kIPL; ++j)
             if (ok[j] && (lds(t.tbase + key[j] * 4u) & kFlag)) bm |= 1u << j;
         if (__any_sync(kFull, bm != 0u)) {
-            enqueue_window<SUM, NS>(a, sh, w, bm, bq, n_bnd);
+            enqueue_window<SUM>(a, sh, sp, kStagePts, bm, bq, n_bnd);
 #pragma unroll
             for (int j = 0; j < kIPL; ++j) ok[j] = ok[j] && !((bm >> j) & 1u);
         }
@@ -131,8 +131,9 @@ __device__ __forceinline__ void process(const PassArgs &a, const Shared &sh, con
 // the queue first, as in process().
 template <bool ACC, int NS, bool FP>
 __device__ __forceinline__ void process_lane_runs(const PassArgs &a, const Shared &sh, const Tile &t,
-                                                  const Consts<NS> &k, const Win<NS> &w, uint32_t first,
-                                                  uint32_t count, BQ &bq, uint32_t &n_pass, uint32_t &n_bnd) {
+                                                  const Consts<NS> &k, const Win<NS> &w, const uint32_t *sp,
+                                                  uint32_t first, uint32_t count, BQ &bq, uint32_t &n_pass,
+                                                  uint32_t &n_bnd) {
     const int lane = threadIdx.x & 31;
     bool ok[kIPL];
     uint32_t key[kIPL];
@@ -148,7 +149,7 @@ __device__ __forceinline__ void process_lane_runs(const PassArgs &a, const Share
         for (int j = 0; j < kIPL; ++j)
             if (ok[j] && (lds(t.tbase + key[j] * 4u) & kFlag)) bm |= 1u << j;
         if (__any_sync(kFull, bm != 0u)) {
-            enqueue_window<false, NS>(a, sh, w, bm, bq, n_bnd);
+            enqueue_window<false>(a, sh, sp, kStagePts, bm, bq, n_bnd);
 #pragma unroll
             for (int j = 0; j < kIPL; ++j) ok[j] = ok[j] && !((bm >> j) & 1u);
         }
@@ -277,12 +278,13 @@ __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a)
             const uint32_t ncopy = ((m.se + 3u) & ~3u) - m.cb;
             if (woff < ncopy && !never) {
                 Win<NS> w;
-                load_win_smem<NS>(w, ring + (size_t)st * ncol * kStagePts, woff + lane * kIPL);
+                const uint32_t *sp = ring + (size_t)st * ncol * kStagePts + woff + lane * kIPL;
+                load_win_smem<NS>(w, sp, 0);
                 const uint32_t first = (m.sb - m.cb) - woff;    // may wrap: unsigned range test
                 if (!SUM && a.lane_runs)
-                    process_lane_runs<ACC, NS, FP>(a, sh, t, k, w, first, m.se - m.sb, bq, n_pass, n_bnd);
+                    process_lane_runs<ACC, NS, FP>(a, sh, t, k, w, sp, first, m.se - m.sb, bq, n_pass, n_bnd);
                 else
-                    process<SUM, ACC, NS, FP>(a, sh, t, k, w, first, m.se - m.sb, bq, n_pass, n_bnd);
+                    process<SUM, ACC, NS, FP>(a, sh, t, k, w, sp, first, m.se - m.sb, bq, n_pass, n_bnd);
             }
             stage_release(smem_u32(&rg.empty[st]));
             if (m.flags & 2u) {

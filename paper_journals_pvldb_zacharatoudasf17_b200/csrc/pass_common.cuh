@@ -225,44 +225,19 @@ static __device__ __forceinline__ void bq_next_chunk(const PassArgs &a, BQ &q) {
     }
 }
 
-// append point j of the lanes with bnd set
-template <bool SUM, int NS>
-__device__ __forceinline__ void enqueue(const PassArgs &a, const Shared &sh, const Win<NS> &w, int j, bool bnd,
-                                        BQ &q, uint32_t &n_bnd) {
-    const unsigned bb = __ballot_sync(kFull, bnd);
-    if (!bb) return;
-    const int lane = threadIdx.x & 31;
-    const uint32_t n = __popc(bb), rank = __popc(bb & ((1u << lane) - 1u));
-    n_bnd += bnd ? 1u : 0u;
-    if (q.global && q.pos + n > q.end) bq_next_chunk(a, q);
-    if (q.pos + n <= q.end) {
-        if (bnd) {
-            a.bq_x[q.pos + rank] = w.x[j];
-            a.bq_y[q.pos + rank] = w.y[j];
-            if (SUM) a.bq_a[q.pos + rank] = agg_bits<NS>(a, w, j);
-        }
-        q.pos += n;
-        return;
-    }
-    if (bnd) {
-        const uint32_t pos = q.qn + rank;
-        sh.qx[pos] = w.x[j];
-        sh.qy[pos] = w.y[j];
-        sh.qa[pos] = SUM ? agg_bits<NS>(a, w, j) : 0u;
-    }
-    q.qn += n;
-    if (q.qn >= 32) drain_queue<SUM>(a, sh, q.qn, false);       // leaves < 32
-}
-
 // Append the boundary points of a whole 256-point window (bit j of bm: this
 // lane's point j is a boundary point) -- one warp scan of the per-lane
-// counts instead of a ballot per point slot.  Ranks follow (lane, j), the
-// order enqueue() would give; a window may fill the current chunk and
-// continue in the next one.  Without a global chunk the points go to the
-// warp's shared queue, tested 32 at a time.
-template <bool SUM, int NS>
-__device__ __forceinline__ void enqueue_window(const PassArgs &a, const Shared &sh, const Win<NS> &w, uint32_t bm,
-                                               BQ &q, uint32_t &n_bnd) {
+// counts instead of a ballot per point slot.  Ranks follow (lane, j); a
+// window may fill the current chunk and continue in the next one.  Without
+// a global chunk the points go to the warp's shared queue, tested 32 at a
+// time.  The points are re-read from the stage in shared memory (sp = this
+// lane's 8 points of the x column, cs = the stage's column stride; y and the
+// aggregated attribute follow at cs and 2 cs), so the window's registers
+// need not stay live through this rare path (r2: 108 B of spills in the
+// accurate label kernel otherwise).
+template <bool SUM>
+__device__ __forceinline__ void enqueue_window(const PassArgs &a, const Shared &sh, const uint32_t *sp, uint32_t cs,
+                                               uint32_t bm, BQ &q, uint32_t &n_bnd) {
     const int lane = threadIdx.x & 31;
     const uint32_t c = __popc(bm);
     uint32_t incl = c;
@@ -286,14 +261,15 @@ __device__ __forceinline__ void enqueue_window(const PassArgs &a, const Shared &
             const uint32_t r = excl + __popc(bm & ((1u << j) - 1u));   // rank of point j
             if (((bm >> j) & 1u) && r >= done && r < done + take) {
                 const uint32_t pos = at + (r - done);
+                const uint32_t x = sp[j], y = sp[cs + j], ab = SUM ? sp[2 * cs + j] : 0u;
                 if (glob) {
-                    a.bq_x[pos] = w.x[j];
-                    a.bq_y[pos] = w.y[j];
-                    if (SUM) a.bq_a[pos] = agg_bits<NS>(a, w, j);
+                    a.bq_x[pos] = x;
+                    a.bq_y[pos] = y;
+                    if (SUM) a.bq_a[pos] = ab;
                 } else {
-                    sh.qx[pos] = w.x[j];
-                    sh.qy[pos] = w.y[j];
-                    sh.qa[pos] = SUM ? agg_bits<NS>(a, w, j) : 0u;
+                    sh.qx[pos] = x;
+                    sh.qy[pos] = y;
+                    sh.qa[pos] = ab;
                 }
             }
         }

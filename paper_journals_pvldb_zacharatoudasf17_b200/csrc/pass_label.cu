@@ -100,9 +100,9 @@ __device__ __forceinline__ void fold(LaneAcc &acc, Carry &cy) {
 
 template <bool ACC, int NS, bool FP, bool AF>
 __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh, const LabTile &t,
-                                            const Consts<NS> &k, const Win<NS> &w, uint32_t first, uint32_t count,
-                                            Carry &cy, LaneAcc &acc, BQ &bq, uint32_t &n_pass,
-                                            uint32_t &n_bnd) {
+                                            const Consts<NS> &k, const Win<NS> &w, const uint32_t *sp,
+                                            uint32_t first, uint32_t count, Carry &cy, LaneAcc &acc, BQ &bq,
+                                            uint32_t &n_pass, uint32_t &n_bnd) {
     const int lane = threadIdx.x & 31;
     uint32_t lab[kIPL];
     bool spec = false, uni = true;
@@ -120,12 +120,13 @@ __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh,
     // fast path: every point of the window carries the carry's label (never
     // MULTI / BND: the carry's label is a polygon or NONE)
     if (__all_sync(kFull, uni)) {
+        // pairwise: three dependent binary64 adds per window instead of eight
+        // (any order is within the 1e-9 bound; integer sums stay exact)
+        double v[kIPL];
 #pragma unroll
-        for (int j = 0; j < kIPL; ++j)
-            if ((okm >> j) & 1u) {
-                acc.cnt += 1u;
-                acc.sum += attr_d<AF>(agg_bits<NS>(a, w, j));
-            }
+        for (int j = 0; j < kIPL; ++j) v[j] = ((okm >> j) & 1u) ? attr_d<AF>(agg_bits<NS>(a, w, j)) : 0.0;
+        acc.cnt += __popc(okm);
+        acc.sum += ((v[0] + v[1]) + (v[2] + v[3])) + ((v[4] + v[5]) + (v[6] + v[7]));
         return;
     }
     fold(acc, cy);
@@ -139,7 +140,7 @@ __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh,
             if (ACC && lab[j] == kBnd) bm |= 1u << j;
             if (lab[j] >= kBnd) lab[j] = kNone;
         }
-        if (ACC) enqueue_window<true, NS>(a, sh, w, bm, bq, n_bnd);
+        if (ACC) enqueue_window<true>(a, sh, sp, kStagePts, bm, bq, n_bnd);
     }
     // Runs of equal labels: inside the lane in registers, across lanes by a
     // segmented scan, and across windows through the warp's carry (Morton
@@ -311,9 +312,10 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
             const uint32_t ncopy = ((m.se + 3u) & ~3u) - m.cb;
             if (woff < ncopy && !never) {
                 Win<NS> w;
-                load_win_smem<NS>(w, ring + (size_t)st * ncol * kStagePts, woff + lane * kIPL);
-                process_lab<ACC, NS, FP, AF>(a, sh, t, k, w, (m.sb - m.cb) - woff, m.se - m.sb, cy, acc, bq, n_pass,
-                                             n_bnd);
+                const uint32_t *sp = ring + (size_t)st * ncol * kStagePts + woff + lane * kIPL;
+                load_win_smem<NS>(w, sp, 0);
+                process_lab<ACC, NS, FP, AF>(a, sh, t, k, w, sp, (m.sb - m.cb) - woff, m.se - m.sb, cy, acc, bq,
+                                             n_pass, n_bnd);
             }
             stage_release(smem_u32(&rg.empty[st]));
             if (++st == nstage) { st = 0; ph ^= 1u; }

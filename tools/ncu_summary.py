@@ -77,6 +77,10 @@ def summarize(rep):
 
 
 def launches(path, steps=0):
+    """Launch list of an ncu --metrics gpu__time_duration.sum capture.  The
+    per-step table covers the launches after the last load-time kernel (the
+    sort / quantise / cell-bounds / edge-grid kernels and torch fills) and
+    counts one query step per launch of the point-pass kernel."""
     rows = list(csv.reader(open(path)))
     hdr = None
     for i, r in enumerate(rows):
@@ -85,31 +89,38 @@ def launches(path, steps=0):
             break
     h = rows[hdr]
     k_i, v_i, u_i = h.index("Kernel Name"), h.index("Metric Value"), h.index("Metric Unit")
-    tot = collections.Counter()
-    cnt = collections.Counter()
+    seq = []
     for r in rows[hdr + 1:]:
         if len(r) <= v_i:
             continue
         v = float(r[v_i].replace(",", ""))
         scale = {"ns": 1e-6, "nsecond": 1e-6, "us": 1e-3, "usecond": 1e-3, "ms": 1.0, "msecond": 1.0}.get(r[u_i], 1.0)
-        name = r[k_i].split("(")[0]
-        tot[name] += v * scale
+        seq.append((r[k_i].split("(")[0], v * scale))
+    tot = collections.Counter()
+    cnt = collections.Counter()
+    for name, ms in seq:
+        tot[name] += ms
         cnt[name] += 1
     all_ms = sum(tot.values())
     lines = [f"# launch list: {path}", "", "| kernel | launches | total ms | share |", "|---|---|---|---|"]
     for k, v in tot.most_common():
         lines.append(f"| {k} | {cnt[k]} | {v:.3f} | {v / all_ms * 100:.1f} % |")
     if steps:
-        # kernels launched once (or a fixed number of times) per query step:
-        # launch count a multiple of the number of query steps in the capture
-        q = {k: v for k, v in tot.items() if cnt[k] % steps == 0 and not k.startswith("void at::")
-             and "radix" not in k and "quantize" not in k and "cell_bounds" not in k and "grid_" not in k}
-        q_ms = sum(q.values())
-        lines += ["", f"## per query step ({steps} steps in the capture; load-time kernels excluded)", "",
-                  "| kernel | launches/step | ms/step | share of the step |", "|---|---|---|---|"]
-        for k, v in sorted(q.items(), key=lambda kv: -kv[1]):
-            lines.append(f"| {k} | {cnt[k] // steps} | {v / steps:.4f} | {v / q_ms * 100:.1f} % |")
-        lines.append(f"| (all) | | {q_ms / steps:.4f} | 100 % |")
+        load = ("radix", "quantize", "cell_bounds", "grid_", "at::", "ring_sigma")
+        last = max([i for i, (n, _) in enumerate(seq) if any(t in n for t in load)], default=-1)
+        qs = seq[last + 1:]
+        n_steps = sum(1 for n, _ in qs if "k_point_pass" in n) or 1
+        qt = collections.Counter()
+        qc = collections.Counter()
+        for name, ms in qs:
+            qt[name] += ms
+            qc[name] += 1
+        q_ms = sum(qt.values())
+        lines += ["", f"## per query step ({n_steps} query steps after the load; serialised, cold: compare shares)",
+                  "", "| kernel | launches/step | ms/step | share of the step |", "|---|---|---|---|"]
+        for k, v in qt.most_common():
+            lines.append(f"| {k} | {qc[k] / n_steps:g} | {v / n_steps:.4f} | {v / q_ms * 100:.1f} % |")
+        lines.append(f"| (all) | | {q_ms / n_steps:.4f} | 100 % |")
     return "\n".join(lines)
 
 

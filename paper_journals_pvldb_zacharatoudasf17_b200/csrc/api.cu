@@ -213,7 +213,7 @@ static void tile_geometry(int W, int H, int L, uint32_t &stride, uint32_t &cap) 
         mh = std::max(mh, cell_pix_hi(k, H, L) - cell_pix_lo(k, H, L) + 1);
     }
     stride = (uint32_t)(mw | 1);
-    cap = (uint32_t)(mh * stride);
+    cap = (uint32_t)((mh * stride + 3) & ~3);    // whole 16-B words: tiles stay aligned, cleared with 16-B stores
 }
 
 // Exact-mode chooser (RJ_EXACT).  Both exact variants
@@ -251,6 +251,8 @@ static int choose_exact(const Ctx *c, int W, int H, float f, uint64_t n_points) 
 }
 
 struct Prepared {
+    bool init_done = false;        // k_pass_init already ran ahead of the polygon pass
+    uint32_t poly_launches = 0;    // kernels the polygon pass launched after it
     int W, H, L;
     View view;
     int mode;                      // executed rj_mode (RJ_EXACT resolved)
@@ -276,7 +278,8 @@ static cudaError_t record_ev(Ctx *c, int i) {
 
 // Everything up to (not including) the point-pass launch.
 static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_polygon_pass = true,
-                         bool bands = false, bool need_mask = false) {
+                         bool bands = false, bool need_mask = false, unsigned long long *d_cnt = nullptr,
+                         double *d_sum = nullptr) {
     rj_status s = check_ready(c, q);
     if (s != RJ_OK) return s;
     if ((s = resolve(c->x0, c->y0, c->x1, c->y1, q, &P.W, &P.H)) != RJ_OK)
@@ -317,9 +320,19 @@ static rj_status prepare(Ctx *c, const rj_query_desc *q, Prepared &P, bool need_
     if (c->timing) RJ_CUDA(c, record_ev(c, 0));
     // the index join needs neither spans nor the boundary mask
     P.pp = PolyPass{};
-    if (need_polygon_pass && !P.index &&
-        (s = polygon_pass(c, P.W, P.H, P.L, P.acc || bands, P.pp, P.view, need_mask && P.acc)) != RJ_OK)
+    const bool poly = need_polygon_pass && !P.index;
+    if (poly && d_cnt) {
+        // the per-query reset runs first, so the point pass's producer warp
+        // may start streaming while the polygon pass's last kernel still runs
+        // (it reads only the work counter and the static items; PDL: that
+        // kernel triggered its dependents after its own wait)
+        RJ_CUDA(c, launch_pass_init(c, wsbuf(c, kWsWork).as<uint32_t>(), d_cnt, P.sum ? d_sum : nullptr, c->n_poly));
+        P.init_done = true;
+    }
+    const uint32_t l0 = c->launches;
+    if (poly && (s = polygon_pass(c, P.W, P.H, P.L, P.acc || bands, P.pp, P.view, need_mask && P.acc)) != RJ_OK)
         return s;
+    P.poly_launches = c->launches - l0;
     if (c->timing) RJ_CUDA(c, record_ev(c, 1));
     a.qx = c->qx.as<uint32_t>();
     a.qy = c->qy.as<uint32_t>();
@@ -389,7 +402,8 @@ static rj_status run_pass(Ctx *c, Prepared &P, unsigned long long *d_cnt, double
     a.A_sum = d_sum;
     rj_status s = setup_bqueue(c, P);
     if (s != RJ_OK) return s;
-    RJ_CUDA(c, launch_pass_init(c, a.work_counter, d_cnt, P.sum ? d_sum : nullptr, c->n_poly));
+    a.early_stream = P.init_done && P.poly_launches > 0;
+    if (!P.init_done) RJ_CUDA(c, launch_pass_init(c, a.work_counter, d_cnt, P.sum ? d_sum : nullptr, c->n_poly));
     s = point_pass(c, a, P.sum, P.acc);
     if (s != RJ_OK) return s;
     if (a.bq_cap && (s = pip_queue_pass(c, a, P.sum)) != RJ_OK) return s;
@@ -827,7 +841,7 @@ rj_status rj_query_device(rj_ctx *c, const rj_query_desc *q, uint64_t *d_count, 
     if (s != RJ_OK) return s;
     return run_graphed(c, query_key(c, q, 1, d_count, d_sum), [&]() -> rj_status {
         Prepared P;
-        rj_status s2 = prepare(c, q, P);
+        rj_status s2 = prepare(c, q, P, true, false, false, reinterpret_cast<unsigned long long *>(d_count), d_sum);
         if (s2 != RJ_OK) return s2;
         if ((s2 = run_pass(c, P, reinterpret_cast<unsigned long long *>(d_count), d_sum)) != RJ_OK) return s2;
         if (c->timing) RJ_CUDA(c, record_ev(c, 3));      // ms_total of this query (rj_get_stats)
@@ -875,7 +889,7 @@ rj_status rj_query(rj_ctx *c, const rj_query_desc *q, uint64_t *count, double *v
         return set_error(c, RJ_ERR_OOM, "result allocation failed");
     s = run_graphed(c, query_key(c, q, 2, nullptr, value ? c->res_val.p : nullptr), [&]() -> rj_status {
         Prepared P;
-        rj_status s2 = prepare(c, q, P);
+        rj_status s2 = prepare(c, q, P, true, false, false, c->res_cnt.as<unsigned long long>(), c->res_sum.as<double>());
         if (s2 != RJ_OK) return s2;
         if ((s2 = run_pass(c, P, c->res_cnt.as<unsigned long long>(), c->res_sum.as<double>())) != RJ_OK) return s2;
         if (value) RJ_CUDA(c, launch_finalize(c, q->agg, (uint32_t)n, c->res_cnt.as<unsigned long long>(),

@@ -54,6 +54,7 @@ struct Tile {
 
 template <bool SUM>
 __device__ __forceinline__ void emit_pixel_run(const Tile &t, uint32_t key, uint32_t cnt, double sum, bool when) {
+    RJ_DCHECK(!(when && cnt) || (key - t.base < t.th * t.stride && (key - t.base) % t.stride < t.tw));
     red_add_if(t.tbase + key * 4u, cnt, when ? 1u : 0u);
     if (SUM && when && cnt) atomicAdd(&t.sum[key - t.base], sum);
 }
@@ -80,8 +81,10 @@ __device__ __forceinline__ void process(const PassArgs &a, const Shared &sh, con
     if (ACC) {
         uint32_t bm = 0;
 #pragma unroll
-        for (int j = 0; j < kIPL; ++j)
+        for (int j = 0; j < kIPL; ++j) {
+            if (ok[j]) RJ_DCHECK(key[j] - t.base < t.th * t.stride && (key[j] - t.base) % t.stride < t.tw);
             if (ok[j] && (lds(t.tbase + key[j] * 4u) & kFlag)) bm |= 1u << j;
+        }
         if (__any_sync(kFull, bm != 0u)) {
             enqueue_window<SUM>(a, sh, sp, kStagePts, bm, bq, n_bnd);
 #pragma unroll
@@ -146,8 +149,10 @@ __device__ __forceinline__ void process_lane_runs(const PassArgs &a, const Share
     if (ACC) {
         uint32_t bm = 0;
 #pragma unroll
-        for (int j = 0; j < kIPL; ++j)
+        for (int j = 0; j < kIPL; ++j) {
+            if (ok[j]) RJ_DCHECK(key[j] - t.base < t.th * t.stride && (key[j] - t.base) % t.stride < t.tw);
             if (ok[j] && (lds(t.tbase + key[j] * 4u) & kFlag)) bm |= 1u << j;
+        }
         if (__any_sync(kFull, bm != 0u)) {
             enqueue_window<false>(a, sh, sp, kStagePts, bm, bq, n_bnd);
 #pragma unroll
@@ -213,8 +218,11 @@ __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a)
             sh.pcnt[kk] = 0;
         }
     // everything above is CTA-local setup; the work counter, the polygon
-    // pass's pieces and the partial vectors are the predecessors' output
-    pdl_wait();
+    // pass's pieces and the partial vectors are the predecessors' output.
+    // early_stream: the work counter was zeroed before the polygon pass, so
+    // the producer streams at once while the last polygon kernel finishes;
+    // only the consumers wait for the pieces
+    if (!a.early_stream) pdl_wait();
     pdl_trigger();
     __syncthreads();
 
@@ -222,6 +230,7 @@ __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a)
         if (lane == 0) produce(a, rg, ring, nstage, ncol);
         __syncwarp();                                      // reconverge before the CTA barrier
     } else {
+        if (a.early_stream) pdl_wait();
         const Consts<NS> k = make_consts<NS>(a);
         const int s_lat = kLatticeBits - a.level;
         const bool never = a.f.never != 0;
@@ -257,7 +266,7 @@ __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a)
                 if (ACC) {
                     clear_tile_acc(t.cnt, t.stride, t.th, t.tw, r0, c0, a.index_join, kFlag, 0u, a.view);
                 } else {
-                    for (uint32_t i = threadIdx.x; i < words; i += kThreads) t.cnt[i] = 0u;
+                    fill_tile(t.cnt, words, 0u);
                 }
                 if (SUM)
                     for (uint32_t i = threadIdx.x; i < words; i += kThreads) t.sum[i] = 0.0;
@@ -297,6 +306,7 @@ __global__ void __maxnreg__(96) k_point_pass(const __grid_constant__ PassArgs a)
                 for (uint32_t kk = pb + threadIdx.x; kk < pe; kk += kThreads) {
                     const uint2 pc = (kk == pb + threadIdx.x) ? pc0 : __ldg(&a.pieces[kk]);
                     const uint32_t lr = pc.y & 255u, lo = (pc.y >> 8) & 255u, hi = pc.y >> 16;
+                    RJ_DCHECK(lr < t.th && lo < hi && hi <= t.tw);
                     const uint32_t *rc = t.cnt + lr * t.stride;
                     uint32_t cnt = 0;
                     for (uint32_t i = lo; i < hi; ++i) cnt += rc[i];

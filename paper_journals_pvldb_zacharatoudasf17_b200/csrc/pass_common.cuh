@@ -261,6 +261,7 @@ __device__ __forceinline__ void enqueue_window(const PassArgs &a, const Shared &
             const uint32_t r = excl + __popc(bm & ((1u << j) - 1u));   // rank of point j
             if (((bm >> j) & 1u) && r >= done && r < done + take) {
                 const uint32_t pos = at + (r - done);
+                RJ_DCHECK(glob ? pos < a.bq_cap : pos < (uint32_t)kQ);
                 const uint32_t x = sp[j], y = sp[cs + j], ab = SUM ? sp[2 * cs + j] : 0u;
                 if (glob) {
                     a.bq_x[pos] = x;
@@ -290,6 +291,13 @@ __device__ __forceinline__ void bq_finish(const PassArgs &a, const Shared &sh, B
     if (q.qn) drain_queue<SUM>(a, sh, q.qn, true);
 }
 
+// words [0, n) of a tile (16-B aligned, capacity a multiple of 4 words) = v,
+// with 16-B stores
+__device__ __forceinline__ void fill_tile(uint32_t *tile, uint32_t n, uint32_t v) {
+    uint4 *t4 = reinterpret_cast<uint4 *>(tile);
+    for (uint32_t i = threadIdx.x; i < (n + 3u) / 4u; i += kThreads) t4[i] = make_uint4(v, v, v, v);
+}
+
 // Accurate-mode tile setup, phase 1: word (r, x) of a th x stride tile
 // becomes `flag` for the pixels (c0 + x, r0 + r), x < tw, inside the viewport
 // window view = (c0, r0, c1, r1) when `all` (the index join: every pixel is a
@@ -299,7 +307,7 @@ __device__ __forceinline__ void clear_tile_acc(uint32_t *tile, uint32_t stride, 
                                                uint32_t r0, uint32_t c0, bool all, uint32_t flag, uint32_t zero,
                                                const int32_t *view) {
     if (!all) {
-        for (uint32_t i = threadIdx.x; i < th * stride; i += kThreads) tile[i] = zero;
+        fill_tile(tile, th * stride, zero);
         return;
     }
     const uint32_t vc0 = (uint32_t)view[0], vr0 = (uint32_t)view[1], vc1 = (uint32_t)view[2], vr1 = (uint32_t)view[3];

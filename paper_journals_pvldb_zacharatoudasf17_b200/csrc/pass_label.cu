@@ -31,6 +31,7 @@ struct LabTile {
     uint32_t lab_base;       // shared byte address of label word 0 minus 4 * (r0 * stride + c0)
     uint32_t stride, c0, r0;
     uint32_t pb, pe;         // the cell's span pieces
+    uint32_t th, tw;         // the cell's pixel rows and columns
 };
 
 // Emit a label run (skipped when !when, cnt == 0 or the label is not a polygon).
@@ -113,6 +114,7 @@ __device__ __forceinline__ void process_lab(const PassArgs &a, const Shared &sh,
         n_pass += ok ? 1u : 0u;
         okm |= ok ? 1u << j : 0u;
         const uint32_t px = mulhi(w.x[j], k.W4), py = mulhi(w.y[j], k.H4);
+        if (ok) RJ_DCHECK(py - t.r0 < t.th && px - t.c0 < t.tw);
         lab[j] = ok ? lds(t.lab_base + (py * t.stride + px) * 4u) : kNone;
         spec |= lab[j] == kMulti || lab[j] == kBnd;
         uni &= !ok || lab[j] == cy.lab;
@@ -223,7 +225,9 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
         for (uint32_t kk = threadIdx.x; kk < a.n_poly; kk += blockDim.x) {
             sh.pcnt[kk] = 0;
         }
-    pdl_wait();                                             // predecessors' output from here on
+    // predecessors' output from here on (early_stream: the producer streams
+    // at once, see pass.cu)
+    if (!a.early_stream) pdl_wait();
     pdl_trigger();
     __syncthreads();
 
@@ -231,6 +235,7 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
         if (lane == 0) produce(a, rg, ring, nstage, ncol);
         __syncwarp();                                      // reconverge before the CTA barrier
     } else {
+        if (a.early_stream) pdl_wait();
         const Consts<NS> k = make_consts<NS>(a);
         const int s_lat = kLatticeBits - a.level;
         const bool never = a.f.never != 0;
@@ -256,6 +261,8 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
                 const uint32_t th = (uint32_t)pix(((cy + 1) << s_lat) - 1, a.H) - t.r0 + 1;
                 const uint32_t tw = (uint32_t)pix(((cx + 1) << s_lat) - 1, a.W) - t.c0 + 1;
                 t.lab_base = smem_u32(lt) - 4u * (t.r0 * t.stride + t.c0);
+                t.th = th;
+                t.tw = tw;
                 t.pb = t.pe = 0u;
                 if (!ACC || !a.index_join) {
                     t.pb = __ldg(&a.piece_off[m.cell]);
@@ -264,7 +271,7 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
                 if (ACC) {
                     clear_tile_acc(lt, t.stride, th, tw, t.r0, t.c0, a.index_join, kBnd, kNone, a.view);
                 } else {
-                    for (uint32_t i = threadIdx.x; i < th * t.stride; i += kThreads) lt[i] = kNone;
+                    fill_tile(lt, th * t.stride, kNone);
                 }
                 consumers_sync();
                 // one thread per piece.  Labels only move up the order
@@ -282,6 +289,7 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
                     const uint2 pc = __ldg(&a.pieces[kk]);
                     uint32_t *row = lt + (pc.y & 255u) * t.stride;
                     const uint32_t plo = (pc.y >> 8) & 255u, phi = pc.y >> 16;
+                    RJ_DCHECK((pc.y & 255u) < th && plo < phi && phi <= tw);
                     const uint32_t lo = plo + (phi - plo) * part / G, hi = plo + (phi - plo) * (part + 1) / G;
                     for (uint32_t x = lo; x < hi; ++x) {
                         uint32_t o = atomicCAS(&row[x], kNone, pc.x);
@@ -299,6 +307,7 @@ __global__ void __maxnreg__(96) k_point_pass_label(const __grid_constant__ PassA
                     const uint32_t bb = __ldg(&a.bpiece_off[m.cell]), be = __ldg(&a.bpiece_off[m.cell + 1]);
                     for (uint32_t kk = bb + threadIdx.x; kk < be; kk += kThreads) {
                         const uint32_t v = __ldg(&a.bpieces[kk]);
+                        RJ_DCHECK((v & 255u) < th && (v >> 16) <= tw);
                         uint32_t *row = lt + (v & 255u) * t.stride;
                         // plain stores: a polygon's CAS never overwrites BND, and BND
                         // landing after a CAS wins either way

@@ -369,7 +369,10 @@ __device__ __forceinline__ void prow_emit_body(uint32_t t0, uint32_t ts, SpanGeo
                     if (q < nb) slot[q] = atomicAdd(&piece_cur[bc[q]], 1u);
 #pragma unroll
                 for (int q = 0; q < kB; ++q)
-                    if (q < nb) pieces[piece_off[bc[q]] + slot[q]] = make_uint2(P, bv[q]);
+                    if (q < nb) {
+                        RJ_DCHECK(piece_off[bc[q]] + slot[q] < piece_off[bc[q] + 1]);
+                        pieces[piece_off[bc[q]] + slot[q]] = make_uint2(P, bv[q]);
+                    }
                 nb = 0;
             };
             for_each_piece(g, r, lo, hi, [&](uint32_t cell, uint32_t lr, uint32_t a, uint32_t bb) {

@@ -60,6 +60,8 @@ struct PassArgs {
     const uint32_t *cell_off10;   // [kCells10 + 1] first point of every level-10 cell
     uint32_t tile_stride;         // row stride of a warp's tile (odd: conflict-free row prefix)
     int32_t lane_runs;            // COUNT tile kernel: merge equal-pixel runs inside lanes only
+    int32_t early_stream;         // the producer may stream before the predecessor grid completes
+                                  // (k_pass_init ran before the polygon pass's PDL kernels)
     const uint32_t *piece_off;    // [4^L + 1]
     const uint2 *pieces;
     const uint32_t *mask;         // accurate: boundary bitmask (diagnostics; the kernels use bpieces)
@@ -317,6 +319,22 @@ rj_status cuda_error(Ctx *c, cudaError_t e, const char *where);
     } while (0)
 
 #define RJ_LAUNCHED(c) do { (c)->launches++; } while (0)
+
+// Device bounds checks (build with RJ_NVCC_EXTRA=-DRJ_CHECKS; off in the
+// product build): shared-tile indices, span-piece rows/columns, queue and
+// piece slots.  A failed check prints its condition and traps, so the query
+// returns RJ_ERR_CUDA.  (compute-sanitizer is closed on this GPU pool.)
+#ifdef RJ_CHECKS
+#define RJ_DCHECK(c)                                                                              \
+    do {                                                                                         \
+        if (!(c)) {                                                                              \
+            printf("RJ_DCHECK failed %s:%d: %s\n", __FILE__, __LINE__, #c);                      \
+            __trap();                                                                            \
+        }                                                                                        \
+    } while (0)
+#else
+#define RJ_DCHECK(c) do { } while (0)
+#endif
 
 // Programmatic dependent launch: the per-query kernel chain (polygon pass ->
 // point pass -> finalisation) is launched with the PDL attribute, so a

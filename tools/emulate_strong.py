@@ -3,8 +3,9 @@ share of a P-way sharded query one after the other on cuda:0 and take the
 slowest rank, for index-range shards (spatially random points, whole-canvas
 polygon pass per rank) and for x-strip shards (dist.strip_splitters'
 quantile rule + per-rank pixel window).  projected efficiency =
-T(1 GPU) / (P x max_r T_r), before the one all-reduce of <= 48 KB of
-partials (not measurable on one GPU).  Not a bench line: evidence for the
+T(1 GPU) / (P x max_r T_r); a second figure adds the one all-reduce of the
+packed partials as measured on one GPU (world size 1, a lower bound of the
+NVSwitch latency; allreduce_standin_ms).  Not a bench line: evidence for the
 shard design until a multi-GPU box is available.
 
     python tools/emulate_strong.py [--config C3] [--points 1e9] [--ranks 2,4,8]
@@ -72,6 +73,31 @@ def time_query(R, desc, stream, steps, graph_step=False):
     return e0.elapsed_time(e1) / steps, h_cnt.numpy().copy(), st
 
 
+def allreduce_standin_ms(n_poly, stream, iters=200):
+    """The one collective of a sharded query, measured the only way one GPU
+    allows: a world-size-1 NCCL all-reduce of the packed partials (2 n_poly
+    binary64, rj_pack_partials' layout) on the query stream.  A lower bound
+    of the 8-rank latency over NVSwitch (NCCL still launches its kernel)."""
+    import torch.distributed as dist
+    os.environ.setdefault("MASTER_ADDR", "127.0.0.1")
+    os.environ.setdefault("MASTER_PORT", str(29500 + os.getpid() % 1000))
+    if not dist.is_initialized():
+        dist.init_process_group("nccl", rank=0, world_size=1, device_id=torch.device("cuda", 0))
+    buf = torch.zeros(2 * n_poly, dtype=torch.float64, device="cuda")
+    with torch.cuda.stream(stream):
+        for _ in range(10):
+            dist.all_reduce(buf)
+    stream.synchronize()
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    with torch.cuda.stream(stream):
+        e0.record(stream)
+        for _ in range(iters):
+            dist.all_reduce(buf)
+        e1.record(stream)
+    stream.synchronize()
+    return e0.elapsed_time(e1) / iters
+
+
 def main():
     ap = argparse.ArgumentParser()
     ap.add_argument("--config", default="C3")
@@ -98,8 +124,9 @@ def main():
         t1, c1, st1 = float("nan"), np.zeros(R.n_poly, np.int64), {"ms_polygon": float("nan")}
     else:
         t1, c1, st1 = time_query(R, desc, stream, args.steps, args.graph_step)
+    ar_ms = allreduce_standin_ms(R.n_poly, stream)
     out = {"config": desc_s, "points": n, "canvas": [W, H], "t1_ms": t1,
-           "t1_polygon_ms": st1["ms_polygon"], "ranks": {}}
+           "t1_polygon_ms": st1["ms_polygon"], "allreduce_1gpu_ms": ar_ms, "ranks": {}}
     sample = torch.from_numpy(x[np.linspace(0, n - 1, 1 << 20).astype(np.int64)].astype(np.float64))
     for P in [int(v) for v in args.ranks.split(",")]:
         sp = rjdist.splitters_from_sample(sample, P, box, args.poly_weight)
@@ -125,6 +152,7 @@ def main():
                             "point_pass_ms": st["ms_point_pass"]})
             worst = max(p["ms"] for p in per)
             res[kind] = {"max_rank_ms": worst, "projected_efficiency": t1 / (P * worst),
+                         "projected_efficiency_with_allreduce": t1 / (P * (worst + ar_ms)),
                          "sum_equals_1gpu": bool(np.array_equal(tot, c1)) if args.only_rank < 0 else None,
                          "per_rank": per}
         out["ranks"][P] = res

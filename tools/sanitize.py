@@ -5,7 +5,7 @@ run under a sanitizer proves the same launches are still correct.
 
     compute-sanitizer --tool racecheck python tools/sanitize.py [--quick]
 
-Variants: tile (COUNT) and label (SUM/AVG) point-pass kernels, bounded and
+Variants: tile (COUNT; in-lane and warp-merged runs) and label (SUM/AVG) point-pass kernels, bounded and
 accurate, index join, the exact chooser, windows, a fine canvas, streamed
 queries (host and device columns, ragged batches), worst-case and expected
 intervals, MIN/MAX and multi-aggregate, graph replay, the debug kernels and
@@ -77,12 +77,15 @@ def main():
             om = "bounded" if mode == "bounded" else "accurate"
             for variant in (-1, 0, 1):
                 R.set_option(rj.OPT_PASS, variant)
+                # COUNT: in-lane runs (default) and warp-merged runs (variant 1)
+                R.set_option(rj.OPT_LANE_RUNS, 2 if variant == 1 else 0)
                 for agg, col in (("count", -1), ("sum", 0), ("avg", 1)):
                     preds = [(0, ">=", -30)]
                     cnt, _ = R.query(W=W, H=W, mode=mode, agg=agg, agg_column=col, preds=preds)
                     ocnt, _, _ = oracle.query(P, x, y, cols=cols, preds=preds, W=W, H=W, mode=om)
                     chk(cnt, ocnt, (W, mode, variant, agg))
     R.set_option(rj.OPT_PASS, -1)
+    R.set_option(rj.OPT_LANE_RUNS, 0)
     for _ in range(3):                            # graph capture + replay
         cnt, _ = R.query(W=1024, H=1024, mode="accurate")
     chk(cnt, oracle.query(P, x, y, W=1024, H=1024, mode="accurate")[0], "graph")

@@ -95,7 +95,8 @@ __global__ void k_membership(const PassArgs a, uint64_t n, int accurate, const u
                 const uint32_t cell = (qy >> kGridShift) * kGrid + (qx >> kGridShift);
                 uint32_t cur = 0xFFFFFFFFu, par = 0;
                 for (uint32_t k = a.grid_off[cell]; k < a.grid_off[cell + 1]; ++k) {
-                    const uint32_t ed = a.grid_ent[k], P = a.edge_poly[ed];
+                    const uint32_t ed = a.grid_ent[k] & 0x7FFFFFFFu, P = a.edge_poly[ed];
+                    const uint32_t left = a.grid_ent[k] >> 31;   // leftward ray: complement test
                     if (P != cur) {
                         if (par && cur < 64) m |= 1ull << cur;
                         cur = P;
@@ -105,7 +106,8 @@ __global__ void k_membership(const PassArgs a, uint64_t n, int accurate, const u
                     if ((E.y > (int)qy) != (E.w > (int)qy)) {
                         const int64_t lhs = ((int64_t)qx - E.x) * (int64_t)(E.w - E.y);
                         const int64_t rhs = (int64_t)(E.z - E.x) * ((int64_t)qy - E.y);
-                        if (E.w > E.y ? lhs < rhs : lhs > rhs) par ^= 1u;
+                        if (E.w > E.y ? lhs < rhs : lhs > rhs) par ^= 1u ^ left;
+                        else par ^= left;
                     }
                 }
                 if (par && cur < 64) m |= 1ull << cur;

@@ -51,20 +51,36 @@ __device__ __forceinline__ uint32_t upper_bound_u32(const uint32_t *a, uint32_t 
 // spread over many threads instead of one thread walking rows x columns.
 constexpr int kGridChunk = 32;
 
+// An edge of polygon P is listed in grid rows [gr0, gr1] (its half-open
+// y-extent) and, per row, in two column runs (reading Z25): the cells of P's
+// MBR left of the MBR's middle column `split` test a LEFTWARD ray -- the
+// edges with min x <= the cell's last column can toggle it -- and the cells
+// from `split` on a RIGHTWARD ray -- the edges with max x > the cell's first
+// column.  Each cell thus walks only the edges between itself and the nearer
+// side of P's MBR.
 struct GridRun {
-    int gr0, gr1, gc0, gc1;   // rows [gr0, gr1], columns [gc0, gc1] (empty: gr1 < gr0)
+    int gr0, gr1;             // rows [gr0, gr1] (empty: gr1 < gr0)
+    int l0, l1, r0, r1;       // leftward-ray columns [l0, l1], rightward-ray columns [r0, r1]
 };
 
 __device__ __forceinline__ GridRun grid_run(const int4 E, const int4 M) {
-    GridRun g{0, -1, 0, -1};
+    GridRun g{0, -1, 0, -1, 0, -1};
     if (E.y == E.w || M.z - 1 < M.x) return g;           // horizontal: never toggles; empty MBR
     const int ymin = min(E.y, E.w), ymax = max(E.y, E.w);
     g.gr0 = ymin >> kGridShift;
     g.gr1 = (ymax - 1) >> kGridShift;
-    g.gc0 = M.x >> kGridShift;
-    g.gc1 = min(min((M.z - 1) >> kGridShift, (max(E.x, E.z) - 1) >> kGridShift), kGrid - 1);
-    if (g.gc1 < g.gc0) g.gr1 = g.gr0 - 1;
+    const int m0 = M.x >> kGridShift, m1 = min((M.z - 1) >> kGridShift, kGrid - 1);
+    const int split = (int)(((int64_t)M.x + M.z) >> 1) >> kGridShift;
+    g.l0 = max(m0, min(E.x, E.z) >> kGridShift);
+    g.l1 = min(m1, split - 1);
+    g.r0 = max(m0, split);
+    g.r1 = min(m1, (max(E.x, E.z) - 1) >> kGridShift);
+    if (g.l1 < g.l0 && g.r1 < g.r0) g.gr1 = g.gr0 - 1;
     return g;
+}
+
+__device__ __forceinline__ uint32_t grid_chunks(int c0, int c1) {
+    return c1 < c0 ? 0u : (uint32_t)(c1 - c0 + kGridChunk) / kGridChunk;
 }
 
 // items[e] = rows x chunks of edge e; *total += its entries (64-bit: the u32
@@ -76,8 +92,9 @@ __global__ void k_grid_items(const int4 *__restrict__ edges, const uint32_t *__r
     unsigned long long ent = 0;
     if (e < n_edges) {
         const GridRun g = grid_run(edges[e], mbr[edge_poly[e]]);
-        const uint32_t rows = (uint32_t)max(0, g.gr1 - g.gr0 + 1), cols = (uint32_t)max(0, g.gc1 - g.gc0 + 1);
-        items[e] = rows * ((cols + kGridChunk - 1) / kGridChunk);
+        const uint32_t rows = (uint32_t)max(0, g.gr1 - g.gr0 + 1);
+        const uint32_t cols = (uint32_t)max(0, g.l1 - g.l0 + 1) + (uint32_t)max(0, g.r1 - g.r0 + 1);
+        items[e] = rows * (grid_chunks(g.l0, g.l1) + grid_chunks(g.r0, g.r1));
         ent = (unsigned long long)rows * cols;
     }
     for (int o = 16; o; o >>= 1) ent += __shfl_xor_sync(0xFFFFFFFFu, ent, o);
@@ -93,12 +110,17 @@ __global__ void k_grid_edges(const int4 *__restrict__ edges, const uint32_t *__r
     for (uint32_t j = blockIdx.x * blockDim.x + threadIdx.x; j < n_items; j += gridDim.x * blockDim.x) {
         const uint32_t e = upper_bound_u32(item_off, n_edges + 1, j) - 1;
         const GridRun g = grid_run(edges[e], mbr[edge_poly[e]]);
-        const uint32_t nch = (uint32_t)(g.gc1 - g.gc0 + kGridChunk) / kGridChunk, k = j - item_off[e];
+        const uint32_t nl = grid_chunks(g.l0, g.l1), nch = nl + grid_chunks(g.r0, g.r1), k = j - item_off[e];
         const int gr = g.gr0 + (int)(k / nch);
-        const int c0 = g.gc0 + (int)(k % nch) * kGridChunk, c1 = min(g.gc1, c0 + kGridChunk - 1);
+        const uint32_t q = k % nch;
+        const bool left = q < nl;                          // leftward-ray run
+        const int c0 = left ? g.l0 + (int)q * kGridChunk : g.r0 + (int)(q - nl) * kGridChunk;
+        const int c1 = min(left ? g.l1 : g.r1, c0 + kGridChunk - 1);
         for (int gc = c0; gc <= c1; ++gc) {
             const uint32_t cell = (uint32_t)gr * kGrid + gc;
-            if (FILL) ent[off[cell] + atomicAdd(&cursor[cell], 1u)] = e;
+            // entry = edge id, bit 31 = leftward ray (a cell's entries of one
+            // polygon share it, so sorting keeps each polygon contiguous)
+            if (FILL) ent[off[cell] + atomicAdd(&cursor[cell], 1u)] = e | (left ? 0x80000000u : 0u);
             else atomicAdd(&cnt[cell], 1u);
         }
     }
@@ -116,12 +138,12 @@ __global__ void k_grid_inline(const uint32_t *__restrict__ ent, uint32_t n, cons
                               uint32_t *__restrict__ gpoly) {
     const uint32_t i = blockIdx.x * blockDim.x + threadIdx.x;
     if (i >= n) return;
-    const uint32_t e = ent[i];
+    const uint32_t e = ent[i] & 0x7FFFFFFFu;
     const int4 E = edges[e];
     const bool up = E.w > E.y;
     const int xl = up ? E.x : E.z, yl = up ? E.y : E.w, xu = up ? E.z : E.x, yu = up ? E.w : E.y;
     gedge[i] = make_int4(xl, yl, xu - xl, yu);
-    gpoly[i] = edge_poly[e];
+    gpoly[i] = edge_poly[e] | (ent[i] & 0x80000000u);   // bit 31: leftward ray
 }
 
 // Sort each cell's entries by edge id (so they group by polygon, which the

@@ -357,7 +357,11 @@ __device__ __forceinline__ void prow_count_body(uint32_t t0, uint32_t ts, SpanGe
             if (!clip_span(g, r, lo, hi)) continue;
             ++ns;
             for_each_piece(g, r, lo, hi, [&](uint32_t cell, uint32_t, uint32_t, uint32_t) {
-                atomicAdd(&piece_cnt[cell], 1u);
+                // consecutive threads are consecutive rows of one polygon and
+                // mostly walk the same cells: the converged lanes of a cell add
+                // their pieces with one atomic
+                const unsigned peers = __match_any_sync(__activemask(), cell);
+                if ((threadIdx.x & 31) == __ffs(peers) - 1) atomicAdd(&piece_cnt[cell], (uint32_t)__popc(peers));
             });
         }
         span_cnt[pr] = ns;
@@ -379,31 +383,19 @@ __device__ __forceinline__ void prow_emit_body(uint32_t t0, uint32_t ts, SpanGeo
             if (!clip_span(g, r, lo, hi)) continue;
             uint32_t *s = spans + 4 * (uint64_t)k++;
             s[0] = P; s[1] = (uint32_t)r; s[2] = (uint32_t)lo; s[3] = (uint32_t)hi;
-            // batches of 8 pieces: the slot atomics of a batch are all in
-            // flight together instead of one L2 round trip per piece
-            constexpr int kB = 8;
-            uint32_t bc[kB], bv[kB];
-            int nb = 0;
-            auto flush = [&]() {
-                uint32_t slot[kB];
-#pragma unroll
-                for (int q = 0; q < kB; ++q)
-                    if (q < nb) slot[q] = atomicAdd(&piece_cur[bc[q]], 1u);
-#pragma unroll
-                for (int q = 0; q < kB; ++q)
-                    if (q < nb) {
-                        RJ_DCHECK(piece_off[bc[q]] + slot[q] < piece_off[bc[q] + 1]);
-                        pieces[piece_off[bc[q]] + slot[q]] = make_uint2(P, bv[q]);
-                    }
-                nb = 0;
-            };
+            // the converged lanes of a cell reserve their slots with one atomic
+            // (consecutive rows of one polygon mostly walk the same cells)
+            const uint32_t pv = P;
             for_each_piece(g, r, lo, hi, [&](uint32_t cell, uint32_t lr, uint32_t a, uint32_t bb) {
-#pragma unroll
-                for (int q = 0; q < kB; ++q)
-                    if (q == nb) { bc[q] = cell; bv[q] = lr | (a << 8) | (bb << 16); }
-                if (++nb == kB) flush();
+                const unsigned peers = __match_any_sync(__activemask(), cell);
+                const int lane = threadIdx.x & 31, leader = __ffs(peers) - 1;
+                uint32_t base = 0;
+                if (lane == leader) base = atomicAdd(&piece_cur[cell], (uint32_t)__popc(peers));
+                base = __shfl_sync(peers, base, leader);
+                const uint32_t slot = base + __popc(peers & ((1u << lane) - 1u));
+                RJ_DCHECK(piece_off[cell] + slot < piece_off[cell + 1]);
+                pieces[piece_off[cell] + slot] = make_uint2(pv, lr | (a << 8) | (bb << 16));
             });
-            if (nb) flush();
         }
     }
 }

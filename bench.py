@@ -213,7 +213,12 @@ def launch_ranks(args):
     s.close()
     cmd = [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", f"--nproc-per-node={args.gpus}",
            "--master-addr", "127.0.0.1", "--master-port", str(port), os.path.abspath(__file__), *sys.argv[1:]]
-    raise SystemExit(subprocess.call(cmd))
+    # NCCL's communicator-init lines (rank / nranks / transport) stay visible,
+    # so a run's rank count can be checked; the JSON line is still printed last
+    env = dict(os.environ)
+    env.setdefault("NCCL_DEBUG", "INFO")
+    env.setdefault("NCCL_DEBUG_SUBSYS", "INIT")
+    raise SystemExit(subprocess.call(cmd, env=env))
 
 
 def run_dry(args):
@@ -438,6 +443,8 @@ def main():
     local = int(os.environ.get("LOCAL_RANK", "0"))
     torch.cuda.set_device(local)
     if world > 1:
+        os.environ.setdefault("NCCL_DEBUG", "INFO")          # communicator-init lines: rank / nranks
+        os.environ.setdefault("NCCL_DEBUG_SUBSYS", "INIT")
         dist.init_process_group("nccl", device_id=torch.device("cuda", local))
     box, polys_name, recipe, q, desc = workload(args.config)
     if args.mode:

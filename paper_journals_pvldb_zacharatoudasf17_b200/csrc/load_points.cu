@@ -5,10 +5,12 @@
 //  1. k_quantize: Q(x) = floor(((x - x0) / (x1 - x0)) * 2^30) in binary64 with
 //     explicitly rounded ops (__dsub_rn, __ddiv_rn, exact *2^30), points with
 //     Q outside [0, 2^30) or NaN marked out-of-domain (reading Z11).
-//  2. Stable LSD radix sort (4 passes x 8 bits) on the 32-bit Morton key of
-//     (Qx >> 14, Qy >> 14); out-of-domain points form a 257th digit and sink
-//     to the end.  Payload columns (Qx, Qy, original index, attributes) move
-//     with the keys, so the point pass later streams contiguous columns.
+//  2. Stable LSD radix sort (4 passes x 8 bits) of (key, original index)
+//     pairs, key = the 32-bit Morton key of (Qx >> 14, Qy >> 14) capped at
+//     0xFFFFFFFE, or 0xFFFFFFFF for an out-of-domain point (it sinks to the
+//     end); then one
+//     gather puts Qx, Qy and the attribute columns in sorted order, so the
+//     point pass streams contiguous columns.
 //  3. cell_off: start of every level-10 (1024x1024) Morton cell; a cell of
 //     any coarser level L is the union of 4^(10-L) consecutive level-10
 //     cells, so the point tiles of every query resolution are contiguous
@@ -41,8 +43,32 @@ __global__ void k_quantize(const T *__restrict__ x, const T *__restrict__ y, uin
     }
 }
 
-__device__ __forceinline__ uint32_t sort_digit(uint32_t qx, uint32_t qy, int shift) {
-    return qx == kInvalid ? 256u : ((morton_key(qx, qy) >> shift) & 255u);
+// Sort key: the 32-bit Morton key of (Qx >> 14, Qy >> 14) (level-16 order),
+// capped at 0xFFFFFFFE; out-of-domain points get 0xFFFFFFFF, so they sort
+// last by the key alone (the cap only merges two level-16 cells inside the
+// last level-10 cell, whose order within a cell is free).
+__global__ void k_keys(const uint32_t *__restrict__ qx, const uint32_t *__restrict__ qy, uint64_t n,
+                       uint32_t *__restrict__ key) {
+    for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n; i += (uint64_t)gridDim.x * blockDim.x) {
+        const uint32_t x = qx[i], y = qy[i];
+        key[i] = x == kInvalid ? 0xFFFFFFFFu : min(morton_key(x, y), 0xFFFFFFFEu);
+    }
+}
+
+__device__ __forceinline__ uint32_t sort_digit(uint32_t key, int shift) { return (key >> shift) & 255u; }
+
+// After the (key, index) sort: every column in sorted order, gathered once
+// (qx, qy and the attribute columns of point idx[i] go to position i).
+struct Gather {
+    const uint32_t *src[2 + RJ_MAX_COLS];
+    uint32_t *dst[2 + RJ_MAX_COLS];
+    int n;
+};
+__global__ void k_gather(const uint32_t *__restrict__ idx, uint64_t n, const Gather g) {
+    for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n; i += (uint64_t)gridDim.x * blockDim.x) {
+        const uint32_t j = idx[i];
+        for (int k = 0; k < g.n; ++k) g.dst[k][i] = __ldg(&g.src[k][j]);
+    }
 }
 
 struct Payload {
@@ -51,8 +77,7 @@ struct Payload {
     int n;
 };
 
-__global__ void __launch_bounds__(kSortThreads) k_radix_hist(const uint32_t *__restrict__ qx,
-                                                             const uint32_t *__restrict__ qy,
+__global__ void __launch_bounds__(kSortThreads) k_radix_hist(const uint32_t *__restrict__ key,
                                                              uint64_t n, int shift,
                                                              uint32_t *__restrict__ counts,
                                                              uint32_t ntiles) {
@@ -63,7 +88,7 @@ __global__ void __launch_bounds__(kSortThreads) k_radix_hist(const uint32_t *__r
     for (int k = threadIdx.x; k < kSortTile; k += kSortThreads) {
         const uint64_t i = base + k;
         if (i < n) {
-            const uint32_t d = sort_digit(qx[i], qy[i], shift);
+            const uint32_t d = sort_digit(key[i], shift);
             const unsigned peers = __match_any_sync(__activemask(), d);
             if ((threadIdx.x & 31) == __ffs(peers) - 1) atomicAdd(&hist[d], __popc(peers));
         }
@@ -95,7 +120,7 @@ __global__ void __launch_bounds__(kSortThreads) k_radix_scatter(Payload pl, uint
 #pragma unroll
     for (int j = 0; j < kSortItems; ++j) {
         const uint64_t i = seg + j * 32 + lane;
-        dig[j] = i < n ? sort_digit(pl.src[0][i], pl.src[1][i], shift) : 511u;
+        dig[j] = i < n ? sort_digit(pl.src[0][i], shift) : 511u;
         peers[j] = __match_any_sync(0xffffffffu, dig[j]);
         if (dig[j] < kDigits && lane == __ffs(peers[j]) - 1) wcount[w][dig[j]] += __popc(peers[j]);
         __syncwarp();
@@ -259,22 +284,24 @@ rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int
         Buf &counts = wsbuf(c, kWsSortCounts);
         if (dreserve(c, counts, ((uint64_t)kDigits * ntiles + 1) * 4) != cudaSuccess)
             return set_error(c, RJ_ERR_OOM, "sort counts allocation failed");
-        // pass p reads `from`, writes `to`; pass 0 reads B[0..1] (quantised),
-        // the implicit index, and the staged raw attribute columns
+        // Sort (key, index) pairs only -- 8 B per point per pass instead of
+        // every column -- then gather the columns once.  Buffers: keys
+        // ping-pong A[0] <-> A[1], indices B[2] <-> A[2]; pass 0 reads the
+        // implicit index.
+        k_keys<<<qb, 256, 0, c->stream>>>(B[0]->as<uint32_t>(), B[1]->as<uint32_t>(), n, A[0]->as<uint32_t>());
+        RJ_LAUNCHED(c);
+        RJ_CUDA(c, cudaGetLastError());
+        uint32_t *key[2] = {A[0]->as<uint32_t>(), A[1]->as<uint32_t>()};
+        uint32_t *ix[2] = {A[2]->as<uint32_t>(), B[2]->as<uint32_t>()};
         for (int pass = 0; pass < 4; ++pass) {
             Payload pl;
-            pl.n = P;
-            Buf **from = (pass % 2 == 0) ? B : A;
-            Buf **to = (pass % 2 == 0) ? A : B;
-            for (int k = 0; k < P; ++k) {
-                if (pass == 0)
-                    pl.src[k] = k < 2 ? from[k]->as<uint32_t>() : (k == 2 ? nullptr : (const uint32_t *)dcol[k - 3]);
-                else
-                    pl.src[k] = from[k]->as<uint32_t>();
-                pl.dst[k] = to[k]->as<uint32_t>();
-            }
-            k_radix_hist<<<ntiles, kSortThreads, 0, c->stream>>>(pl.src[0], pl.src[1], n, 8 * pass,
-                                                                 counts.as<uint32_t>(), ntiles);
+            pl.n = 2;
+            pl.src[0] = key[pass & 1];
+            pl.src[1] = pass == 0 ? nullptr : ix[pass & 1];
+            pl.dst[0] = key[(pass + 1) & 1];
+            pl.dst[1] = ix[(pass + 1) & 1];
+            k_radix_hist<<<ntiles, kSortThreads, 0, c->stream>>>(pl.src[0], n, 8 * pass, counts.as<uint32_t>(),
+                                                                 ntiles);
             RJ_LAUNCHED(c);
             RJ_CUDA(c, cudaGetLastError());
             RJ_CUDA(c, scan_u32(c, counts.as<uint32_t>(), counts.as<uint32_t>(), (uint64_t)kDigits * ntiles, kWsScan));
@@ -282,7 +309,25 @@ rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int
             RJ_LAUNCHED(c);
             RJ_CUDA(c, cudaGetLastError());
         }
-        // after 4 passes the sorted payload is in B (the context's columns)
+        // sorted indices in A[2] (pass 3 wrote ix[0]); keys are dead.  Gather
+        // qx -> A[0], qy -> A[1], attributes -> B[3 + k], then the context
+        // takes A[0..2] as its qx, qy, idx.
+        Gather g;
+        g.n = 2 + n_cols;
+        g.src[0] = B[0]->as<uint32_t>();
+        g.src[1] = B[1]->as<uint32_t>();
+        g.dst[0] = A[0]->as<uint32_t>();
+        g.dst[1] = A[1]->as<uint32_t>();
+        for (int k = 0; k < n_cols; ++k) {
+            g.src[2 + k] = (const uint32_t *)dcol[k];
+            g.dst[2 + k] = B[3 + k]->as<uint32_t>();
+        }
+        k_gather<<<qb, 256, 0, c->stream>>>(A[2]->as<uint32_t>(), n, g);
+        RJ_LAUNCHED(c);
+        RJ_CUDA(c, cudaGetLastError());
+        std::swap(c->qx, c->load_alt[0]);
+        std::swap(c->qy, c->load_alt[1]);
+        std::swap(c->idx, c->load_alt[2]);
     }
     for (int k = 0; k < n_cols; ++k) c->col_dtype[k] = dtypes[k];
     c->n_cols = n_cols;

@@ -739,6 +739,8 @@ rj_status rj_destroy(rj_ctx *c) {
     dfree(c, c->res_cnt); dfree(c, c->res_sum); dfree(c, c->res_val); dfree(c, c->res_eps); dfree(c, c->res_agg);
     stream_release(c);
     for (auto &e : c->ev) if (e) cudaEventDestroy(e);
+    for (auto &e : c->load_ev) if (e) cudaEventDestroy(e);
+    if (c->load_stream) cudaStreamDestroy(c->load_stream);
     if (c->h_stats) cudaFreeHost(c->h_stats);
     if (c->own_stream) cudaStreamDestroy(c->stream);
     delete c;

@@ -219,13 +219,13 @@ bool is_device_ptr(const void *p) {
 // Stage a column on the device (copy if host memory). Returns the device pointer.
 // Stage a column on the device (copy if host memory) into a grow-only
 // context buffer. Returns the device pointer.
-static rj_status stage(Ctx *c, const void *p, size_t bytes, Buf &tmp, const void **out) {
+static rj_status stage(Ctx *c, const void *p, size_t bytes, Buf &tmp, const void **out, cudaStream_t st = nullptr) {
     if (is_device_ptr(p)) {
         *out = p;
         return RJ_OK;
     }
     if (dreserve_exact(c, tmp, bytes) != cudaSuccess) return set_error(c, RJ_ERR_OOM, "staging allocation failed");
-    RJ_CUDA(c, cudaMemcpyAsync(tmp.p, p, bytes, cudaMemcpyHostToDevice, c->stream));
+    RJ_CUDA(c, cudaMemcpyAsync(tmp.p, p, bytes, cudaMemcpyHostToDevice, st ? st : c->stream));
     *out = tmp.p;
     return RJ_OK;
 }
@@ -252,8 +252,19 @@ rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int
     if (n) {
         if ((s = stage(c, x, n * esz, c->load_stage[0], &dx)) != RJ_OK) return s;
         if ((s = stage(c, y, n * esz, c->load_stage[1], &dy)) != RJ_OK) return s;
+        // the attribute columns are needed only by the final gather: their
+        // host-to-device copies run on a second stream beside the sort
+        if (n_cols) {
+            if (!c->load_stream) {
+                RJ_CUDA(c, cudaStreamCreateWithFlags(&c->load_stream, cudaStreamNonBlocking));
+                for (auto &e : c->load_ev) RJ_CUDA(c, cudaEventCreateWithFlags(&e, cudaEventDisableTiming));
+            }
+            RJ_CUDA(c, cudaEventRecord(c->load_ev[0], c->stream));        // staging buffers free
+            RJ_CUDA(c, cudaStreamWaitEvent(c->load_stream, c->load_ev[0], 0));
+        }
         for (int k = 0; k < n_cols; ++k)
-            if ((s = stage(c, cols[k], n * 4, c->load_stage[2 + k], &dcol[k])) != RJ_OK) return s;
+            if ((s = stage(c, cols[k], n * 4, c->load_stage[2 + k], &dcol[k], c->load_stream)) != RJ_OK) return s;
+        if (n_cols) RJ_CUDA(c, cudaEventRecord(c->load_ev[1], c->load_stream));
     }
     const int P = 3 + n_cols;
     Buf *B[kMaxPayload] = {&c->qx, &c->qy, &c->idx};
@@ -322,6 +333,7 @@ rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int
             g.src[2 + k] = (const uint32_t *)dcol[k];
             g.dst[2 + k] = B[3 + k]->as<uint32_t>();
         }
+        if (n_cols) RJ_CUDA(c, cudaStreamWaitEvent(c->stream, c->load_ev[1], 0));
         k_gather<<<qb, 256, 0, c->stream>>>(A[2]->as<uint32_t>(), n, g);
         RJ_LAUNCHED(c);
         RJ_CUDA(c, cudaGetLastError());

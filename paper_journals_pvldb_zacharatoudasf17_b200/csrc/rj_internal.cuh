@@ -170,6 +170,8 @@ struct Ctx {
     unsigned long long *h_stats = nullptr;   // pinned
     rj_stats last{};
     cudaEvent_t ev[6] = {};
+    cudaStream_t load_stream = nullptr;           // load: attribute-column copies beside the sort
+    cudaEvent_t load_ev[2] = {};
     uint32_t launches = 0;
     int last_stages = 0, last_ctas_per_sm = 0;   // point-pass launch shape of the last query
     PassArgs last_bq{};                           // last accurate query with a global boundary queue (bq_cap > 0)

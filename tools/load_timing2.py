@@ -15,7 +15,7 @@ R = rj.RasterJoin(box)
 R.load_polygons(C.array_polys(polys))
 desc = rj.make_desc(**q)
 cnt = np.zeros(R.n_poly, np.uint64); val = np.zeros(R.n_poly, np.float64)
-for it in range(4):
+for it in range(int(os.environ.get("ITERS", "4"))):
     torch.cuda.synchronize()
     t0 = time.perf_counter(); R.load_points(x, y, cols); t1 = time.perf_counter()
     rj.rj_query(R.ctx, desc, cnt, val); t2 = time.perf_counter()

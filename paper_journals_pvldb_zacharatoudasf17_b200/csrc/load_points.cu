@@ -24,22 +24,21 @@ namespace rj {
 namespace {
 constexpr uint32_t kInvalid = 0xFFFFFFFFu;
 constexpr int kSortThreads = 256;
-constexpr int kSortItems = 16;                       // per thread
+constexpr int kSortItems = 8;                        // per thread
 constexpr int kSortTile = kSortThreads * kSortItems; // 4096
 constexpr int kDigits = 257;                         // 256 + out-of-domain
 constexpr int kMaxPayload = 3 + RJ_MAX_COLS;
 
 template <typename T>
 __global__ void k_quantize(const T *__restrict__ x, const T *__restrict__ y, uint64_t n, double x0,
-                           double sx, double y0, double sy, uint32_t *__restrict__ qx,
-                           uint32_t *__restrict__ qy) {
+                           double sx, double y0, double sy, uint2 *__restrict__ qxy) {
     for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n;
          i += (uint64_t)gridDim.x * blockDim.x) {
         const double fx = floor(__dmul_rn(__ddiv_rn(__dsub_rn((double)x[i], x0), sx), 1073741824.0));
         const double fy = floor(__dmul_rn(__ddiv_rn(__dsub_rn((double)y[i], y0), sy), 1073741824.0));
         const bool ok = fx >= 0.0 && fx < 1073741824.0 && fy >= 0.0 && fy < 1073741824.0;
-        qx[i] = ok ? (uint32_t)fx : kInvalid;
-        qy[i] = ok ? (uint32_t)fy : kInvalid;
+        // (Qx, Qy) interleaved: the final gather reads both with one 8-B access
+        qxy[i] = ok ? make_uint2((uint32_t)fx, (uint32_t)fy) : make_uint2(kInvalid, kInvalid);
     }
 }
 
@@ -47,26 +46,30 @@ __global__ void k_quantize(const T *__restrict__ x, const T *__restrict__ y, uin
 // capped at 0xFFFFFFFE; out-of-domain points get 0xFFFFFFFF, so they sort
 // last by the key alone (the cap only merges two level-16 cells inside the
 // last level-10 cell, whose order within a cell is free).
-__global__ void k_keys(const uint32_t *__restrict__ qx, const uint32_t *__restrict__ qy, uint64_t n,
-                       uint32_t *__restrict__ key) {
+__global__ void k_keys(const uint2 *__restrict__ qxy, uint64_t n, uint32_t *__restrict__ key) {
     for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n; i += (uint64_t)gridDim.x * blockDim.x) {
-        const uint32_t x = qx[i], y = qy[i];
-        key[i] = x == kInvalid ? 0xFFFFFFFFu : min(morton_key(x, y), 0xFFFFFFFEu);
+        const uint2 q = qxy[i];
+        key[i] = q.x == kInvalid ? 0xFFFFFFFFu : min(morton_key(q.x, q.y), 0xFFFFFFFEu);
     }
 }
 
 __device__ __forceinline__ uint32_t sort_digit(uint32_t key, int shift) { return (key >> shift) & 255u; }
 
 // After the (key, index) sort: every column in sorted order, gathered once
-// (qx, qy and the attribute columns of point idx[i] go to position i).
+// (Qx, Qy and the attribute columns of point idx[i] go to position i).
 struct Gather {
-    const uint32_t *src[2 + RJ_MAX_COLS];
-    uint32_t *dst[2 + RJ_MAX_COLS];
+    const uint2 *qxy;
+    uint32_t *qx, *qy;
+    const uint32_t *src[RJ_MAX_COLS];
+    uint32_t *dst[RJ_MAX_COLS];
     int n;
 };
 __global__ void k_gather(const uint32_t *__restrict__ idx, uint64_t n, const Gather g) {
     for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < n; i += (uint64_t)gridDim.x * blockDim.x) {
         const uint32_t j = idx[i];
+        const uint2 q = __ldg(&g.qxy[j]);
+        g.qx[i] = q.x;
+        g.qy[i] = q.y;
         for (int k = 0; k < g.n; ++k) g.dst[k][i] = __ldg(&g.src[k][j]);
     }
 }
@@ -234,6 +237,7 @@ static rj_status stage(Ctx *c, const void *p, size_t bytes, Buf &tmp, const void
 void free_load_scratch(Ctx *c) {
     for (auto &b : c->load_stage) dfree(c, b);
     for (auto &b : c->load_alt) dfree(c, b);
+    dfree(c, c->load_qxy);
 }
 
 rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int xy_f64, int n_cols,
@@ -280,14 +284,15 @@ rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int
 
     if (n) {
         const unsigned qb = (unsigned)std::min<uint64_t>(blocks_for(n, 256), (uint64_t)c->num_sms * 16);
+        if (dreserve_exact(c, c->load_qxy, n * 8) != cudaSuccess)
+            return set_error(c, RJ_ERR_OOM, "point buffers allocation failed");
+        uint2 *qxy = c->load_qxy.as<uint2>();
         if (xy_f64)
             k_quantize<double><<<qb, 256, 0, c->stream>>>((const double *)dx, (const double *)dy, n, c->x0,
-                                                          c->x1 - c->x0, c->y0, c->y1 - c->y0,
-                                                          B[0]->as<uint32_t>(), B[1]->as<uint32_t>());
+                                                          c->x1 - c->x0, c->y0, c->y1 - c->y0, qxy);
         else
             k_quantize<float><<<qb, 256, 0, c->stream>>>((const float *)dx, (const float *)dy, n, c->x0,
-                                                         c->x1 - c->x0, c->y0, c->y1 - c->y0,
-                                                         B[0]->as<uint32_t>(), B[1]->as<uint32_t>());
+                                                         c->x1 - c->x0, c->y0, c->y1 - c->y0, qxy);
         RJ_LAUNCHED(c);
         RJ_CUDA(c, cudaGetLastError());
 
@@ -299,7 +304,7 @@ rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int
         // every column -- then gather the columns once.  Buffers: keys
         // ping-pong A[0] <-> A[1], indices B[2] <-> A[2]; pass 0 reads the
         // implicit index.
-        k_keys<<<qb, 256, 0, c->stream>>>(B[0]->as<uint32_t>(), B[1]->as<uint32_t>(), n, A[0]->as<uint32_t>());
+        k_keys<<<qb, 256, 0, c->stream>>>(qxy, n, A[0]->as<uint32_t>());
         RJ_LAUNCHED(c);
         RJ_CUDA(c, cudaGetLastError());
         uint32_t *key[2] = {A[0]->as<uint32_t>(), A[1]->as<uint32_t>()};
@@ -324,14 +329,13 @@ rj_status load_points_impl(Ctx *c, uint64_t n, const void *x, const void *y, int
         // qx -> A[0], qy -> A[1], attributes -> B[3 + k], then the context
         // takes A[0..2] as its qx, qy, idx.
         Gather g;
-        g.n = 2 + n_cols;
-        g.src[0] = B[0]->as<uint32_t>();
-        g.src[1] = B[1]->as<uint32_t>();
-        g.dst[0] = A[0]->as<uint32_t>();
-        g.dst[1] = A[1]->as<uint32_t>();
+        g.n = n_cols;
+        g.qxy = qxy;
+        g.qx = A[0]->as<uint32_t>();
+        g.qy = A[1]->as<uint32_t>();
         for (int k = 0; k < n_cols; ++k) {
-            g.src[2 + k] = (const uint32_t *)dcol[k];
-            g.dst[2 + k] = B[3 + k]->as<uint32_t>();
+            g.src[k] = (const uint32_t *)dcol[k];
+            g.dst[k] = B[3 + k]->as<uint32_t>();
         }
         if (n_cols) RJ_CUDA(c, cudaStreamWaitEvent(c->stream, c->load_ev[1], 0));
         k_gather<<<qb, 256, 0, c->stream>>>(A[2]->as<uint32_t>(), n, g);

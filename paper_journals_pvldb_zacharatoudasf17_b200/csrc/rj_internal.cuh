@@ -119,6 +119,7 @@ struct Ctx {
     Buf qx, qy, idx, col[RJ_MAX_COLS];
     Buf load_stage[2 + RJ_MAX_COLS];           // H2D staging (grow-only)
     Buf load_alt[3 + RJ_MAX_COLS];             // the sort's second buffer (grow-only)
+    Buf load_qxy;                              // quantised (Qx, Qy) interleaved, before the gather (grow-only)
     int keep_load_scratch = 1;                 // RJ_OPT_KEEP_LOAD_SCRATCH
     Buf cell_off;                 // [kCells10 + 1]
     std::vector<uint32_t> h_cell_off;          // host copy (work-item planning)

@@ -21,9 +21,11 @@
 //       1. clear the tile (accurate mode: boundary pixels carry kFlag);
 //       2. per stage, one 256-point window per warp (8 points per lane):
 //          filter, project (pix = umulhi(q, 4W)), merge runs of equal pixels
-//          (Morton order: inside a lane in registers, across lanes with a
-//          warp segmented scan) and add each run with one shared reduction;
-//          boundary points go to a per-warp queue tested 32 at a time;
+//          (Morton order: inside a lane in registers -- process_lane_runs,
+//          the default; or also across lanes with a warp segmented scan --
+//          process, RJ_OPT_LANE_RUNS = 2) and add each run with one shared
+//          reduction; accurate mode: boundary points go to the global queue
+//          (k_pip_queue tests them after the pass);
 //       3. at the cell's last stage, every span piece (polygon P, row,
 //          [lo, hi)) sums its pixels straight from the tile into P's
 //          per-CTA partial (S4).

@@ -25,7 +25,7 @@ namespace {
 constexpr uint32_t kInvalid = 0xFFFFFFFFu;
 constexpr int kSortThreads = 256;
 constexpr int kSortItems = 8;                        // per thread
-constexpr int kSortTile = kSortThreads * kSortItems; // 4096
+constexpr int kSortTile = kSortThreads * kSortItems; // 2048
 constexpr int kDigits = 257;                         // 256 + out-of-domain
 constexpr int kMaxPayload = 3 + RJ_MAX_COLS;
 
@@ -88,13 +88,19 @@ __global__ void __launch_bounds__(kSortThreads) k_radix_hist(const uint32_t *__r
     for (int d = threadIdx.x; d < kDigits; d += kSortThreads) hist[d] = 0;
     __syncthreads();
     const uint64_t base = (uint64_t)blockIdx.x * kSortTile;
-    for (int k = threadIdx.x; k < kSortTile; k += kSortThreads) {
-        const uint64_t i = base + k;
-        if (i < n) {
-            const uint32_t d = sort_digit(key[i], shift);
-            const unsigned peers = __match_any_sync(__activemask(), d);
-            if ((threadIdx.x & 31) == __ffs(peers) - 1) atomicAdd(&hist[d], __popc(peers));
-        }
+    // all of the thread's keys in flight at once, then the per-key matching
+    uint32_t kv[kSortItems];
+#pragma unroll
+    for (int j = 0; j < kSortItems; ++j) {
+        const uint64_t i = base + threadIdx.x + j * kSortThreads;
+        kv[j] = i < n ? key[i] : 0u;
+    }
+#pragma unroll
+    for (int j = 0; j < kSortItems; ++j) {
+        const uint64_t i = base + threadIdx.x + j * kSortThreads;
+        const uint32_t d = i < n ? sort_digit(kv[j], shift) : 511u;   // 511: past the end, not counted
+        const unsigned peers = __match_any_sync(0xFFFFFFFFu, d);
+        if (d < (uint32_t)kDigits && (threadIdx.x & 31) == __ffs(peers) - 1) atomicAdd(&hist[d], __popc(peers));
     }
     __syncthreads();
     for (int d = threadIdx.x; d < kDigits; d += kSortThreads)
@@ -121,9 +127,14 @@ __global__ void __launch_bounds__(kSortThreads) k_radix_scatter(Payload pl, uint
     __syncwarp();
     uint32_t dig[kSortItems], peers[kSortItems];
 #pragma unroll
+    for (int j = 0; j < kSortItems; ++j) {                // keys in flight together
+        const uint64_t i = seg + j * 32 + lane;
+        dig[j] = i < n ? pl.src[0][i] : 0u;
+    }
+#pragma unroll
     for (int j = 0; j < kSortItems; ++j) {
         const uint64_t i = seg + j * 32 + lane;
-        dig[j] = i < n ? sort_digit(pl.src[0][i], shift) : 511u;
+        dig[j] = i < n ? sort_digit(dig[j], shift) : 511u;
         peers[j] = __match_any_sync(0xffffffffu, dig[j]);
         if (dig[j] < kDigits && lane == __ffs(peers[j]) - 1) wcount[w][dig[j]] += __popc(peers[j]);
         __syncwarp();
